@@ -1,0 +1,33 @@
+# Native build for ocelot-b200.  sm_100a only (B200); nvcc cross-compiles without a GPU.
+NVCC      ?= /usr/local/cuda/bin/nvcc
+CXX       ?= g++
+CC        ?= gcc
+ARCH      := -gencode arch=compute_100a,code=sm_100a
+NVFLAGS   := $(ARCH) -O3 -lineinfo -std=c++17 -Xcompiler -fPIC -Xcompiler -Wall --expt-relaxed-constexpr -Xptxas -v
+PKG       := paper_journals_pvldb_heimelspmm13_b200
+LIB       := $(PKG)/_lib/libocelot_b200.so
+CSRC      := $(wildcard $(PKG)/csrc/*.cu)
+CHDR      := $(wildcard $(PKG)/csrc/*.cuh) include/ocelot_b200.h
+
+all: $(LIB) oracle/liboracle.so datagen/liboclgen_host.so datagen/liboclgen_dev.so
+
+# product library: hand-written CUDA kernels + C ABI (no torch types)
+$(LIB): $(CSRC) $(CHDR)
+	@mkdir -p $(PKG)/_lib
+	$(NVCC) $(NVFLAGS) -Iinclude -shared -o $@ $(CSRC) -lcudart 2> $(PKG)/_lib/ptxas.log || (cat $(PKG)/_lib/ptxas.log; exit 1)
+
+# oracle: test infrastructure only; plain C++17, single-threaded, no FMA contraction
+oracle/liboracle.so: oracle/oracle.cpp oracle/oracle.h
+	$(CXX) -O2 -std=c++17 -ffp-contract=off -fno-fast-math -fPIC -shared -o $@ oracle/oracle.cpp
+
+# seeded input generators shared by both sides (no method arithmetic)
+datagen/liboclgen_host.so: datagen/datagen_host.c datagen/ocl_datagen.h
+	$(CC) -O2 -pthread -ffp-contract=off -fPIC -shared -o $@ datagen/datagen_host.c -lm
+
+datagen/liboclgen_dev.so: datagen/datagen_dev.cu datagen/ocl_datagen.h
+	$(NVCC) $(ARCH) -O3 -Xcompiler -fPIC -shared -o $@ datagen/datagen_dev.cu -lcudart
+
+clean:
+	rm -f $(LIB) oracle/liboracle.so datagen/liboclgen_host.so datagen/liboclgen_dev.so
+
+.PHONY: all clean
