@@ -1,0 +1,337 @@
+#!/usr/bin/env python
+"""Benchmark: fused select -> hash GROUP BY -> aggregate on B200 (BASELINE.json metric).
+
+One step = one pass of the whole hot path (predicate, grouping, aggregation,
+finalisation; + allgather/merge when N > 1) over the workload's rows, inputs
+already resident in HBM.  Default workload = config C4 (600M-row lineitem,
+TPC-H-Q1-style filter + GROUP BY returnflag, linestatus, int64 decimals), the
+configuration the north-star target (>= 60% of HBM bandwidth on one B200) is
+quoted on.  N > 1 (torchrun): rows are sharded across ranks (fixed total work,
+"strong" scaling) and the partial group tables are merged with an NCCL allgather.
+
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload c4|c2|c1|c3] [--impl ours|reference]
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import sys
+import threading
+import time
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+import numpy as np  # noqa: E402
+import torch  # noqa: E402
+
+import datagen  # noqa: E402
+
+METRIC = "rows/s and % HBM roofline, fused select+GROUP BY at 1/2/4/8 B200"
+Q1_AGGS = [
+    {"op": "sum", "a": 0}, {"op": "sum", "a": 1},
+    {"op": "sum", "expr": "mul_1minus", "a": 1, "b": 2, "scale": 2},
+    {"op": "sum", "expr": "mul_1minus_1plus", "a": 1, "b": 2, "c": 3, "scale": 2},
+    {"op": "avg", "a": 0}, {"op": "avg", "a": 1}, {"op": "avg", "a": 2}, {"op": "count"},
+]
+Q1_PRED = {"hi": datagen.Q1_SHIP_CUTOFF}
+
+WORKLOADS = {
+    "c4": dict(desc="C4: lineitem SF100, 600,000,000 rows; TPC-H-Q1-style fused select l_shipdate<=1998-09-02 "
+                    "+ GROUP BY (l_returnflag, l_linestatus) = 4 groups; int64 decimal SUM/AVG (int128 exact) + COUNT",
+               rows=600_000_000, seed=datagen.BASE_SEED + 4, kind="q1", f64=False, groups=4),
+    "c2": dict(desc="C2: lineitem SF1, 6,000,000 rows; Q1-style 4-group aggregation on fp64 columns with AVG",
+               rows=6_000_000, seed=datagen.BASE_SEED + 2, kind="q1", f64=True, groups=4),
+    "c1": dict(desc="C1: lineitem SF0.01, 60,000 rows; Q1-style 4 groups, int64 decimals",
+               rows=60_000, seed=datagen.BASE_SEED + 1, kind="q1", f64=False, groups=4),
+    "c3": dict(desc="C3: lineitem SF10, 60,000,000 rows; GROUP BY l_orderkey (15M groups, HBM hash table), "
+                    "COUNT/SUM/MIN/MAX(l_quantity), clustered row order",
+               rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000),
+}
+
+
+def q1_fields(f64):
+    return (("shipdate", "returnflag", "linestatus") +
+            (("quantity_f", "extendedprice_f", "discount_f", "tax_f") if f64 else
+             ("quantity", "extendedprice", "discount", "tax")))
+
+
+def workload_columns(wl, cols):
+    """(preds, keys, vals, aggs, bytes_per_row) for a dict of columns."""
+    if wl["kind"] == "q1":
+        v = ["quantity", "extendedprice", "discount", "tax"]
+        if wl["f64"]:
+            v = [x + "_f" for x in v]
+        aggs = [dict(a, scale=0) if wl["f64"] and a.get("expr", "col") != "col" else a for a in Q1_AGGS]
+        return ([(cols["shipdate"], Q1_PRED)], [cols["returnflag"], cols["linestatus"]], [cols[x] for x in v],
+                aggs, 4 + 1 + 1 + 4 * 8)
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    return [], [cols["orderkey"]], [cols["quantity"]], aggs, 16
+
+
+def wl_fields(wl):
+    return q1_fields(wl["f64"]) if wl["kind"] == "q1" else ("orderkey", "quantity")
+
+
+class ClockSampler:
+    """NVML sampling of SM clock and throttle reasons during the timed region."""
+
+    REASONS = {0x1: "gpu_idle", 0x2: "applications_clocks_setting", 0x4: "sw_power_cap", 0x8: "hw_slowdown",
+               0x20: "sw_thermal_slowdown", 0x40: "hw_thermal_slowdown", 0x80: "hw_power_brake_slowdown",
+               0x100: "display_clock_setting"}
+
+    def __init__(self, index):
+        self.samples, self.reasons, self.ok = [], set(), False
+        try:
+            import pynvml
+            pynvml.nvmlInit()
+            self.nv = pynvml
+            self.h = pynvml.nvmlDeviceGetHandleByIndex(index)
+            self.max_mhz = pynvml.nvmlDeviceGetMaxClockInfo(self.h, pynvml.NVML_CLOCK_SM)
+            self.ok = True
+        except Exception:  # noqa: BLE001
+            self.max_mhz = None
+        self._stop = threading.Event()
+
+    def _run(self):
+        while not self._stop.is_set():
+            try:
+                self.samples.append(self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM))
+                r = self.nv.nvmlDeviceGetCurrentClocksEventReasons(self.h)
+                for bit, name in self.REASONS.items():
+                    if r & bit:
+                        self.reasons.add(name)
+            except Exception:  # noqa: BLE001
+                pass
+            time.sleep(0.002)
+
+    def __enter__(self):
+        if self.ok:
+            self.t = threading.Thread(target=self._run, daemon=True)
+            self.t.start()
+        return self
+
+    def __exit__(self, *a):
+        self._stop.set()
+        if self.ok:
+            self.t.join()
+
+    def summary(self):
+        if not self.samples:
+            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": sorted(self.reasons), "samples": 0}
+        return {"sm_mhz": statistics.median(self.samples), "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(self.reasons - {"gpu_idle"}), "samples": len(self.samples)}
+
+
+def measured_peak_gbs():
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            return float(json.load(f)["hbm_gbs"]), "measured (MEASURED_PEAKS.json hbm_gbs)"
+    except Exception:  # noqa: BLE001
+        return 6650.0, "fallback (B200_PROFILING.md)"
+
+
+def profiled_traffic(workload, rows):
+    """dram read+write bytes per launch of the fused kernel from the committed ncu summary, scaled per row."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "traffic.json")) as f:
+            t = json.load(f)[workload]
+        return t["dram_bytes_per_row"] * rows
+    except Exception:  # noqa: BLE001
+        return None
+
+
+def oracle_time(wl, cols, rows):
+    import oracle
+    p, k, v, a, _ = workload_columns(wl, {f: c[:rows] for f, c in cols.items()})
+    t0 = time.perf_counter()
+    oracle.sga(p, k, v, a, order_by_key=(wl["kind"] == "q1"))
+    return time.perf_counter() - t0
+
+
+def run_reference(args, wl, rank):
+    """--impl reference: the CPU oracle (as it stands, 1 thread) on a bounded sample per step."""
+    if rank != 0:
+        return
+    sample = min(wl["rows"], args.ref_rows)
+    cols = datagen.lineitem_host(sample, wl["seed"], fields=wl_fields(wl), n_total=wl["rows"])
+    for _ in range(args.warmup):
+        oracle_time(wl, cols, sample)
+    ts = [oracle_time(wl, cols, sample) for _ in range(args.steps)]
+    ms = 1e3 * statistics.mean(ts)
+    value = sample / (ms / 1e3)
+    desc = f"first {sample:,} rows of the {wl['rows']:,}-row workload per step, oracle.sga single-threaded"
+    line = {"impl": "reference", "metric": METRIC, "value": value, "unit": "rows/s", "n_gpus": args.gpus,
+            "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
+            "scaling": "strong", "vs_baseline": None, "dtype": "int64" if not wl["f64"] else "f64",
+            "data": "synthetic (seeded lineitem-shaped generator, datagen/)",
+            "config": {"workload": wl["desc"], "rows": wl["rows"], "sample_rows": sample},
+            "cpu_baseline": {"value": value, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": desc},
+            "e2e": {"value": value, "unit": "rows/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
+    print(json.dumps(line), flush=True)
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--workload", default="c4", choices=sorted(WORKLOADS))
+    ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
+    ap.add_argument("--ref-rows", type=int, default=20_000_000)
+    ap.add_argument("--cpu-rows", type=int, default=200_000_000, help="cpu_baseline sample (rows)")
+    ap.add_argument("--e2e-steps", type=int, default=3)
+    ap.add_argument("--no-e2e", action="store_true")
+    ap.add_argument("--no-cpu", action="store_true")
+    ap.add_argument("--tier", type=int, default=0)
+    args = ap.parse_args()
+    wl = WORKLOADS[args.workload]
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local = int(os.environ.get("LOCAL_RANK", "0"))
+    if args.impl == "reference":
+        run_reference(args, wl, rank)
+        return
+    torch.cuda.set_device(local)
+    dev = torch.device("cuda", local)
+    if world > 1:
+        import torch.distributed as dist
+        dist.init_process_group("nccl", device_id=dev)
+    import paper_journals_pvldb_heimelspmm13_b200 as ocl
+    from paper_journals_pvldb_heimelspmm13_b200.distributed import distributed_select_group_aggregate, shard_range
+
+    n = wl["rows"]
+    start, length = shard_range(n, rank, world)
+    cols = datagen.lineitem_device(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, device=dev)
+    torch.cuda.synchronize()
+    p, k, v, aggs, bpr = workload_columns(wl, cols)
+    order = wl["kind"] == "q1"
+    eg = wl["groups"] if world == 1 else wl["groups"]
+    call = ocl.SgaCall(p, k, v, aggs, expected_groups=eg, out_capacity=max(16, 2 * eg), order_by_key=order,
+                       tier=args.tier)
+    ctx = call.ctx
+
+    def step():
+        if world == 1:
+            call.launch()
+        else:
+            distributed_select_group_aggregate(call)
+
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    keys, outs = call.result()           # raises on a device status error
+    G = len(keys)
+
+    K = args.steps
+    kev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(K)]
+    t0, t1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    if world > 1:
+        dist.barrier()
+    torch.cuda.synchronize()
+    launches0 = ocl.launch_count()
+    with ClockSampler(local) as clk:
+        t0.record()
+        for i in range(K):
+            ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
+            step()
+        t1.record()
+        torch.cuda.synchronize()
+    ocl.set_kernel_events(ctx, None, None)
+    launches = ocl.launch_count() - launches0
+    if world > 1:
+        dist.barrier()
+    ms = t0.elapsed_time(t1) / K
+    kms = statistics.mean(a.elapsed_time(b) for a, b in kev)
+    if world > 1:
+        tt = torch.tensor([ms, kms], dtype=torch.float64, device=dev)
+        dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+        ms, kms = tt.tolist()
+    value = n / (ms / 1e3)
+    peak, peak_src = measured_peak_gbs()
+    algo_bytes = bpr * length
+    achieved = algo_bytes / (kms / 1e3) / 1e9
+
+    # ---- end to end: host (pinned) buffers through the public API, copies inside the timed region
+    e2e = None
+    if not args.no_e2e:
+        host = {f: torch.empty(length, dtype=c.dtype, pin_memory=True) for f, c in cols.items()}
+        datagen.lineitem_host(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n,
+                              out={f: h.numpy() for f, h in host.items()})
+        hp, hk, hv, haggs, _ = workload_columns(wl, host)
+        h2d = sum(h.numel() * h.element_size() for h in host.values())
+        if world == 1:
+            hcall = ocl.SgaCall(hp, hk, hv, haggs, expected_groups=eg, out_capacity=max(16, 2 * eg),
+                                order_by_key=order, tier=args.tier, host=True, chunk_rows=1 << 24)
+            hcall.launch()                                     # warm-up
+            ke = max(1, args.e2e_steps)
+            torch.cuda.synchronize()
+            te = time.perf_counter()
+            for _ in range(ke):
+                hcall.launch()                                 # blocks until results are on the host
+            e2e_s = (time.perf_counter() - te) / ke
+            hk_, ho_ = hcall.result()
+            d2h = 8 + 4 + len(hk_) * 8 + sum(o.numel() * o.element_size() for o in ho_)
+        else:
+            dcols = {f: torch.empty_like(c) for f, c in cols.items()}
+            dp, dk, dv, daggs, _ = workload_columns(wl, dcols)
+            dcall = ocl.SgaCall(dp, dk, dv, daggs, expected_groups=eg, out_capacity=max(16, 2 * eg),
+                                order_by_key=order, tier=args.tier)
+            ke = max(1, args.e2e_steps)
+            dist.barrier()
+            torch.cuda.synchronize()
+            te = time.perf_counter()
+            for _ in range(ke):
+                for f in dcols:
+                    dcols[f].copy_(host[f], non_blocking=True)
+                distributed_select_group_aggregate(dcall)
+                hk_ = dcall.keys_out.cpu()
+                ho_ = [o.cpu() for o in dcall.outs]
+            torch.cuda.synchronize()
+            e2e_s = (time.perf_counter() - te) / ke
+            tt = torch.tensor([e2e_s], dtype=torch.float64, device=dev)
+            dist.all_reduce(tt, op=dist.ReduceOp.MAX)
+            e2e_s = tt.item()
+            d2h = int(hk_.numel() * 8 + sum(o.numel() * o.element_size() for o in ho_))
+        e2e = {"value": n / e2e_s, "unit": "rows/s", "h2d_bytes_per_step": int(h2d),
+               "d2h_bytes_per_step": int(d2h), "steps": ke,
+               "path": "ocl_select_group_aggregate_host (pinned host columns, chunked H2D overlapped with the "
+                       "fused kernel, D2H of the result)" if world == 1 else
+                       "torch H2D copies + distributed fused step + D2H of the result"}
+
+    cpu = None
+    if rank == 0 and world == 1 and not args.no_cpu:
+        sample = min(n, args.cpu_rows)
+        hcols = {f: h.numpy()[:sample] for f, h in host.items()} if e2e is not None else \
+            datagen.lineitem_host(sample, wl["seed"], fields=wl_fields(wl), n_total=n)
+        dt = oracle_time(wl, hcols, sample)
+        cpu = {"value": sample / dt, "unit": "rows/s", "cores": 1, "kind": "oracle",
+               "sample": f"first {sample:,} rows of the same workload, oracle.sga (C++17, single thread), "
+                         f"{dt:.1f} s"}
+
+    if rank == 0:
+        line = {
+            "metric": METRIC, "value": value, "unit": "rows/s", "n_gpus": world, "steps": K, "warmup": args.warmup,
+            "ms_per_step": ms, "higher_is_better": True, "scaling": "strong", "vs_baseline": None,
+            "dtype": "f64" if wl["f64"] else "int64",
+            "data": "synthetic (seeded lineitem-shaped generator datagen/, generated in place on each GPU)",
+            "config": {"workload": wl["desc"], "rows": n, "rows_per_gpu": length, "groups": G,
+                       "bytes_per_row": bpr, "parallelism": f"row-sharded dp{world}",
+                       "l2": f"inputs {bpr * length / 1e9:.1f} GB per GPU >> 126 MB L2, no flush needed"
+                             if bpr * length > 2e9 else "inputs smaller than L2: L2-resident"},
+            "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
+                         "traffic": profiled_traffic(args.workload, length), "kernel": "ocl::k_sga_reg (fused)" if
+                         (args.tier == 1 or (args.tier == 0 and eg <= 4)) else "ocl::k_sga_glb (fused)",
+                         "kernel_ms": kms, "algorithmic_bytes_per_launch": algo_bytes, "peak_source": peak_src},
+            "hbm_frac_step": algo_bytes / (ms / 1e3) / 1e9 / peak,
+            "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clk.summary(),
+        }
+        print(json.dumps(line), flush=True)
+    if world > 1:
+        dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    main()

@@ -1,0 +1,486 @@
+// fused.cu — K9: fused select -> hash group -> aggregate, one pass over the columns.
+//
+// Paper steps fused here: selection (§4.1.1), hash group-by
+// with dense group ids (L551-561 §4.1.6; hashing L511-533 §4.1.4), multi-column
+// grouping on combined ids (L559-561), hierarchical grouped aggregation with
+// per-work-group tables and several accumulators per group for few groups
+// (L562-600 §4.1.7).  Nothing is materialised: no bitmap (unless requested for
+// tests), no oid list, no gid column.
+//
+// B200 design:
+//  * persistent grid (#SMs x resident CTAs); a warp owns tiles of 64*U rows; lane
+//    l handles rows (2l, 2l+1) of each 64-row unit, so every column is read with one
+//    vector load per lane per unit (u8: 2 B, i32: 8 B, i64/f64: 16 B) and every
+//    warp-wide load is a contiguous, fully-used run (P:L619-633 GPU pattern).
+//  * REGISTER tier (few groups): each thread keeps L private accumulator slots in
+//    registers — the limit of the paper's "multiple accumulators per group" idea:
+//    one accumulator set per thread, no atomics in the row loop.  A block-wide
+//    slot directory in shared memory gives every thread the same key -> slot map.
+//    Integer SUMs use 96-bit (lo64 + hi32) predicated add-with-carry chains: exact
+//    for any per-thread row count < 2^31 (the int128 state is formed at flush).
+//  * GLOBAL tier (many groups): find-or-insert in the HBM open-addressing table
+//    and update the entry with atomics (native f64 add, int128 as two u64 atomics).
+//  * Rows a tier cannot place (more than L keys in a block, int32-overflowing
+//    factors, the key ~0) take the exact int128 global path, so every tier is
+//    correct for every input; the tier only decides speed.
+#include "launch.cuh"
+#include "rowops.cuh"
+
+namespace ocl {
+
+constexpr int kFusedThreads = 256;
+
+__device__ __forceinline__ void add96(bool pr, uint32_t& a0, uint32_t& a1, uint32_t& a2, int64_t v) {
+  uint32_t v0 = (uint32_t)(uint64_t)v, v1 = (uint32_t)((uint64_t)v >> 32), v2 = (uint32_t)(v >> 63);
+  asm("{\n\t.reg .pred p;\n\t"
+      "setp.ne.u32 p, %3, 0;\n\t"
+      "@p add.cc.u32 %0, %0, %4;\n\t"
+      "@p addc.cc.u32 %1, %1, %5;\n\t"
+      "@p addc.u32 %2, %2, %6;\n\t}"
+      : "+r"(a0), "+r"(a1), "+r"(a2)
+      : "r"((uint32_t)pr), "r"(v0), "r"(v1), "r"(v2));
+}
+
+__device__ __forceinline__ I128 warp_sum_i128(I128 x) {
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) {
+    I128 y;
+    y.lo = __shfl_xor_sync(0xffffffffu, x.lo, o);
+    y.hi = __shfl_xor_sync(0xffffffffu, x.hi, o);
+    x = i128_add(x, y);
+  }
+  return x;
+}
+
+// Block-wide slot directory: stored keys (~key), 0 = free.  Returns slot or -1.
+template <int L>
+__device__ __forceinline__ int dir_find_or_insert(uint64_t* dir, uint64_t key) {
+  uint64_t sk = ~key;
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    uint64_t cur = *(volatile uint64_t*)&dir[s];
+    if (cur == sk) return s;
+    if (cur == 0) {
+      uint64_t prev = atomicCAS((unsigned long long*)&dir[s], 0ULL, (unsigned long long)sk);
+      if (prev == 0 || prev == sk) return s;
+    }
+  }
+  return -1;
+}
+
+// Per-row inputs after predicate / key / value evaluation.
+template <int NV, bool F64>
+struct RowIn {
+  bool q;
+  bool fast;
+  uint64_t key;
+  int64_t vi[F64 ? 1 : NV];
+  double vd[F64 ? NV : 1];
+};
+
+// Evaluate values of one row from raw operands (vector path: loaded as pairs).
+template <int NV, bool F64>
+__device__ __forceinline__ void eval_values_pair(const Plan& p, int64_t r, RowIn<NV, F64>& x0, RowIn<NV, F64>& x1) {
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (!F64) {
+      if (d.is_f64) {   // mixed int/fp64 plan: fp64 values take the exact slow path
+        x0.fast = x1.fast = false;
+        continue;
+      }
+    }
+    uint64_t a0, a1, b0 = 0, b1 = 0, c0 = 0, c1 = 0;
+    load_pair(d.a, r, a0, a1);
+    if (d.expr >= OCL_EXPR_MUL_1MINUS) load_pair(d.b, r, b0, b1);
+    if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS) load_pair(d.c, r, c0, c1);
+    if constexpr (F64) {
+      x0.vd[v] = value_f64(d, a0, b0, c0);
+      x1.vd[v] = value_f64(d, a1, b1, c1);
+    } else {
+      x0.vi[v] = value_i64_fast(d, a0, b0, c0, x0.fast);
+      x1.vi[v] = value_i64_fast(d, a1, b1, c1, x1.fast);
+    }
+  }
+}
+
+template <int NV, bool F64>
+__device__ __forceinline__ void eval_row_scalar(const Plan& p, int64_t r, RowIn<NV, F64>& x) {
+  x.fast = true;
+  x.q = r < p.n && row_pred_scalar(p, r);
+  x.key = 0;
+  if (!x.q) return;
+  x.key = row_key_scalar(p, r);
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (!F64) {
+      if (d.is_f64) {
+        x.fast = false;
+        continue;
+      }
+    }
+    uint64_t a = load_one(d.a, r);
+    uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? load_one(d.b, r) : 0;
+    uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? load_one(d.c, r) : 0;
+    if constexpr (F64) x.vd[v] = value_f64(d, a, b, c);
+    else x.vi[v] = value_i64_fast(d, a, b, c, x.fast);
+  }
+}
+
+template <int NV, bool F64>
+__device__ __forceinline__ void eval_pair_vec(const Plan& p, int64_t r, RowIn<NV, F64>& x0, RowIn<NV, F64>& x1) {
+  x0.q = true;
+  x1.q = true;
+#pragma unroll
+  for (int i = 0; i < kMaxPreds; ++i) {
+    if (i >= p.npreds) break;
+    uint64_t u0, u1;
+    load_pair(p.preds[i].col, r, u0, u1);
+    x0.q = x0.q && eval_pred(p.preds[i], u0);
+    x1.q = x1.q && eval_pred(p.preds[i], u1);
+  }
+  x0.key = 0;
+  x1.key = 0;
+#pragma unroll
+  for (int i = 0; i < kMaxKeys; ++i) {
+    if (i >= p.nkeys) break;
+    uint64_t u0, u1;
+    load_pair(p.keys[i].col, r, u0, u1);
+    x0.key |= (u0 & p.keys[i].mask) << p.keys[i].shift;
+    x1.key |= (u1 & p.keys[i].mask) << p.keys[i].shift;
+  }
+  x0.fast = true;
+  x1.fast = true;
+  eval_values_pair<NV, F64>(p, r, x0, x1);
+}
+
+// Optional bitmap output for a 64-row unit: rows base + 2*lane + {0,1}.
+__device__ __forceinline__ void emit_bitmap_unit(const Plan& p, int64_t base, int lane, bool q0, bool q1) {
+  uint32_t b = (uint32_t)q0 | ((uint32_t)q1 << 1);
+  uint32_t w0 = __reduce_or_sync(0xffffffffu, lane < 16 ? b << (2 * lane) : 0u);
+  uint32_t w1 = __reduce_or_sync(0xffffffffu, lane >= 16 ? b << (2 * (lane - 16)) : 0u);
+  int64_t words = (p.n + 31) >> 5;
+  int64_t wi = base >> 5;
+  if (lane == 0 && wi < words) p.bitmap_out[wi] = w0;
+  if (lane == 1 && wi + 1 < words) p.bitmap_out[wi + 1] = w1;
+}
+
+// ------------------------------------------------------------------ register tier
+template <int L, int NV, bool F64, bool MINMAX>
+struct RegState {
+  uint64_t rk[L];                      // real keys of the block directory (~0 = none)
+  uint32_t cnt[L];
+  uint32_t s0[F64 ? 1 : L][F64 ? 1 : NV], s1[F64 ? 1 : L][F64 ? 1 : NV], s2[F64 ? 1 : L][F64 ? 1 : NV];
+  double fs[F64 ? L : 1][F64 ? NV : 1];
+  int64_t mn[MINMAX && !F64 ? L : 1][MINMAX && !F64 ? NV : 1], mx[MINMAX && !F64 ? L : 1][MINMAX && !F64 ? NV : 1];
+  double fmn[MINMAX && F64 ? L : 1][MINMAX && F64 ? NV : 1], fmx[MINMAX && F64 ? L : 1][MINMAX && F64 ? NV : 1];
+};
+
+template <int L, int NV, bool F64, bool MINMAX>
+__device__ __forceinline__ void reg_row(const Plan& p, uint64_t* dir, RegState<L, NV, F64, MINMAX>& st,
+                                        const RowIn<NV, F64>& x, int64_t r) {
+  bool m[L];
+  bool hit = false;
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    m[s] = x.key == st.rk[s];
+    hit = hit || m[s];
+  }
+  const bool special = x.key == ~0ULL;
+  bool go = x.q && x.fast && hit && !special;
+  if (x.q && !go) {                       // divergent, rare after warm-up
+    int slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, x.key) : -1;
+    if (slot >= 0) {
+#pragma unroll
+      for (int s = 0; s < L; ++s) {
+        st.rk[s] = ~*(volatile uint64_t*)&dir[s];
+        m[s] = s == slot;
+      }
+      go = true;
+    } else {
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+      if (e) update_entry_slow(p, e, r);
+    }
+  }
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    const bool mm = go && m[s];
+    st.cnt[s] += mm ? 1u : 0u;
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if constexpr (F64) {
+        if (mm) st.fs[s][v] += x.vd[v];
+        if constexpr (MINMAX) {
+          if (mm) {
+            st.fmn[s][v] = fmin(st.fmn[s][v], x.vd[v]);
+            st.fmx[s][v] = fmax(st.fmx[s][v], x.vd[v]);
+          }
+        }
+      } else {
+        add96(mm, st.s0[s][v], st.s1[s][v], st.s2[s][v], x.vi[v]);
+        if constexpr (MINMAX) {
+          if (mm) {
+            st.mn[s][v] = min(st.mn[s][v], x.vi[v]);
+            st.mx[s][v] = max(st.mx[s][v], x.vi[v]);
+          }
+        }
+      }
+    }
+  }
+}
+
+template <int L, int NV, bool F64, bool MINMAX, int U>
+__global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant__ Plan p) {
+  __shared__ uint64_t dir[L];
+  __shared__ __align__(16) uint64_t blk[L * 32];   // block accumulators, entry layout (stride <= 256 B)
+  const int lane = threadIdx.x & 31;
+  for (int i = threadIdx.x; i < L * 32; i += blockDim.x) blk[i] = 0;
+  if (threadIdx.x < L) dir[threadIdx.x] = 0;
+  __syncthreads();
+
+  RegState<L, NV, F64, MINMAX> st;
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    st.rk[s] = ~0ULL;
+    st.cnt[s] = 0;
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if constexpr (F64) {
+        st.fs[s][v] = 0.0;
+        if constexpr (MINMAX) { st.fmn[s][v] = __longlong_as_double(0x7FF0000000000000LL); st.fmx[s][v] = -st.fmn[s][v]; }
+      } else {
+        st.s0[s][v] = st.s1[s][v] = st.s2[s][v] = 0;
+        if constexpr (MINMAX) { st.mn[s][v] = INT64_MAX; st.mx[s][v] = INT64_MIN; }
+      }
+    }
+  }
+
+  constexpr int kTile = 64 * U;
+  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
+  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+  const int64_t ntiles = (p.n + kTile - 1) / kTile;
+  for (int64_t t = warp; t < ntiles; t += nwarps) {
+    const int64_t base = t * kTile;
+    if (p.vec_ok && base + kTile <= p.n) {
+#pragma unroll
+      for (int u = 0; u < U; ++u) {
+        const int64_t r = base + 64 * u + 2 * lane;
+        RowIn<NV, F64> x0, x1;
+        eval_pair_vec<NV, F64>(p, r, x0, x1);
+        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+        reg_row<L, NV, F64, MINMAX>(p, dir, st, x0, r);
+        reg_row<L, NV, F64, MINMAX>(p, dir, st, x1, r + 1);
+      }
+    } else {
+      for (int u = 0; u < U; ++u) {
+        const int64_t r = base + 64 * u + 2 * lane;
+        RowIn<NV, F64> x0, x1;
+        eval_row_scalar<NV, F64>(p, r, x0);
+        eval_row_scalar<NV, F64>(p, r + 1, x1);
+        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+        reg_row<L, NV, F64, MINMAX>(p, dir, st, x0, r);
+        reg_row<L, NV, F64, MINMAX>(p, dir, st, x1, r + 1);
+      }
+    }
+  }
+
+  // ---- flush: warp reduce -> shared block entry -> one global update per slot
+  __syncthreads();
+  uint8_t* blkb = (uint8_t*)blk;
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    if (dir[s] == 0) continue;                       // uniform: slot never used in this block
+    uint8_t* be = blkb + s * 256;
+    uint32_t c = __reduce_add_sync(0xffffffffu, st.cnt[s]);
+    if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)c);
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if (v >= p.nvals) break;
+      const DevValue& d = p.vals[v];
+      if constexpr (F64) {
+        double sum = st.fs[s][v];
+        for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
+        if (lane == 0 && d.off_sum >= 0) atomicAdd((double*)(be + d.off_sum), sum);
+        if constexpr (MINMAX) {
+          double a = st.fmn[s][v], b = st.fmx[s][v];
+          for (int o = 16; o > 0; o >>= 1) {
+            a = fmin(a, __shfl_xor_sync(0xffffffffu, a, o));
+            b = fmax(b, __shfl_xor_sync(0xffffffffu, b, o));
+          }
+          if (lane == 0 && c > 0) {
+            if (d.off_min >= 0) atomicMax((unsigned long long*)(be + d.off_min), (unsigned long long)enc_min_f(a));
+            if (d.off_max >= 0) atomicMax((unsigned long long*)(be + d.off_max), (unsigned long long)enc_max_f(b));
+          }
+        }
+      } else {
+        if (d.is_f64) continue;   // mixed plan: accumulated by the slow path only
+        I128 x;
+        x.lo = (uint64_t)st.s0[s][v] | ((uint64_t)st.s1[s][v] << 32);
+        x.hi = (uint64_t)(int64_t)(int32_t)st.s2[s][v];
+        x = warp_sum_i128(x);
+        if (lane == 0 && d.off_sum >= 0) atomic_add_i128((uint64_t*)(be + d.off_sum), x.lo, x.hi);
+        if constexpr (MINMAX) {
+          int64_t a = st.mn[s][v], b = st.mx[s][v];
+          for (int o = 16; o > 0; o >>= 1) {
+            a = min(a, (int64_t)__shfl_xor_sync(0xffffffffu, (long long)a, o));
+            b = max(b, (int64_t)__shfl_xor_sync(0xffffffffu, (long long)b, o));
+          }
+          if (lane == 0 && c > 0) {
+            if (d.off_min >= 0) atomicMax((unsigned long long*)(be + d.off_min), (unsigned long long)enc_min_i(a));
+            if (d.off_max >= 0) atomicMax((unsigned long long*)(be + d.off_max), (unsigned long long)enc_max_i(b));
+          }
+        }
+      }
+    }
+  }
+  __syncthreads();
+  // one thread per (slot, state word) pushes the block entry into the global table
+  if (threadIdx.x < L) {
+    const int s = threadIdx.x;
+    uint64_t sk = dir[s];
+    if (sk != 0) {
+      const uint8_t* be = blkb + s * 256;
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
+      if (e) {
+        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(be + 8));
+        for (int v = 0; v < p.nvals; ++v) {
+          const DevValue& d = p.vals[v];
+          if (d.off_sum >= 0) {
+            if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(be + d.off_sum));
+            else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(be + d.off_sum),
+                                 *(const uint64_t*)(be + d.off_sum + 8));
+          }
+          if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(be + d.off_min));
+          if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(be + d.off_max));
+        }
+      }
+    }
+  }
+}
+
+// ------------------------------------------------------------------ global tier
+template <int NV, bool F64>
+__device__ __forceinline__ void glb_row(const Plan& p, const RowIn<NV, F64>& x, int64_t r) {
+  if (!x.q) return;
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+  if (!e) return;
+  if (!x.fast) {
+    update_entry_slow(p, e, r);
+    return;
+  }
+  atomicAdd((unsigned long long*)(e + 8), 1ULL);
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (F64) {
+      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), x.vd[v]);
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(x.vd[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(x.vd[v]));
+    } else {
+      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)x.vi[v], (uint64_t)(x.vi[v] >> 63));
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(x.vi[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(x.vi[v]));
+    }
+  }
+}
+
+template <int NV, bool F64, int U>
+__global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant__ Plan p) {
+  const int lane = threadIdx.x & 31;
+  constexpr int kTile = 64 * U;
+  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
+  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+  const int64_t ntiles = (p.n + kTile - 1) / kTile;
+  for (int64_t t = warp; t < ntiles; t += nwarps) {
+    const int64_t base = t * kTile;
+    const bool vec = p.vec_ok && base + kTile <= p.n;
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      const int64_t r = base + 64 * u + 2 * lane;
+      RowIn<NV, F64> x0, x1;
+      if (vec) {
+        eval_pair_vec<NV, F64>(p, r, x0, x1);
+      } else {
+        eval_row_scalar<NV, F64>(p, r, x0);
+        eval_row_scalar<NV, F64>(p, r + 1, x1);
+      }
+      if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+      glb_row<NV, F64>(p, x0, r);
+      glb_row<NV, F64>(p, x1, r + 1);
+    }
+  }
+}
+
+// ------------------------------------------------------------------ dispatch
+constexpr int kRegSlots = 4;
+constexpr int kUnits = 2;
+
+template <int NV, bool F64, bool MM>
+static cudaError_t launch_reg_nv(const Plan& p, int grid, cudaStream_t s) {
+  count_launch();
+  k_sga_reg<kRegSlots, NV, F64, MM, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  return cudaGetLastError();
+}
+
+template <int NV, bool F64>
+static cudaError_t launch_reg_mm(const Plan& p, int grid, cudaStream_t s) {
+  return p.has_minmax ? launch_reg_nv<NV, F64, true>(p, grid, s) : launch_reg_nv<NV, F64, false>(p, grid, s);
+}
+
+template <bool F64>
+static cudaError_t launch_reg_f(const Plan& p, int grid, cudaStream_t s) {
+  if (p.nvals <= 1) return launch_reg_mm<1, F64>(p, grid, s);
+  if (p.nvals <= 2) return launch_reg_mm<2, F64>(p, grid, s);
+  if (p.nvals <= 4) return launch_reg_mm<4, F64>(p, grid, s);
+  return launch_reg_mm<6, F64>(p, grid, s);
+}
+
+template <bool F64>
+static cudaError_t launch_glb_f(const Plan& p, int grid, cudaStream_t s) {
+  if (p.nvals <= 1) { count_launch(); k_sga_glb<1, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
+  else if (p.nvals <= 2) { count_launch(); k_sga_glb<2, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
+  else if (p.nvals <= 4) { count_launch(); k_sga_glb<4, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
+  else { count_launch(); k_sga_glb<6, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
+  return cudaGetLastError();
+}
+
+int reg_tier_slots() { return kRegSlots; }
+
+template <int NV, bool F64>
+static const void* reg_kernel_ptr(bool mm) {
+  return mm ? (const void*)k_sga_reg<kRegSlots, NV, F64, true, kUnits> : (const void*)k_sga_reg<kRegSlots, NV, F64, false, kUnits>;
+}
+
+// Resident CTAs per SM of the instantiation launch_fused would pick (persistent grid sizing).
+int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64) {
+  const void* fn;
+  int nv = p.nvals <= 1 ? 1 : (p.nvals <= 2 ? 2 : (p.nvals <= 4 ? 4 : 6));
+  bool mm = p.has_minmax != 0;
+  if (reg_tier) {
+    if (values_f64) fn = nv == 1 ? reg_kernel_ptr<1, true>(mm) : nv == 2 ? reg_kernel_ptr<2, true>(mm) : nv == 4 ? reg_kernel_ptr<4, true>(mm) : reg_kernel_ptr<6, true>(mm);
+    else fn = nv == 1 ? reg_kernel_ptr<1, false>(mm) : nv == 2 ? reg_kernel_ptr<2, false>(mm) : nv == 4 ? reg_kernel_ptr<4, false>(mm) : reg_kernel_ptr<6, false>(mm);
+  } else {
+    if (values_f64) fn = nv == 1 ? (const void*)k_sga_glb<1, true, kUnits> : nv == 2 ? (const void*)k_sga_glb<2, true, kUnits> : nv == 4 ? (const void*)k_sga_glb<4, true, kUnits> : (const void*)k_sga_glb<6, true, kUnits>;
+    else fn = nv == 1 ? (const void*)k_sga_glb<1, false, kUnits> : nv == 2 ? (const void*)k_sga_glb<2, false, kUnits> : nv == 4 ? (const void*)k_sga_glb<4, false, kUnits> : (const void*)k_sga_glb<6, false, kUnits>;
+  }
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, 0) != cudaSuccess || nb < 1) nb = 1;
+  return nb;
+}
+
+// values_f64: all value expressions are fp64 (mixed int/fp64 plans use the
+// integer kernels, whose slow path handles fp64 values exactly too).
+cudaError_t launch_fused(const Plan& p, bool reg_tier, bool values_f64, int grid, cudaStream_t s) {
+  if (p.n == 0) return cudaSuccess;
+  int64_t tiles = (p.n + 64 * kUnits - 1) / (64 * kUnits);
+  int64_t g = (tiles + (kFusedThreads / 32) - 1) / (kFusedThreads / 32);
+  if (g > grid) g = grid;
+  if (reg_tier) return values_f64 ? launch_reg_f<true>(p, (int)g, s) : launch_reg_f<false>(p, (int)g, s);
+  return values_f64 ? launch_glb_f<true>(p, (int)g, s) : launch_glb_f<false>(p, (int)g, s);
+}
+
+}  // namespace ocl

@@ -1,0 +1,59 @@
+// launch.cuh — host-side launcher interface between abi.cu and the kernel files.
+#pragma once
+
+#include <atomic>
+
+#include "common.cuh"
+
+namespace ocl {
+// Kernel launches issued by this library (evidence for the benchmark's gpu_launches).
+extern std::atomic<unsigned long long> g_launches;
+inline void count_launch(unsigned long long k = 1) { g_launches.fetch_add(k, std::memory_order_relaxed); }
+
+struct SelParams {
+  const void* col;
+  int64_t n;
+  int32_t dtype;
+  int32_t is_f64;
+  int32_t anti;
+  int32_t vec_ok;      // column pointer 16-byte aligned
+  int64_t lo, hi;      // normalised inclusive bounds
+  double flo, fhi;
+  uint32_t* out;
+};
+struct EmitArgs {
+  int32_t kind;
+  FinPlan fin;
+  int64_t* keys_out;
+  int64_t out_capacity;
+  uint8_t* partial_out;
+  int32_t* status;
+};
+enum EmitKind : int32_t { EMIT_FINAL = 0, EMIT_GROUP_IDS = 1, EMIT_PARTIAL = 2 };
+
+cudaError_t launch_select_bitmap(const SelParams& p, int grid, cudaStream_t s);
+cudaError_t launch_bitmap_combine(int op, const uint32_t* a, const uint32_t* b, uint32_t* out, int64_t n, int grid,
+                                  cudaStream_t s);
+size_t prefix_compact_ws_bytes(int64_t n);
+cudaError_t launch_prefix_compact(const uint32_t* bitmap, int64_t n, uint32_t* oids, int64_t* m_out, void* ws,
+                                  int grid, cudaStream_t s);
+size_t emit_ws_bytes(int grid);
+cudaError_t launch_emit(uint8_t* table, uint64_t cap, int32_t stride, const EmitArgs& a, int64_t* ngroups_out,
+                        int64_t out_capacity, int32_t* status, bool sorted, void* ws, int grid, cudaStream_t s);
+bool sorted_emit_supported(uint64_t cap);
+cudaError_t launch_finalize_dense(const uint8_t* table, int32_t stride, const int64_t* ngroups, int64_t max_groups,
+                                  const FinPlan& f, int grid, cudaStream_t s);
+cudaError_t launch_group_insert(const Plan& p, int32_t* gid_out, int64_t max_rows, int grid, cudaStream_t s);
+cudaError_t launch_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
+                                int32_t* gid_out, int grid, cudaStream_t s);
+cudaError_t launch_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
+                          void* out, int grid, cudaStream_t s);
+cudaError_t launch_merge_partials(const uint8_t* partials, int32_t nparts, int64_t part_capacity,
+                                  const int64_t* part_counts, const FinPlan& f, uint8_t* table, uint64_t mask,
+                                  int32_t* status, int grid, cudaStream_t s);
+cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
+                                   int grid, cudaStream_t s);
+cudaError_t launch_fused(const Plan& p, bool reg_tier, bool values_f64, int grid, cudaStream_t s);
+int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64);
+int reg_tier_slots();
+}  // namespace ocl

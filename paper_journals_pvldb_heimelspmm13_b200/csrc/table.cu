@@ -1,0 +1,367 @@
+// table.cu — hash-table lifecycle: dense group ids from occupied slots,
+// finalisation of accumulator states into output columns (K10), group build
+// (K6 + K7), projection (K4), partial-table export and multi-GPU merge (K11).
+//
+// Paper: the hash table yields dense group ids (§4.1.6); after
+// the per-work-group aggregation "a single thread is scheduled per group to
+// compute the final aggregate" (L567-568 §4.1.7).  Here one thread per table
+// slot decodes the states (AVG = SUM / COUNT) and writes the dense output row.
+#include "launch.cuh"
+#include "rowops.cuh"
+
+namespace ocl {
+
+constexpr int kOccThreads = 256;
+constexpr int kSortSlots = 4096;   // order_by_key in one CTA up to this many table slots
+
+__device__ __forceinline__ bool slot_occupied(const uint8_t* table, uint64_t cap, int32_t stride, uint64_t i) {
+  return *(const uint64_t*)(table + i * (uint64_t)stride) != 0;   // side entry: occupancy flag
+}
+__device__ __forceinline__ uint64_t slot_key(const uint8_t* table, uint64_t cap, int32_t stride, uint64_t i) {
+  return i == cap ? ~0ULL : ~*(const uint64_t*)(table + i * (uint64_t)stride);
+}
+
+// ------------------------------------------------------------------ emitters
+// Decode one entry into output row g (finalize).
+__device__ __forceinline__ void emit_final(const FinPlan& f, const uint8_t* e, uint64_t key, int64_t g) {
+  if (g >= f.out_capacity) return;
+  if (f.keys_out) f.keys_out[g] = (int64_t)key;
+  const uint64_t count = *(const uint64_t*)(e + 8);
+  for (int i = 0; i < f.naggs; ++i) {
+    const OutAgg& a = f.aggs[i];
+    const uint8_t* s = e + a.off;
+    switch (a.op) {
+      case OCL_AGG_COUNT: ((int64_t*)a.out)[g] = (int64_t)count; break;
+      case OCL_AGG_SUM:
+        if (a.is_f64) ((double*)a.out)[g] = *(const double*)s;
+        else {
+          ((uint64_t*)a.out)[2 * g] = *(const uint64_t*)s;
+          ((uint64_t*)a.out)[2 * g + 1] = *(const uint64_t*)(s + 8);
+        }
+        break;
+      case OCL_AGG_AVG: {
+        double sum = a.is_f64 ? *(const double*)s : i128_to_double(*(const uint64_t*)s, *(const uint64_t*)(s + 8));
+        ((double*)a.out)[g] = __ddiv_rn(sum, __ull2double_rn(count));
+        break;
+      }
+      case OCL_AGG_MIN:
+        if (a.is_f64) ((double*)a.out)[g] = dec_min_f(*(const uint64_t*)s);
+        else ((int64_t*)a.out)[g] = dec_min_i(*(const uint64_t*)s);
+        break;
+      case OCL_AGG_MAX:
+        if (a.is_f64) ((double*)a.out)[g] = dec_max_f(*(const uint64_t*)s);
+        else ((int64_t*)a.out)[g] = dec_max_i(*(const uint64_t*)s);
+        break;
+    }
+  }
+}
+
+__device__ __forceinline__ void emit_slot(const EmitArgs& a, uint8_t* e, uint64_t key, int64_t g, int32_t stride) {
+  if (a.kind == EMIT_FINAL) {
+    emit_final(a.fin, e, key, g);
+  } else if (a.kind == EMIT_GROUP_IDS) {
+    *(int64_t*)(e + 8) = g;                         // slot -> dense gid (read by k_group_lookup)
+    if (g < a.out_capacity && a.keys_out) a.keys_out[g] = (int64_t)key;
+  } else if (g < a.out_capacity) {
+    uint64_t* dst = (uint64_t*)(a.partial_out + g * (int64_t)stride);
+    const uint64_t* src = (const uint64_t*)e;
+    dst[0] = key;
+    for (int w = 1; w < stride / 8; ++w) dst[w] = src[w];
+  }
+}
+
+// ------------------------------------------------------------------ occupied-slot compaction
+// Pass 1: occupied slots per CTA chunk.  Pass 2: exclusive scan (one CTA).
+// Pass 3: ordered rank inside each chunk -> emit.  Deterministic slot order.
+__global__ void __launch_bounds__(kOccThreads) k_occ_count(const uint8_t* table, uint64_t cap, int32_t stride,
+                                                           uint64_t chunk, uint32_t* counts) {
+  const uint64_t nslots = cap + 1;
+  uint64_t b0 = blockIdx.x * chunk, b1 = b0 + chunk < nslots ? b0 + chunk : nslots;
+  uint32_t c = 0;
+  for (uint64_t i = b0 + threadIdx.x; i < b1; i += blockDim.x) c += slot_occupied(table, cap, stride, i) ? 1u : 0u;
+  c = __reduce_add_sync(0xffffffffu, c);
+  __shared__ uint32_t ws[kOccThreads / 32];
+  if ((threadIdx.x & 31) == 0) ws[threadIdx.x >> 5] = c;
+  __syncthreads();
+  if (threadIdx.x == 0) {
+    uint32_t t = 0;
+    for (int w = 0; w < kOccThreads / 32; ++w) t += ws[w];
+    counts[blockIdx.x] = t;
+  }
+}
+
+__global__ void __launch_bounds__(1024) k_occ_scan(const uint32_t* counts, int nblocks, uint64_t* offsets,
+                                                   int64_t* ngroups_out, int64_t out_capacity, int32_t* status) {
+  __shared__ uint64_t carry;
+  __shared__ uint64_t wsum[32];
+  if (threadIdx.x == 0) carry = 0;
+  __syncthreads();
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  for (int base = 0; base < nblocks; base += 1024) {
+    int i = base + threadIdx.x;
+    uint64_t v = i < nblocks ? counts[i] : 0;
+    uint64_t incl = v;
+    for (int o = 1; o < 32; o <<= 1) {
+      uint64_t y = __shfl_up_sync(0xffffffffu, incl, o);
+      if (lane >= o) incl += y;
+    }
+    if (lane == 31) wsum[warp] = incl;
+    __syncthreads();
+    uint64_t woff = 0;
+    for (int w = 0; w < warp; ++w) woff += wsum[w];
+    uint64_t c0 = carry;
+    if (i < nblocks) offsets[i] = c0 + woff + incl - v;
+    __syncthreads();
+    if (threadIdx.x == 1023) carry = c0 + woff + incl;
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) {
+    if (ngroups_out) *ngroups_out = (int64_t)carry;
+    if ((int64_t)carry > out_capacity) set_status(status, OCL_ERR_CAPACITY);
+  }
+}
+
+__global__ void __launch_bounds__(kOccThreads) k_occ_emit(uint8_t* table, uint64_t cap, int32_t stride, uint64_t chunk,
+                                                          const uint64_t* offsets, const __grid_constant__ EmitArgs a) {
+  __shared__ uint32_t ws[kOccThreads / 32];
+  const uint64_t nslots = cap + 1;
+  uint64_t b0 = blockIdx.x * chunk, b1 = b0 + chunk < nslots ? b0 + chunk : nslots;
+  uint64_t base = offsets[blockIdx.x];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  for (uint64_t s0 = b0; s0 < b1; s0 += blockDim.x) {
+    uint64_t i = s0 + threadIdx.x;
+    bool occ = i < b1 && slot_occupied(table, cap, stride, i);
+    uint32_t bal = __ballot_sync(0xffffffffu, occ);
+    if (lane == 0) ws[warp] = __popc(bal);
+    __syncthreads();
+    uint32_t woff = 0, tot = 0;
+    for (int w = 0; w < kOccThreads / 32; ++w) {
+      woff += w < warp ? ws[w] : 0;
+      tot += ws[w];
+    }
+    if (occ) {
+      int64_t g = (int64_t)(base + woff + __popc(bal & ((1u << lane) - 1)));
+      emit_slot(a, table + i * (uint64_t)stride, slot_key(table, cap, stride, i), g, stride);
+    }
+    base += tot;
+    __syncthreads();
+  }
+}
+
+// order_by_key: one CTA gathers the occupied slots, bitonic-sorts (key, slot), emits.
+__global__ void __launch_bounds__(1024) k_sorted_emit(uint8_t* table, uint64_t cap, int32_t stride,
+                                                      int64_t* ngroups_out, int64_t out_capacity, int32_t* status,
+                                                      const __grid_constant__ EmitArgs a) {
+  __shared__ uint64_t skey[kSortSlots];
+  __shared__ uint16_t sslot[kSortSlots];
+  __shared__ uint32_t cnt;
+  if (threadIdx.x == 0) cnt = 0;
+  __syncthreads();
+  for (uint64_t i = threadIdx.x; i <= cap; i += blockDim.x) {
+    if (slot_occupied(table, cap, stride, i)) {
+      uint32_t k = atomicAdd(&cnt, 1u);
+      skey[k] = slot_key(table, cap, stride, i);
+      sslot[k] = (uint16_t)i;
+    }
+  }
+  __syncthreads();
+  const uint32_t G = cnt;
+  uint32_t P = 1;
+  while (P < G) P <<= 1;
+  for (uint32_t i = G + threadIdx.x; i < P; i += blockDim.x) {
+    skey[i] = ~0ULL;
+    sslot[i] = 0xFFFF;        // padding sorts after a real ~0 key (slots < kSortSlots)
+  }
+  __syncthreads();
+  for (uint32_t k = 2; k <= P; k <<= 1) {
+    for (uint32_t j = k >> 1; j > 0; j >>= 1) {
+      for (uint32_t i = threadIdx.x; i < P; i += blockDim.x) {
+        uint32_t ixj = i ^ j;
+        if (ixj > i) {
+          bool up = (i & k) == 0;
+          uint64_t ka = skey[i], kb = skey[ixj];
+          uint16_t sa = sslot[i], sb = sslot[ixj];
+          bool gt = ka > kb || (ka == kb && sa > sb);
+          if (gt == up) {
+            skey[i] = kb; skey[ixj] = ka;
+            sslot[i] = sb; sslot[ixj] = sa;
+          }
+        }
+      }
+      __syncthreads();
+    }
+  }
+  for (uint32_t g = threadIdx.x; g < G; g += blockDim.x)
+    emit_slot(a, table + (uint64_t)sslot[g] * stride, skey[g], g, stride);
+  if (threadIdx.x == 0) {
+    if (ngroups_out) *ngroups_out = G;
+    if ((int64_t)G > out_capacity) set_status(status, OCL_ERR_CAPACITY);
+  }
+}
+
+// Unfused aggregate finalisation: table indexed directly by gid, g < *ngroups.
+__global__ void k_finalize_dense(const uint8_t* table, int32_t stride, const int64_t* ngroups, int64_t max_groups,
+                                 const __grid_constant__ FinPlan f) {
+  int64_t G = ngroups ? *ngroups : max_groups;
+  if (G > max_groups) G = max_groups;
+  for (int64_t g = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; g < G; g += (int64_t)gridDim.x * blockDim.x)
+    emit_final(f, table + g * stride, 0, g);
+}
+
+// ------------------------------------------------------------------ group build (K6/K7)
+__global__ void k_group_insert(const __grid_constant__ Plan p, int32_t* gid_out, int64_t max_rows) {
+  const int64_t m = p.m_dev ? *p.m_dev : max_rows;
+  for (int64_t j0 = blockIdx.x * (int64_t)blockDim.x; j0 < m; j0 += (int64_t)gridDim.x * blockDim.x) {
+    int64_t j = j0 + threadIdx.x;
+    bool act = j < m;
+    unsigned amask = __ballot_sync(0xffffffffu, act);
+    if (!act) continue;
+    int64_t r = p.oids ? (int64_t)p.oids[j] : j;
+    uint64_t key = row_key_scalar(p, r);
+    // warp-aggregated insert: one probe per distinct key per warp
+    unsigned peers = __match_any_sync(amask, key);
+    int leader = __ffs(peers) - 1;
+    int64_t slot = -1;
+    if ((threadIdx.x & 31) == leader) {
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
+      slot = e ? (int64_t)((e - p.table) / p.stride) : -1;
+    }
+    slot = __shfl_sync(amask, slot, leader);
+    gid_out[j] = (int32_t)slot;
+  }
+}
+
+__global__ void k_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
+                               int32_t* gid_out) {
+  const int64_t m = m_dev ? *m_dev : max_rows;
+  for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
+    int32_t s = gid_out[j];
+    gid_out[j] = s >= 0 ? (int32_t)*(const int64_t*)(table + (int64_t)s * stride + 8) : -1;
+  }
+}
+
+// ------------------------------------------------------------------ projection (K4)
+__global__ void k_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
+                         void* out) {
+  int64_t m = m_dev ? *m_dev : max_m;
+  if (m > max_m) m = max_m;
+  for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
+    uint32_t r = __ldg(oids + j);
+    if (width == 1) ((uint8_t*)out)[j] = __ldg((const uint8_t*)col + r);
+    else if (width == 4) ((int32_t*)out)[j] = __ldg((const int32_t*)col + r);
+    else ((long long*)out)[j] = __ldg((const long long*)col + r);
+  }
+}
+
+// ------------------------------------------------------------------ merge partials (K11)
+__global__ void k_merge_partials(const uint8_t* partials, int32_t nparts, int64_t part_capacity,
+                                 const int64_t* part_counts, const __grid_constant__ FinPlan f, uint8_t* table,
+                                 uint64_t mask, int32_t* status) {
+  const int32_t stride = f.stride;
+  for (int32_t part = 0; part < nparts; ++part) {
+    int64_t cnt = part_counts[part];
+    if (cnt > part_capacity) cnt = part_capacity;
+    for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < cnt; j += (int64_t)gridDim.x * blockDim.x) {
+      const uint8_t* row = partials + ((int64_t)part * part_capacity + j) * stride;
+      uint64_t key = *(const uint64_t*)row;
+      uint8_t* e = table_find_or_insert(table, mask, stride, key, status);
+      if (!e) continue;
+      atomicAdd((unsigned long long*)(e + 8), *(const unsigned long long*)(row + 8));
+      for (int s = 0; s < f.nstates; ++s) {
+        const StateDesc& d = f.states[s];
+        const uint8_t* src = row + d.off;
+        uint8_t* dst = e + d.off;
+        if (d.kind == ACC_SUM_I) atomic_add_i128((uint64_t*)dst, *(const uint64_t*)src, *(const uint64_t*)(src + 8));
+        else if (d.kind == ACC_SUM_F) atomicAdd((double*)dst, *(const double*)src);
+        else atomicMax((unsigned long long*)dst, *(const unsigned long long*)src);
+      }
+    }
+  }
+}
+
+// ------------------------------------------------------------------ host launchers
+static uint64_t occ_chunk(uint64_t nslots, int grid, int* nblocks) {
+  uint64_t chunk = (nslots + grid - 1) / grid;
+  chunk = (chunk + kOccThreads - 1) / kOccThreads * kOccThreads;
+  if (chunk < kOccThreads) chunk = kOccThreads;
+  *nblocks = (int)((nslots + chunk - 1) / chunk);
+  return chunk;
+}
+
+size_t emit_ws_bytes(int grid) { return (size_t)grid * 16 + 256; }
+
+// Emit all occupied slots of a table (cap = mask + 1) in slot order (or key order).
+cudaError_t launch_emit(uint8_t* table, uint64_t cap, int32_t stride, const EmitArgs& a, int64_t* ngroups_out,
+                        int64_t out_capacity, int32_t* status, bool sorted, void* ws, int grid, cudaStream_t s) {
+  if (sorted) {
+    if (cap + 1 > (uint64_t)kSortSlots) return cudaErrorInvalidValue;
+    count_launch();
+    k_sorted_emit<<<1, 1024, 0, s>>>(table, cap, stride, ngroups_out, out_capacity, status, a);
+    return cudaGetLastError();
+  }
+  int nblocks = 0;
+  uint64_t chunk = occ_chunk(cap + 1, grid, &nblocks);
+  uint32_t* counts = (uint32_t*)ws;
+  uint64_t* offsets = (uint64_t*)((uint8_t*)ws + (((size_t)grid * 4 + 255) / 256) * 256);
+  count_launch();
+  k_occ_count<<<nblocks, kOccThreads, 0, s>>>(table, cap, stride, chunk, counts);
+  count_launch();
+  k_occ_scan<<<1, 1024, 0, s>>>(counts, nblocks, offsets, ngroups_out, out_capacity, status);
+  count_launch();
+  k_occ_emit<<<nblocks, kOccThreads, 0, s>>>(table, cap, stride, chunk, offsets, a);
+  return cudaGetLastError();
+}
+
+bool sorted_emit_supported(uint64_t cap) { return cap + 1 <= (uint64_t)kSortSlots; }
+
+cudaError_t launch_finalize_dense(const uint8_t* table, int32_t stride, const int64_t* ngroups, int64_t max_groups,
+                                  const FinPlan& f, int grid, cudaStream_t s) {
+  if (max_groups == 0) return cudaSuccess;
+  int64_t g = (max_groups + 255) / 256;
+  if (g > grid) g = grid;
+  count_launch();
+  k_finalize_dense<<<(int)g, 256, 0, s>>>(table, stride, ngroups, max_groups, f);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_group_insert(const Plan& p, int32_t* gid_out, int64_t max_rows, int grid, cudaStream_t s) {
+  if (max_rows == 0) return cudaSuccess;
+  int64_t g = (max_rows + 255) / 256;
+  if (g > grid) g = grid;
+  count_launch();
+  k_group_insert<<<(int)g, 256, 0, s>>>(p, gid_out, max_rows);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
+                                int32_t* gid_out, int grid, cudaStream_t s) {
+  if (max_rows == 0) return cudaSuccess;
+  int64_t g = (max_rows + 255) / 256;
+  if (g > grid) g = grid;
+  count_launch();
+  k_group_lookup<<<(int)g, 256, 0, s>>>(table, stride, m_dev, max_rows, gid_out);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
+                          void* out, int grid, cudaStream_t s) {
+  if (max_m == 0) return cudaSuccess;
+  int64_t g = (max_m + 255) / 256;
+  if (g > grid) g = grid;
+  count_launch();
+  k_gather<<<(int)g, 256, 0, s>>>(col, width, oids, m_dev, max_m, out);
+  return cudaGetLastError();
+}
+
+cudaError_t launch_merge_partials(const uint8_t* partials, int32_t nparts, int64_t part_capacity,
+                                  const int64_t* part_counts, const FinPlan& f, uint8_t* table, uint64_t mask,
+                                  int32_t* status, int grid, cudaStream_t s) {
+  if (nparts == 0 || part_capacity == 0) return cudaSuccess;
+  int64_t g = (part_capacity + 255) / 256;
+  if (g > grid) g = grid;
+  count_launch();
+  k_merge_partials<<<(int)g, 256, 0, s>>>(partials, nparts, part_capacity, part_counts, f, table, mask, status);
+  return cudaGetLastError();
+}
+
+}  // namespace ocl
