@@ -11,10 +11,18 @@ CHDR      := $(wildcard $(PKG)/csrc/*.cuh) include/ocelot_b200.h
 
 all: $(LIB) oracle/liboracle.so datagen/liboclgen_host.so datagen/liboclgen_dev.so
 
+OBJDIR    := build/obj
+COBJ      := $(patsubst $(PKG)/csrc/%.cu,$(OBJDIR)/%.o,$(CSRC))
+
 # product library: hand-written CUDA kernels + C ABI (no torch types)
-$(LIB): $(CSRC) $(CHDR)
+$(OBJDIR)/%.o: $(PKG)/csrc/%.cu $(CHDR)
+	@mkdir -p $(OBJDIR)
+	$(NVCC) $(NVFLAGS) -Iinclude -c -o $@ $< 2> $(OBJDIR)/$*.ptxas.log || (cat $(OBJDIR)/$*.ptxas.log; exit 1)
+
+$(LIB): $(COBJ)
 	@mkdir -p $(PKG)/_lib
-	$(NVCC) $(NVFLAGS) -Iinclude -shared -o $@ $(CSRC) -lcudart 2> $(PKG)/_lib/ptxas.log || (cat $(PKG)/_lib/ptxas.log; exit 1)
+	$(NVCC) $(ARCH) -shared -o $@ $(COBJ) -lcudart
+	@cat $(OBJDIR)/*.ptxas.log > $(PKG)/_lib/ptxas.log
 
 # oracle: test infrastructure only; plain C++17, single-threaded, no FMA contraction
 oracle/liboracle.so: oracle/oracle.cpp oracle/oracle.h
@@ -28,6 +36,7 @@ datagen/liboclgen_dev.so: datagen/datagen_dev.cu datagen/ocl_datagen.h
 	$(NVCC) $(ARCH) -O3 -Xcompiler -fPIC -shared -o $@ datagen/datagen_dev.cu -lcudart
 
 clean:
+	rm -rf $(OBJDIR)
 	rm -f $(LIB) oracle/liboracle.so datagen/liboclgen_host.so datagen/liboclgen_dev.so
 
 .PHONY: all clean

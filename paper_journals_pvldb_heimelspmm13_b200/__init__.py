@@ -405,7 +405,7 @@ def select_group_aggregate(preds, keys, vals, aggs, expected_groups=4, out_capac
             if e.status != OCL_ERR_CAPACITY:
                 raise
             G = int(call.ngroups.item())
-            eg = max(2 * eg, G)
+            eg = max(4 * eg, 2 * G)              # table full -> G reads as the capacity: grow geometrically
             if out_capacity is not None and out_capacity < G:
                 out_capacity = G
     raise OcelotError(OCL_ERR_CAPACITY, "hash table still full after retries")

@@ -21,6 +21,7 @@ std::atomic<unsigned long long> g_launches{0};
 
 struct ocl_ctx {
   cudaEvent_t prof_begin = nullptr, prof_end = nullptr;   // optional: bracket the fused kernel
+  int last_kernel = 0;                                     // 0 generic, >0 specialised signature id
   int device;
   int sms;
   int grid;                 // generic grid-stride kernels
@@ -311,7 +312,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
 }
 
 bool use_reg_tier(const ocl_sga_args* a) {
-  if (a->tier == 1) return true;
+  if (a->tier == 1 || a->tier == 3) return true;
   if (a->tier == 2) return false;
   return a->expected_groups <= reg_tier_slots();
 }
@@ -334,9 +335,13 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   if (a->dev_status) OCL_CUDA(cudaMemsetAsync(a->dev_status, 0, sizeof(int32_t), s), "status init");
   if (P.plan.n > 0) {
     bool reg = use_reg_tier(a);
-    int grid = fused_grid(ctx, P, reg);
     if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, s), "profile event");
-    OCL_CUDA(launch_fused(P.plan, reg, P.values_f64, grid, s), "fused kernel launch");
+    cudaError_t err = cudaSuccess;
+    int kind = 0;
+    if (!(reg && a->tier != 3 && launch_fused_spec(P.plan, ctx->sms, s, &err, &kind)))
+      err = launch_fused(P.plan, reg, P.values_f64, fused_grid(ctx, P, reg), s);
+    OCL_CUDA(err, "fused kernel launch");
+    ctx->last_kernel = kind;
     if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, s), "profile event");
   }
   return OCL_OK;

@@ -56,4 +56,6 @@ cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_
 cudaError_t launch_fused(const Plan& p, bool reg_tier, bool values_f64, int grid, cudaStream_t s);
 int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64);
 int reg_tier_slots();
+// Plan-specialised register-tier kernels (fused_spec.cu); false if no signature matches.
+bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 }  // namespace ocl

@@ -131,4 +131,43 @@ __device__ __forceinline__ void update_entry_slow(const Plan& p, uint8_t* e, int
   }
 }
 
+
+__device__ __forceinline__ I128 warp_sum_i128(I128 x) {
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) {
+    I128 y;
+    y.lo = __shfl_xor_sync(0xffffffffu, x.lo, o);
+    y.hi = __shfl_xor_sync(0xffffffffu, x.hi, o);
+    x = i128_add(x, y);
+  }
+  return x;
+}
+
+// Block-wide slot directory: stored keys (~key), 0 = free.  Returns slot or -1.
+template <int L>
+__device__ __forceinline__ int dir_find_or_insert(uint64_t* dir, uint64_t key) {
+  uint64_t sk = ~key;
+#pragma unroll
+  for (int s = 0; s < L; ++s) {
+    uint64_t cur = *(volatile uint64_t*)&dir[s];
+    if (cur == sk) return s;
+    if (cur == 0) {
+      uint64_t prev = atomicCAS((unsigned long long*)&dir[s], 0ULL, (unsigned long long)sk);
+      if (prev == 0 || prev == sk) return s;
+    }
+  }
+  return -1;
+}
+
+// Optional bitmap output for a 64-row unit: rows base + 2*lane + {0,1}.
+__device__ __forceinline__ void emit_bitmap_unit(const Plan& p, int64_t base, int lane, bool q0, bool q1) {
+  uint32_t b = (uint32_t)q0 | ((uint32_t)q1 << 1);
+  uint32_t w0 = __reduce_or_sync(0xffffffffu, lane < 16 ? b << (2 * lane) : 0u);
+  uint32_t w1 = __reduce_or_sync(0xffffffffu, lane >= 16 ? b << (2 * (lane - 16)) : 0u);
+  int64_t words = (p.n + 31) >> 5;
+  int64_t wi = base >> 5;
+  if (lane == 0 && wi < words) p.bitmap_out[wi] = w0;
+  if (lane == 1 && wi + 1 < words) p.bitmap_out[wi + 1] = w1;
+}
+
 }  // namespace ocl
