@@ -93,6 +93,12 @@ __device__ __forceinline__ uint64_t ld1(const void* base, int64_t r) {
   else return (uint64_t)__ldg((const long long*)base + r);
 }
 
+__device__ __forceinline__ int64_t mul_wide_s32(int32_t a, int32_t b) {
+  int64_t r;
+  asm("mul.wide.s32 %0, %1, %2;" : "=l"(r) : "r"(a), "r"(b));
+  return r;
+}
+
 template <class S>
 using KeyT = typename std::conditional<(S::KBITS <= 32), uint32_t, uint64_t>::type;
 
@@ -140,11 +146,11 @@ __device__ __forceinline__ void spec_values(const SpecPlan& p, const uint64_t (&
       } else {
         int64_t t = (int64_t)((uint64_t)p.g.vals[v].S - c[vx_b(op)]);
         x.fast = x.fast && fits_i32(a) && fits_i32(t);
-        int64_t e = (int64_t)(int32_t)a * (int64_t)(int32_t)t;
+        int64_t e = mul_wide_s32((int32_t)a, (int32_t)t);
         if (kind == VX_M1P) {
           int64_t u = (int64_t)((uint64_t)p.g.vals[v].S + c[vx_c(op)]);
           x.fast = x.fast && fits_i32(e) && fits_i32(u);
-          e = (int64_t)(int32_t)e * (int64_t)(int32_t)u;
+          e = mul_wide_s32((int32_t)e, (int32_t)u);
         }
         x.vi[v] = e;
       }
@@ -152,29 +158,41 @@ __device__ __forceinline__ void spec_values(const SpecPlan& p, const uint64_t (&
   }
 }
 
-// Predicated accumulate helpers (one predicate, carry chain).
-__device__ __forceinline__ void add64_i32(bool pr, uint32_t& lo, uint32_t& hi, int32_t v) {
-  asm("{\n\t.reg .pred p;\n\tsetp.ne.u32 p, %2, 0;\n\t"
-      "@p add.cc.u32 %0, %0, %3;\n\t@p addc.u32 %1, %1, %4;\n\t}"
-      : "+r"(lo), "+r"(hi)
-      : "r"((uint32_t)pr), "r"((uint32_t)v), "r"((uint32_t)(v >> 31)));
-}
-__device__ __forceinline__ void add96_i64(bool pr, uint32_t& a0, uint32_t& a1, uint32_t& a2, int64_t v) {
-  asm("{\n\t.reg .pred p;\n\tsetp.ne.u32 p, %3, 0;\n\t"
-      "@p add.cc.u32 %0, %0, %4;\n\t@p addc.cc.u32 %1, %1, %5;\n\t@p addc.u32 %2, %2, %6;\n\t}"
-      : "+r"(a0), "+r"(a1), "+r"(a2)
-      : "r"((uint32_t)pr), "r"((uint32_t)(uint64_t)v), "r"((uint32_t)((uint64_t)v >> 32)),
-        "r"((uint32_t)(v >> 63)));
-}
-
-constexpr int kSpecSlots = 4;
+// ------------------------------------------------------------------ private accumulators
+// Low-G tier: every thread owns one accumulator set per group slot, laid out in
+// shared memory as [slot][accumulator][thread] (conflict-free: lane t always hits
+// the same banks whatever its slot).  A row costs one slot-indexed read-modify-
+// write per accumulator — no atomics, no per-slot predication — the limit of the
+// paper's "multiple accumulators per group" in local memory.
+//   count      u32   (rows per thread < 2^32)
+//   COL value  i64   (fast path: the value fits int32, so < 2^32 of them fit)
+//   product    96-bit = u64 lo [..] + u32 hi [..] (fast-path products < 2^62)
+//   fp64       double
+constexpr int kPrivThreads = 256;
+constexpr int kPrivSlots = 4;
 
 template <class S>
-struct SState {
-  KeyT<S> rk[kSpecSlots];
-  uint32_t cnt[kSpecSlots];
-  uint32_t a0[kSpecSlots][S::NV], a1[kSpecSlots][S::NV], a2[kSpecSlots][S::NV];   // int class
-  double fs[S::F64 ? kSpecSlots : 1][S::F64 ? S::NV : 1];
+struct Acc {
+  static constexpr int nnar() {
+    int c = 0;
+    for (int v = 0; v < S::NV; ++v) c += vx_kind(S::OP(v)) == VX_COL ? 1 : 0;
+    return c;
+  }
+  static constexpr int NNAR = S::F64 ? 0 : nnar();
+  static constexpr int NWIDE = S::F64 ? 0 : S::NV - nnar();
+  static constexpr int NDBL = S::F64 ? S::NV : 0;
+  __host__ __device__ static constexpr int nar_idx(int v) {
+    int c = 0;
+    for (int i = 0; i < v; ++i) c += vx_kind(S::OP(i)) == VX_COL ? 1 : 0;
+    return c;
+  }
+  __host__ __device__ static constexpr int wide_idx(int v) { return v - nar_idx(v); }
+  // byte offsets of the arrays for L slots and T threads
+  static constexpr size_t off_nar(int L, int T) { return (size_t)4 * L * T; }
+  static constexpr size_t off_wlo(int L, int T) { return off_nar(L, T) + (size_t)8 * L * NNAR * T; }
+  static constexpr size_t off_whi(int L, int T) { return off_wlo(L, T) + (size_t)8 * L * NWIDE * T; }
+  static constexpr size_t off_dbl(int L, int T) { return off_whi(L, T) + (size_t)4 * L * NWIDE * T; }
+  static constexpr size_t bytes(int L, int T) { return off_dbl(L, T) + (size_t)8 * L * NDBL * T; }
 };
 
 template <class S>
@@ -183,27 +201,53 @@ __device__ __forceinline__ bool spec_is_special(KeyT<S> k) {
   else return k == (KeyT<S>)~0ULL;   // never placed in a slot (64-bit key ~0, or 32-bit sentinel)
 }
 
-template <class S>
-__device__ __forceinline__ void spec_row(const SpecPlan& p, uint64_t* dir, SState<S>& st, const SRow<S>& x,
-                                         int64_t r) {
-  constexpr int L = kSpecSlots;
-  bool m[L];
-  bool hit = false;
+template <class S, int L>
+__device__ __forceinline__ void priv_add(uint8_t* sm, int slot, int tid, const SRow<S>& x) {
+  using A = Acc<S>;
+  constexpr int T = kPrivThreads;
+  uint32_t* cnt = (uint32_t*)sm;
+  cnt[slot * T + tid] += 1u;
 #pragma unroll
-  for (int s = 0; s < L; ++s) {
-    m[s] = x.key == st.rk[s];
-    hit = hit || m[s];
+  for (int v = 0; v < S::NV; ++v) {
+    if constexpr (S::F64) {
+      double* d = (double*)(sm + A::off_dbl(L, T));
+      d[(slot * S::NV + v) * T + tid] += x.vd[v];
+    } else if (vx_kind(S::OP(v)) == VX_COL) {
+      int64_t* a = (int64_t*)(sm + A::off_nar(L, T));
+      a[(slot * A::NNAR + A::nar_idx(v)) * T + tid] += (int64_t)(int32_t)x.vi[v];
+    } else {
+      const int k = (slot * A::NWIDE + A::wide_idx(v)) * T + tid;
+      uint64_t* lo = (uint64_t*)(sm + A::off_wlo(L, T));
+      uint32_t* hi = (uint32_t*)(sm + A::off_whi(L, T));
+      uint64_t l = lo[k];
+      uint32_t h = hi[k];
+      uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
+      asm("add.cc.u32 %0, %0, %3;\n\taddc.cc.u32 %1, %1, %4;\n\taddc.u32 %2, %2, %5;"
+          : "+r"(l0), "+r"(l1), "+r"(h)
+          : "r"((uint32_t)(uint64_t)x.vi[v]), "r"((uint32_t)((uint64_t)x.vi[v] >> 32)),
+            "r"((uint32_t)(x.vi[v] >> 63)));
+      lo[k] = (uint64_t)l0 | ((uint64_t)l1 << 32);
+      hi[k] = h;
+    }
   }
+}
+
+template <class S, int L>
+__device__ __forceinline__ void priv_row(const SpecPlan& p, uint64_t* dir, KeyT<S> (&rk)[L], uint8_t* sm, int tid,
+                                         const SRow<S>& x, int64_t r) {
+  int slot = -1;
+#pragma unroll
+  for (int s = L - 1; s >= 0; --s)
+    if (x.key == rk[s]) slot = s;
   const bool special = spec_is_special<S>(x.key);
-  bool go = x.q && x.fast && hit && !special;
+  bool go = x.q && x.fast && slot >= 0 && !special;
   if (x.q && !go) {                                    // rare: new key in this CTA, or slow value
-    int slot = (x.fast && !special) ? dir_find_or_insert<kSpecSlots>(dir, (uint64_t)x.key) : -1;
+    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, (uint64_t)x.key) : -1;
     if (slot >= 0) {
 #pragma unroll
       for (int s = 0; s < L; ++s) {
         uint64_t sk = *(volatile uint64_t*)&dir[s];
-        st.rk[s] = sk ? (KeyT<S>)~sk : (KeyT<S>)~0ULL;
-        m[s] = s == slot;
+        rk[s] = sk ? (KeyT<S>)~sk : (KeyT<S>)~0ULL;
       }
       go = true;
     } else {
@@ -211,21 +255,7 @@ __device__ __forceinline__ void spec_row(const SpecPlan& p, uint64_t* dir, SStat
       if (e) update_entry_slow(p.g, e, r);
     }
   }
-#pragma unroll
-  for (int s = 0; s < L; ++s) {
-    const bool mm = go && m[s];
-    st.cnt[s] += mm ? 1u : 0u;
-#pragma unroll
-    for (int v = 0; v < S::NV; ++v) {
-      if constexpr (S::F64) {
-        if (mm) st.fs[s][v] += x.vd[v];
-      } else if (vx_kind(S::OP(v)) == VX_COL) {
-        add64_i32(mm, st.a0[s][v], st.a1[s][v], (int32_t)x.vi[v]);
-      } else {
-        add96_i64(mm, st.a0[s][v], st.a1[s][v], st.a2[s][v], x.vi[v]);
-      }
-    }
-  }
+  if (go) priv_add<S, L>(sm, slot, tid, x);
 }
 
 template <class S>
@@ -245,36 +275,34 @@ __device__ __forceinline__ void spec_row_scalar(const SpecPlan& p, int64_t r, SR
   spec_values<S>(p, c, x);
 }
 
-template <class S>
-__global__ void __launch_bounds__(256, 2) k_sga_reg_spec(const __grid_constant__ SpecPlan p) {
-  constexpr int L = kSpecSlots;
+template <class S, int L>
+__global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant__ SpecPlan p) {
+  using A = Acc<S>;
+  constexpr int T = kPrivThreads;
+  extern __shared__ __align__(16) uint8_t sm[];
   __shared__ uint64_t dir[L];
   __shared__ __align__(16) uint64_t blk[L * 32];
-  const int lane = threadIdx.x & 31;
-  for (int i = threadIdx.x; i < L * 32; i += blockDim.x) blk[i] = 0;
-  if (threadIdx.x < L) dir[threadIdx.x] = 0;
-  __syncthreads();
-  SState<S> st;
-#pragma unroll
-  for (int s = 0; s < L; ++s) {
-    st.rk[s] = (KeyT<S>)~0ULL;
-    st.cnt[s] = 0;
-#pragma unroll
-    for (int v = 0; v < S::NV; ++v) {
-      st.a0[s][v] = st.a1[s][v] = st.a2[s][v] = 0;
-      if constexpr (S::F64) st.fs[s][v] = 0.0;
-    }
+  const int tid = threadIdx.x, lane = tid & 31;
+  {
+    uint4* z = (uint4*)sm;
+    for (int i = tid; i < (int)(A::bytes(L, T) / 16); i += T) z[i] = make_uint4(0, 0, 0, 0);
   }
+  for (int i = tid; i < L * 32; i += T) blk[i] = 0;
+  if (tid < L) dir[tid] = 0;
+  __syncthreads();
+  KeyT<S> rk[L];
+#pragma unroll
+  for (int s = 0; s < L; ++s) rk[s] = (KeyT<S>)~0ULL;
+
   constexpr int U = 2;
   constexpr int kTile = 64 * U;
-  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
-  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+  const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
+  const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
   const int64_t n = p.g.n;
   const int64_t ntiles = (n + kTile - 1) / kTile;
   for (int64_t t = warp; t < ntiles; t += nwarps) {
     const int64_t base = t * kTile;
     if (base + kTile <= n) {
-      // issue every load of the tile first (2 units x (pred + keys + NC columns))
       uint64_t pr[U][2], k0[U][2], k1[U][2], c[U][2][S::NC];
 #pragma unroll
       for (int u = 0; u < U; ++u) {
@@ -298,8 +326,8 @@ __global__ void __launch_bounds__(256, 2) k_sga_reg_spec(const __grid_constant__
           spec_values<S>(p, c[u][k], x[k]);
         }
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base + 64 * u, lane, x[0].q, x[1].q);
-        spec_row<S>(p, dir, st, x[0], r);
-        spec_row<S>(p, dir, st, x[1], r + 1);
+        priv_row<S, L>(p, dir, rk, sm, tid, x[0], r);
+        priv_row<S, L>(p, dir, rk, sm, tid, x[1], r + 1);
       }
     } else {
       for (int u = 0; u < U; ++u) {
@@ -308,40 +336,44 @@ __global__ void __launch_bounds__(256, 2) k_sga_reg_spec(const __grid_constant__
         spec_row_scalar<S>(p, r, x0);
         spec_row_scalar<S>(p, r + 1, x1);
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base + 64 * u, lane, x0.q, x1.q);
-        spec_row<S>(p, dir, st, x0, r);
-        spec_row<S>(p, dir, st, x1, r + 1);
+        priv_row<S, L>(p, dir, rk, sm, tid, x0, r);
+        priv_row<S, L>(p, dir, rk, sm, tid, x1, r + 1);
       }
     }
   }
-  // ---- flush (same protocol as k_sga_reg): warp reduce -> shared entry -> global table
+  // ---- flush: each warp reduces its lanes' private accumulators -> CTA entry -> global table
   __syncthreads();
   uint8_t* blkb = (uint8_t*)blk;
 #pragma unroll
   for (int s = 0; s < L; ++s) {
     if (dir[s] == 0) continue;
     uint8_t* be = blkb + s * 256;
-    uint32_t cw = __reduce_add_sync(0xffffffffu, st.cnt[s]);
+    uint32_t cw = __reduce_add_sync(0xffffffffu, ((const uint32_t*)sm)[s * T + tid]);
     if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)cw);
 #pragma unroll
     for (int v = 0; v < S::NV; ++v) {
       const int off = p.g.vals[v].off_sum;
       if constexpr (S::F64) {
-        double sum = st.fs[s][v];
+        double sum = ((const double*)(sm + A::off_dbl(L, T)))[(s * S::NV + v) * T + tid];
         for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
         if (lane == 0 && off >= 0) atomicAdd((double*)(be + off), sum);
       } else {
         I128 x;
-        x.lo = (uint64_t)st.a0[s][v] | ((uint64_t)st.a1[s][v] << 32);
-        if (vx_kind(S::OP(v)) == VX_COL) x.hi = (uint64_t)((int64_t)x.lo >> 63);     // 64-bit accumulator
-        else x.hi = (uint64_t)(int64_t)(int32_t)st.a2[s][v];                          // 96-bit accumulator
+        if (vx_kind(S::OP(v)) == VX_COL) {
+          x = i128_from_i64(((const int64_t*)(sm + A::off_nar(L, T)))[(s * A::NNAR + A::nar_idx(v)) * T + tid]);
+        } else {
+          const int k = (s * A::NWIDE + A::wide_idx(v)) * T + tid;
+          x.lo = ((const uint64_t*)(sm + A::off_wlo(L, T)))[k];
+          x.hi = (uint64_t)(int64_t)(int32_t)((const uint32_t*)(sm + A::off_whi(L, T)))[k];
+        }
         x = warp_sum_i128(x);
         if (lane == 0 && off >= 0) atomic_add_i128((uint64_t*)(be + off), x.lo, x.hi);
       }
     }
   }
   __syncthreads();
-  if (threadIdx.x < L) {
-    const int s = threadIdx.x;
+  if (tid < L) {
+    const int s = tid;
     uint64_t sk = dir[s];
     if (sk != 0) {
       const uint8_t* be = blkb + s * 256;
@@ -414,29 +446,36 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
 }
 
 template <class S>
-static int spec_blocks_per_sm() {
+static int spec_blocks_per_sm(size_t smem) {
   int nb = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, k_sga_reg_spec<S>, 256, 0) != cudaSuccess || nb < 1) nb = 1;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, k_sga_priv<S, kPrivSlots>, kPrivThreads, smem) != cudaSuccess ||
+      nb < 1)
+    nb = 1;
   return nb;
 }
 
-// Try the specialised register-tier kernels; returns false if no signature matches.
+// Try the specialised low-G kernels; returns false if no signature matches.
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind) {
   SpecPlan sp;
   int64_t tiles = (g.n + 127) / 128;
-  auto go = [&](auto sig, const void* fn) -> bool {
+  auto go = [&](auto sig) -> bool {
     using S = decltype(sig);
-    int grid = sms * spec_blocks_per_sm<S>();
+    const size_t smem = Acc<S>::bytes(kPrivSlots, kPrivThreads);
+    static bool attr = false;
+    if (!attr) {
+      cudaFuncSetAttribute(k_sga_priv<S, kPrivSlots>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+      attr = true;
+    }
+    int grid = sms * spec_blocks_per_sm<S>(smem);
     int64_t need = (tiles + 7) / 8;
     if (need < grid) grid = (int)(need > 0 ? need : 1);
     count_launch();
-    k_sga_reg_spec<S><<<grid, 256, 0, s>>>(sp);
+    k_sga_priv<S, kPrivSlots><<<grid, kPrivThreads, smem, s>>>(sp);
     *err = cudaGetLastError();
-    (void)fn;
     return true;
   };
-  if (spec_match<SigQ1I>(g, &sp)) { *kind = 1; return go(SigQ1I{}, nullptr); }
-  if (spec_match<SigQ1F>(g, &sp)) { *kind = 2; return go(SigQ1F{}, nullptr); }
+  if (spec_match<SigQ1I>(g, &sp)) { *kind = 1; return go(SigQ1I{}); }
+  if (spec_match<SigQ1F>(g, &sp)) { *kind = 2; return go(SigQ1F{}); }
   return false;
 }
 

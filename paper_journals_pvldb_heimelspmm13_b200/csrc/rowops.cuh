@@ -46,7 +46,10 @@ __device__ __forceinline__ bool eval_pred(const DevPred& p, uint64_t raw) {
   return ok != (bool)p.anti;
 }
 
-__device__ __forceinline__ bool fits_i32(int64_t x) { return x == (int64_t)(int32_t)x; }
+// x fits int32 <=> its high word is the sign extension of its low word (2 SASS ops)
+__device__ __forceinline__ bool fits_i32(int64_t x) {
+  return (uint32_t)((uint64_t)x >> 32) == (uint32_t)((int32_t)(uint32_t)x >> 31);
+}
 
 // Integer value expression, fast path: exact in int64 when every factor fits in
 // int32 (true for all TPC-H-ranged decimals); otherwise *fast = false and the row

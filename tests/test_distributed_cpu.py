@@ -1,0 +1,106 @@
+"""Multi-GPU host logic on CPU: row sharding and the partial-table allgather, world size 2 over gloo.
+
+The CUDA merge kernel is covered on the GPU by test_gpu_parity.py::test_sharded_partials_merge
+(fake exchange).  Here the partial tables are produced by the oracle on each rank's shard, sent
+through exchange_partials (the same function the NCCL path uses) and merged by key in Python;
+the result must equal the oracle over all rows (sharding changes no integer bit).
+"""
+import os
+import socket
+
+import numpy as np
+import pytest
+import torch
+import torch.distributed as dist
+import torch.multiprocessing as mp
+
+from paper_journals_pvldb_heimelspmm13_b200.distributed import exchange_partials, shard_range
+
+
+@pytest.mark.parametrize("n,world", [(0, 2), (1, 2), (7, 3), (1000, 8), (600_000_001, 8)])
+def test_shard_range_partition(n, world):
+    spans = [shard_range(n, r, world) for r in range(world)]
+    pos = 0
+    for s, ln in spans:
+        assert s == pos and ln >= 0
+        pos += ln
+    assert pos == n
+    lens = [ln for _, ln in spans]
+    assert max(lens) - min(lens) <= 1
+
+
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def _worker(rank, world, port, n, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import datagen
+        import oracle
+        start, ln = shard_range(n, rank, world)
+        li = datagen.lineitem_host(ln, 77, row0=start, n_total=n)
+        vals = [li["quantity"], li["extendedprice"], li["discount"]]
+        aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 1}, {"op": "max", "a": 2}]
+        keys, outs = oracle.sga([(li["shipdate"], {"hi": 10471})], [li["returnflag"], li["linestatus"]], vals, aggs)
+        # partial rows: key, count, sum lo, sum hi, min, max  (6 x int64 = 48 bytes)
+        G = len(keys)
+        cap = 8
+        rows = np.zeros((cap, 6), np.int64)
+        rows[:G, 0] = keys
+        rows[:G, 1] = outs[0]
+        rows[:G, 2:4] = outs[1].view(np.int64).reshape(G, 2)
+        rows[:G, 4] = outs[2]
+        rows[:G, 5] = outs[3]
+        part = torch.from_numpy(rows.view(np.uint8).reshape(cap, 48).copy())
+        cnt = torch.tensor([G], dtype=torch.int64)
+        allp, counts, cap_x = exchange_partials(part, cnt)
+        assert allp.shape == (world, cap_x, 48)
+        merged = {}
+        for r in range(world):
+            t = allp[r].numpy().view(np.int64).reshape(cap_x, 6)
+            for j in range(int(counts[r])):
+                k, c, lo, hi, mn, mx = (int(x) for x in t[j])
+                s = ((hi & 0xFFFFFFFFFFFFFFFF) << 64) | (lo & 0xFFFFFFFFFFFFFFFF)
+                s = s - (1 << 128) if s >= 1 << 127 else s
+                m = merged.setdefault(k, [0, 0, None, None])
+                m[0] += c
+                m[1] += s
+                m[2] = mn if m[2] is None else min(m[2], mn)
+                m[3] = mx if m[3] is None else max(m[3], mx)
+        if rank == 0:
+            q.put(merged)
+    finally:
+        dist.destroy_process_group()
+
+
+def test_gloo_allgather_merge_equals_oracle():
+    import datagen
+    import oracle
+    n, world = 200_003, 2
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_worker, args=(r, world, port, n, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    merged = q.get(timeout=300)
+    for p in procs:
+        p.join(timeout=120)
+        assert p.exitcode == 0
+    li = datagen.lineitem_host(n, 77)
+    vals = [li["quantity"], li["extendedprice"], li["discount"]]
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 1}, {"op": "max", "a": 2}]
+    keys, outs = oracle.sga([(li["shipdate"], {"hi": 10471})], [li["returnflag"], li["linestatus"]], vals, aggs)
+    ref = {}
+    sums = outs[1].view(np.int64).reshape(len(keys), 2)
+    for i, k in enumerate(keys.tolist()):
+        s = ((int(sums[i, 1]) & 0xFFFFFFFFFFFFFFFF) << 64) | (int(sums[i, 0]) & 0xFFFFFFFFFFFFFFFF)
+        ref[k] = [int(outs[0][i]), s, int(outs[2][i]), int(outs[3][i])]
+    assert merged == ref
