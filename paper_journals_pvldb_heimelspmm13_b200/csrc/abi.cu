@@ -205,6 +205,22 @@ ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* agg
       p.has_minmax = 1;
     }
   }
+  // private accumulator record of the register tier: [count u32 | per value: sum lo u64 + hi u32 (int) or
+  // f64 | min u64 | max u64], 8-byte fields 8-aligned
+  int rec = 4;
+  for (int v = 0; v < p.nvals; ++v) {
+    DevValue& d = p.vals[v];
+    d.po_sum = d.po_hi = d.po_min = d.po_max = -1;
+    if (need_sum[v]) {
+      rec = (int)align_up((size_t)rec, 8);
+      d.po_sum = rec;
+      rec += 8;
+      if (!d.is_f64) { d.po_hi = rec; rec += 4; }
+    }
+    if (need_min[v]) { rec = (int)align_up((size_t)rec, 8); d.po_min = rec; rec += 8; }
+    if (need_max[v]) { rec = (int)align_up((size_t)rec, 8); d.po_max = rec; rec += 8; }
+  }
+  p.priv_rec = (int)align_up((size_t)rec, 8);
   int stride = (int)align_up((size_t)off, 16);
   if (stride <= 32) stride = 32;
   else if (stride <= 64) stride = 64;

@@ -134,6 +134,7 @@ struct DevValue {
   int32_t expr;
   int32_t is_f64;
   int32_t off_sum, off_min, off_max;  // entry byte offsets, -1 if that state is not needed
+  int32_t po_sum, po_hi, po_min, po_max;  // private-accumulator field offsets (bytes per thread), -1 if absent
   int64_t S;                          // 10^scale
   double Sf;
 };
@@ -150,6 +151,8 @@ struct Plan {
   uint64_t mask;        // cap - 1 (cap is a power of two)
   int32_t stride;       // entry bytes
   int32_t has_minmax;
+  int32_t priv_rec;     // private accumulator record: bytes per thread per group slot
+  int32_t pad_;
   int32_t* status;      // device status word (may be null)
   uint32_t* bitmap_out; // optional selection bitmap
   const int32_t* gids;  // unfused aggregate: direct group ids (table indexed by gid)

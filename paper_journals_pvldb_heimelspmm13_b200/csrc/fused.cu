@@ -130,178 +130,171 @@ __device__ __forceinline__ void eval_pair_vec(const Plan& p, int64_t r, RowIn<NV
   eval_values_pair<NV, F64>(p, r, x0, x1);
 }
 
-// ------------------------------------------------------------------ register tier
-template <int L, int NV, bool F64, bool MINMAX>
-struct RegState {
-  uint64_t rk[L];                      // real keys of the block directory (~0 = none)
-  uint32_t cnt[L];
-  uint32_t s0[F64 ? 1 : L][F64 ? 1 : NV], s1[F64 ? 1 : L][F64 ? 1 : NV], s2[F64 ? 1 : L][F64 ? 1 : NV];
-  double fs[F64 ? L : 1][F64 ? NV : 1];
-  int64_t mn[MINMAX && !F64 ? L : 1][MINMAX && !F64 ? NV : 1], mx[MINMAX && !F64 ? L : 1][MINMAX && !F64 ? NV : 1];
-  double fmn[MINMAX && F64 ? L : 1][MINMAX && F64 ? NV : 1], fmx[MINMAX && F64 ? L : 1][MINMAX && F64 ? NV : 1];
-};
+// ------------------------------------------------------------------ register (private accumulator) tier
+// Few groups: each thread owns one accumulator record per group slot in shared
+// memory, laid out [slot][field][thread] (field offsets from the host planner,
+// Plan::priv_rec bytes per thread per slot): count u32; per value: SUM as 96-bit
+// (u64 lo + u32 hi) or double; MIN / MAX as order-preserving u64 encodings (zero
+// = identity).  A row costs one slot-indexed read-modify-write per accumulator:
+// no atomics in the row loop — the limit of the paper's "multiple accumulators
+// per group" in local memory.  A block-wide slot directory in shared
+// memory gives every thread the same key -> slot map.
+constexpr int kRegSlots = 4;
 
-template <int L, int NV, bool F64, bool MINMAX>
-__device__ __forceinline__ void reg_row(const Plan& p, uint64_t* dir, RegState<L, NV, F64, MINMAX>& st,
-                                        const RowIn<NV, F64>& x, int64_t r) {
-  bool m[L];
-  bool hit = false;
+template <int NV, bool F64>
+__device__ __forceinline__ void privg_add(const Plan& p, uint8_t* sm, int slot, int tid, const RowIn<NV, F64>& x) {
+  constexpr int T = kFusedThreads;
+  uint8_t* base = sm + (size_t)slot * p.priv_rec * T;
+  ((uint32_t*)base)[tid] += 1u;
 #pragma unroll
-  for (int s = 0; s < L; ++s) {
-    m[s] = x.key == st.rk[s];
-    hit = hit || m[s];
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (F64) {
+      const double val = x.vd[v];
+      if (d.po_sum >= 0) ((double*)(base + d.po_sum * T))[tid] += val;
+      if (d.po_min >= 0) {
+        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
+        *m = max(*m, enc_min_f(val));
+      }
+      if (d.po_max >= 0) {
+        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
+        *m = max(*m, enc_max_f(val));
+      }
+    } else {
+      if (d.is_f64) continue;                       // mixed plan: fp64 values went to the slow path
+      const int64_t val = x.vi[v];
+      if (d.po_sum >= 0) {
+        uint64_t* lo = (uint64_t*)(base + d.po_sum * T) + tid;
+        uint32_t* hi = (uint32_t*)(base + d.po_hi * T) + tid;
+        uint64_t l = *lo;
+        uint32_t h = *hi;
+        uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
+        asm("add.cc.u32 %0, %0, %3;\n\taddc.cc.u32 %1, %1, %4;\n\taddc.u32 %2, %2, %5;"
+            : "+r"(l0), "+r"(l1), "+r"(h)
+            : "r"((uint32_t)(uint64_t)val), "r"((uint32_t)((uint64_t)val >> 32)), "r"((uint32_t)(val >> 63)));
+        *lo = (uint64_t)l0 | ((uint64_t)l1 << 32);
+        *hi = h;
+      }
+      if (d.po_min >= 0) {
+        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
+        *m = max(*m, enc_min_i(val));
+      }
+      if (d.po_max >= 0) {
+        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
+        *m = max(*m, enc_max_i(val));
+      }
+    }
   }
+}
+
+template <int NV, bool F64>
+__device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t (&rk)[kRegSlots], uint8_t* sm, int tid,
+                                          const RowIn<NV, F64>& x, int64_t r) {
+  constexpr int L = kRegSlots;
+  int slot = -1;
+#pragma unroll
+  for (int s = L - 1; s >= 0; --s)
+    if (x.key == rk[s]) slot = s;
   const bool special = x.key == ~0ULL;
-  bool go = x.q && x.fast && hit && !special;
-  if (x.q && !go) {                       // divergent, rare after warm-up
-    int slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, x.key) : -1;
+  bool go = x.q && x.fast && slot >= 0 && !special;
+  if (x.q && !go) {                       // rare after warm-up: new key in this CTA, or slow value
+    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, x.key) : -1;
     if (slot >= 0) {
 #pragma unroll
-      for (int s = 0; s < L; ++s) {
-        st.rk[s] = ~*(volatile uint64_t*)&dir[s];
-        m[s] = s == slot;
-      }
+      for (int s = 0; s < L; ++s) rk[s] = ~*(volatile uint64_t*)&dir[s];
       go = true;
     } else {
       uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
       if (e) update_entry_slow(p, e, r);
     }
   }
-#pragma unroll
-  for (int s = 0; s < L; ++s) {
-    const bool mm = go && m[s];
-    st.cnt[s] += mm ? 1u : 0u;
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if constexpr (F64) {
-        if (mm) st.fs[s][v] += x.vd[v];
-        if constexpr (MINMAX) {
-          if (mm) {
-            st.fmn[s][v] = fmin(st.fmn[s][v], x.vd[v]);
-            st.fmx[s][v] = fmax(st.fmx[s][v], x.vd[v]);
-          }
-        }
-      } else {
-        add96(mm, st.s0[s][v], st.s1[s][v], st.s2[s][v], x.vi[v]);
-        if constexpr (MINMAX) {
-          if (mm) {
-            st.mn[s][v] = min(st.mn[s][v], x.vi[v]);
-            st.mx[s][v] = max(st.mx[s][v], x.vi[v]);
-          }
-        }
-      }
-    }
-  }
+  if (go) privg_add<NV, F64>(p, sm, slot, tid, x);
 }
 
-template <int L, int NV, bool F64, bool MINMAX, int U>
+template <int NV, bool F64, int U>
 __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant__ Plan p) {
+  constexpr int L = kRegSlots;
+  constexpr int T = kFusedThreads;
+  extern __shared__ __align__(16) uint8_t sm[];
   __shared__ uint64_t dir[L];
   __shared__ __align__(16) uint64_t blk[L * 32];   // block accumulators, entry layout (stride <= 256 B)
-  const int lane = threadIdx.x & 31;
-  for (int i = threadIdx.x; i < L * 32; i += blockDim.x) blk[i] = 0;
-  if (threadIdx.x < L) dir[threadIdx.x] = 0;
-  __syncthreads();
-
-  RegState<L, NV, F64, MINMAX> st;
-#pragma unroll
-  for (int s = 0; s < L; ++s) {
-    st.rk[s] = ~0ULL;
-    st.cnt[s] = 0;
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if constexpr (F64) {
-        st.fs[s][v] = 0.0;
-        if constexpr (MINMAX) { st.fmn[s][v] = __longlong_as_double(0x7FF0000000000000LL); st.fmx[s][v] = -st.fmn[s][v]; }
-      } else {
-        st.s0[s][v] = st.s1[s][v] = st.s2[s][v] = 0;
-        if constexpr (MINMAX) { st.mn[s][v] = INT64_MAX; st.mx[s][v] = INT64_MIN; }
-      }
-    }
+  const int tid = threadIdx.x, lane = tid & 31;
+  {
+    uint4* z = (uint4*)sm;
+    const int n16 = (int)((size_t)L * p.priv_rec * T / 16);
+    for (int i = tid; i < n16; i += T) z[i] = make_uint4(0, 0, 0, 0);
   }
+  for (int i = tid; i < L * 32; i += T) blk[i] = 0;
+  if (tid < L) dir[tid] = 0;
+  __syncthreads();
+  uint64_t rk[L];
+#pragma unroll
+  for (int s = 0; s < L; ++s) rk[s] = ~0ULL;   // ~0 never matches a slot (special key)
 
   constexpr int kTile = 64 * U;
-  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
-  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+  const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
+  const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
   const int64_t ntiles = (p.n + kTile - 1) / kTile;
   for (int64_t t = warp; t < ntiles; t += nwarps) {
     const int64_t base = t * kTile;
-    if (p.vec_ok && base + kTile <= p.n) {
+    const bool vec = p.vec_ok && base + kTile <= p.n;
 #pragma unroll
-      for (int u = 0; u < U; ++u) {
-        const int64_t r = base + 64 * u + 2 * lane;
-        RowIn<NV, F64> x0, x1;
+    for (int u = 0; u < U; ++u) {
+      const int64_t r = base + 64 * u + 2 * lane;
+      RowIn<NV, F64> x0, x1;
+      if (vec) {
         eval_pair_vec<NV, F64>(p, r, x0, x1);
-        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-        reg_row<L, NV, F64, MINMAX>(p, dir, st, x0, r);
-        reg_row<L, NV, F64, MINMAX>(p, dir, st, x1, r + 1);
-      }
-    } else {
-      for (int u = 0; u < U; ++u) {
-        const int64_t r = base + 64 * u + 2 * lane;
-        RowIn<NV, F64> x0, x1;
+      } else {
         eval_row_scalar<NV, F64>(p, r, x0);
         eval_row_scalar<NV, F64>(p, r + 1, x1);
-        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-        reg_row<L, NV, F64, MINMAX>(p, dir, st, x0, r);
-        reg_row<L, NV, F64, MINMAX>(p, dir, st, x1, r + 1);
       }
+      if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+      privg_row<NV, F64>(p, dir, rk, sm, tid, x0, r);
+      privg_row<NV, F64>(p, dir, rk, sm, tid, x1, r + 1);
     }
   }
 
-  // ---- flush: warp reduce -> shared block entry -> one global update per slot
+  // ---- flush: warp reduce of the private records -> shared block entry -> one global update per slot
   __syncthreads();
   uint8_t* blkb = (uint8_t*)blk;
-#pragma unroll
   for (int s = 0; s < L; ++s) {
     if (dir[s] == 0) continue;                       // uniform: slot never used in this block
     uint8_t* be = blkb + s * 256;
-    uint32_t c = __reduce_add_sync(0xffffffffu, st.cnt[s]);
+    const uint8_t* rec = sm + (size_t)s * p.priv_rec * T;
+    uint32_t c = __reduce_add_sync(0xffffffffu, ((const uint32_t*)rec)[tid]);
     if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)c);
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if (v >= p.nvals) break;
+    for (int v = 0; v < p.nvals; ++v) {
       const DevValue& d = p.vals[v];
-      if constexpr (F64) {
-        double sum = st.fs[s][v];
-        for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
-        if (lane == 0 && d.off_sum >= 0) atomicAdd((double*)(be + d.off_sum), sum);
-        if constexpr (MINMAX) {
-          double a = st.fmn[s][v], b = st.fmx[s][v];
-          for (int o = 16; o > 0; o >>= 1) {
-            a = fmin(a, __shfl_xor_sync(0xffffffffu, a, o));
-            b = fmax(b, __shfl_xor_sync(0xffffffffu, b, o));
-          }
-          if (lane == 0 && c > 0) {
-            if (d.off_min >= 0) atomicMax((unsigned long long*)(be + d.off_min), (unsigned long long)enc_min_f(a));
-            if (d.off_max >= 0) atomicMax((unsigned long long*)(be + d.off_max), (unsigned long long)enc_max_f(b));
-          }
+      if (d.po_sum >= 0) {
+        if (d.is_f64) {
+          double sum = ((const double*)(rec + d.po_sum * T))[tid];
+          for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
+          if (lane == 0) atomicAdd((double*)(be + d.off_sum), sum);
+        } else {
+          I128 x;
+          x.lo = ((const uint64_t*)(rec + d.po_sum * T))[tid];
+          x.hi = (uint64_t)(int64_t)(int32_t)((const uint32_t*)(rec + d.po_hi * T))[tid];
+          x = warp_sum_i128(x);
+          if (lane == 0) atomic_add_i128((uint64_t*)(be + d.off_sum), x.lo, x.hi);
         }
-      } else {
-        if (d.is_f64) continue;   // mixed plan: accumulated by the slow path only
-        I128 x;
-        x.lo = (uint64_t)st.s0[s][v] | ((uint64_t)st.s1[s][v] << 32);
-        x.hi = (uint64_t)(int64_t)(int32_t)st.s2[s][v];
-        x = warp_sum_i128(x);
-        if (lane == 0 && d.off_sum >= 0) atomic_add_i128((uint64_t*)(be + d.off_sum), x.lo, x.hi);
-        if constexpr (MINMAX) {
-          int64_t a = st.mn[s][v], b = st.mx[s][v];
-          for (int o = 16; o > 0; o >>= 1) {
-            a = min(a, (int64_t)__shfl_xor_sync(0xffffffffu, (long long)a, o));
-            b = max(b, (int64_t)__shfl_xor_sync(0xffffffffu, (long long)b, o));
-          }
-          if (lane == 0 && c > 0) {
-            if (d.off_min >= 0) atomicMax((unsigned long long*)(be + d.off_min), (unsigned long long)enc_min_i(a));
-            if (d.off_max >= 0) atomicMax((unsigned long long*)(be + d.off_max), (unsigned long long)enc_max_i(b));
-          }
-        }
+      }
+      if (d.po_min >= 0) {
+        unsigned long long m = ((const uint64_t*)(rec + d.po_min * T))[tid];
+        for (int o = 16; o > 0; o >>= 1) m = max(m, __shfl_xor_sync(0xffffffffu, m, o));
+        if (lane == 0 && m) atomicMax((unsigned long long*)(be + d.off_min), m);
+      }
+      if (d.po_max >= 0) {
+        unsigned long long m = ((const uint64_t*)(rec + d.po_max * T))[tid];
+        for (int o = 16; o > 0; o >>= 1) m = max(m, __shfl_xor_sync(0xffffffffu, m, o));
+        if (lane == 0 && m) atomicMax((unsigned long long*)(be + d.off_max), m);
       }
     }
   }
   __syncthreads();
-  // one thread per (slot, state word) pushes the block entry into the global table
-  if (threadIdx.x < L) {
-    const int s = threadIdx.x;
+  // one thread per slot pushes the block entry into the global table
+  if (tid < L) {
+    const int s = tid;
     uint64_t sk = dir[s];
     if (sk != 0) {
       const uint8_t* be = blkb + s * 256;
@@ -378,59 +371,62 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant
 }
 
 // ------------------------------------------------------------------ dispatch
-constexpr int kRegSlots = 4;
 constexpr int kUnits = 2;
 
-template <int NV, bool F64, bool MM>
-static cudaError_t launch_reg_nv(const Plan& p, int grid, cudaStream_t s) {
-  count_launch();
-  k_sga_reg<kRegSlots, NV, F64, MM, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  return cudaGetLastError();
-}
+static size_t reg_smem(const Plan& p) { return (size_t)kRegSlots * p.priv_rec * kFusedThreads; }
 
 template <int NV, bool F64>
-static cudaError_t launch_reg_mm(const Plan& p, int grid, cudaStream_t s) {
-  return p.has_minmax ? launch_reg_nv<NV, F64, true>(p, grid, s) : launch_reg_nv<NV, F64, false>(p, grid, s);
+static cudaError_t launch_reg_nv(const Plan& p, int grid, cudaStream_t s) {
+  const size_t smem = reg_smem(p);
+  cudaError_t e = cudaFuncSetAttribute(k_sga_reg<NV, F64, kUnits>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                       (int)smem);
+  if (e != cudaSuccess) return e;
+  count_launch();
+  k_sga_reg<NV, F64, kUnits><<<grid, kFusedThreads, smem, s>>>(p);
+  return cudaGetLastError();
 }
 
 template <bool F64>
 static cudaError_t launch_reg_f(const Plan& p, int grid, cudaStream_t s) {
-  if (p.nvals <= 1) return launch_reg_mm<1, F64>(p, grid, s);
-  if (p.nvals <= 2) return launch_reg_mm<2, F64>(p, grid, s);
-  if (p.nvals <= 4) return launch_reg_mm<4, F64>(p, grid, s);
-  return launch_reg_mm<6, F64>(p, grid, s);
+  if (p.nvals <= 1) return launch_reg_nv<1, F64>(p, grid, s);
+  if (p.nvals <= 2) return launch_reg_nv<2, F64>(p, grid, s);
+  if (p.nvals <= 4) return launch_reg_nv<4, F64>(p, grid, s);
+  return launch_reg_nv<6, F64>(p, grid, s);
 }
 
 template <bool F64>
 static cudaError_t launch_glb_f(const Plan& p, int grid, cudaStream_t s) {
-  if (p.nvals <= 1) { count_launch(); k_sga_glb<1, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
-  else if (p.nvals <= 2) { count_launch(); k_sga_glb<2, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
-  else if (p.nvals <= 4) { count_launch(); k_sga_glb<4, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
-  else { count_launch(); k_sga_glb<6, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p); }
+  count_launch();
+  if (p.nvals <= 1) k_sga_glb<1, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 2) k_sga_glb<2, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 4) k_sga_glb<4, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else k_sga_glb<6, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
   return cudaGetLastError();
 }
 
 int reg_tier_slots() { return kRegSlots; }
 
 template <int NV, bool F64>
-static const void* reg_kernel_ptr(bool mm) {
-  return mm ? (const void*)k_sga_reg<kRegSlots, NV, F64, true, kUnits> : (const void*)k_sga_reg<kRegSlots, NV, F64, false, kUnits>;
-}
+static const void* reg_kernel_ptr() { return (const void*)k_sga_reg<NV, F64, kUnits>; }
+template <int NV, bool F64>
+static const void* glb_kernel_ptr() { return (const void*)k_sga_glb<NV, F64, kUnits>; }
 
 // Resident CTAs per SM of the instantiation launch_fused would pick (persistent grid sizing).
 int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64) {
+  const int nv = p.nvals <= 1 ? 1 : (p.nvals <= 2 ? 2 : (p.nvals <= 4 ? 4 : 6));
   const void* fn;
-  int nv = p.nvals <= 1 ? 1 : (p.nvals <= 2 ? 2 : (p.nvals <= 4 ? 4 : 6));
-  bool mm = p.has_minmax != 0;
   if (reg_tier) {
-    if (values_f64) fn = nv == 1 ? reg_kernel_ptr<1, true>(mm) : nv == 2 ? reg_kernel_ptr<2, true>(mm) : nv == 4 ? reg_kernel_ptr<4, true>(mm) : reg_kernel_ptr<6, true>(mm);
-    else fn = nv == 1 ? reg_kernel_ptr<1, false>(mm) : nv == 2 ? reg_kernel_ptr<2, false>(mm) : nv == 4 ? reg_kernel_ptr<4, false>(mm) : reg_kernel_ptr<6, false>(mm);
+    if (values_f64) fn = nv == 1 ? reg_kernel_ptr<1, true>() : nv == 2 ? reg_kernel_ptr<2, true>() : nv == 4 ? reg_kernel_ptr<4, true>() : reg_kernel_ptr<6, true>();
+    else fn = nv == 1 ? reg_kernel_ptr<1, false>() : nv == 2 ? reg_kernel_ptr<2, false>() : nv == 4 ? reg_kernel_ptr<4, false>() : reg_kernel_ptr<6, false>();
+    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)reg_smem(p));
   } else {
-    if (values_f64) fn = nv == 1 ? (const void*)k_sga_glb<1, true, kUnits> : nv == 2 ? (const void*)k_sga_glb<2, true, kUnits> : nv == 4 ? (const void*)k_sga_glb<4, true, kUnits> : (const void*)k_sga_glb<6, true, kUnits>;
-    else fn = nv == 1 ? (const void*)k_sga_glb<1, false, kUnits> : nv == 2 ? (const void*)k_sga_glb<2, false, kUnits> : nv == 4 ? (const void*)k_sga_glb<4, false, kUnits> : (const void*)k_sga_glb<6, false, kUnits>;
+    if (values_f64) fn = nv == 1 ? glb_kernel_ptr<1, true>() : nv == 2 ? glb_kernel_ptr<2, true>() : nv == 4 ? glb_kernel_ptr<4, true>() : glb_kernel_ptr<6, true>();
+    else fn = nv == 1 ? glb_kernel_ptr<1, false>() : nv == 2 ? glb_kernel_ptr<2, false>() : nv == 4 ? glb_kernel_ptr<4, false>() : glb_kernel_ptr<6, false>();
   }
   int nb = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, 0) != cudaSuccess || nb < 1) nb = 1;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, reg_tier ? reg_smem(p) : 0) != cudaSuccess ||
+      nb < 1)
+    nb = 1;
   return nb;
 }
 
