@@ -98,31 +98,42 @@ class ClockSampler:
     def _run(self):
         while not self._stop.is_set():
             try:
-                self.samples.append(self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM))
+                t = time.perf_counter()
+                mhz = self.nv.nvmlDeviceGetClockInfo(self.h, self.nv.NVML_CLOCK_SM)
                 r = self.nv.nvmlDeviceGetCurrentClocksEventReasons(self.h)
-                for bit, name in self.REASONS.items():
-                    if r & bit:
-                        self.reasons.add(name)
+                self.trace.append((t, mhz, r))
             except Exception:  # noqa: BLE001
                 pass
-            time.sleep(0.002)
+            time.sleep(0.0005)
 
-    def __enter__(self):
+    def start(self):
+        """Start sampling (before warm-up, so the thread is running when the timed region opens)."""
+        self.trace = []
         if self.ok:
             self.t = threading.Thread(target=self._run, daemon=True)
             self.t.start()
         return self
 
-    def __exit__(self, *a):
+    def window(self, t0, t1):
+        self.t0, self.t1 = t0, t1
+
+    def stop(self):
         self._stop.set()
         if self.ok:
             self.t.join()
 
     def summary(self):
-        if not self.samples:
-            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": sorted(self.reasons), "samples": 0}
-        return {"sm_mhz": statistics.median(self.samples), "sm_max_mhz": self.max_mhz,
-                "reasons": sorted(self.reasons - {"gpu_idle"}), "samples": len(self.samples)}
+        """Median SM clock and the union of throttle reasons over samples taken inside the timed window."""
+        inside = [(m, r) for t, m, r in self.trace if self.t0 <= t <= self.t1]
+        reasons = set()
+        for _, r in inside:
+            for bit, name in self.REASONS.items():
+                if r & bit:
+                    reasons.add(name)
+        if not inside:
+            return {"sm_mhz": None, "sm_max_mhz": self.max_mhz, "reasons": [], "samples": 0}
+        return {"sm_mhz": statistics.median(m for m, _ in inside), "sm_max_mhz": self.max_mhz,
+                "reasons": sorted(reasons - {"gpu_idle"}), "samples": len(inside)}
 
 
 def measured_peak_gbs():
@@ -176,7 +187,7 @@ def run_reference(args, wl, rank):
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
-    ap.add_argument("--steps", type=int, default=20)
+    ap.add_argument("--steps", type=int, default=50)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--workload", default="c4", choices=sorted(WORKLOADS))
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
@@ -219,6 +230,7 @@ def main():
         else:
             distributed_select_group_aggregate(call)
 
+    clk = ClockSampler(local).start()
     for _ in range(args.warmup):
         step()
     torch.cuda.synchronize()
@@ -235,13 +247,16 @@ def main():
         dist.barrier()
     torch.cuda.synchronize()
     launches0 = ocl.launch_count()
-    with ClockSampler(local) as clk:
-        t0.record()
-        for i in range(K):
-            ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
-            step()
-        t1.record()
-        torch.cuda.synchronize()
+    h0 = time.perf_counter()
+    t0.record()
+    for i in range(K):
+        ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
+        step()
+    t1.record()
+    torch.cuda.synchronize()
+    h1 = time.perf_counter()
+    clk.window(h0, h1)
+    clk.stop()
     ocl.set_kernel_events(ctx, None, None)
     launches = ocl.launch_count() - launches0
     if world > 1:

@@ -108,3 +108,20 @@ def canon_gids(gids):
             mapping[g] = len(mapping)
         out[j] = mapping[g]
     return out
+
+
+def assert_results_equal_np(gkeys, gouts, rkeys, routs, aggs, vals_dtypes, rtol=1e-9):
+    """Vectorised version of assert_results_equal for large G: sort both sides by key."""
+    gk = np.asarray(gkeys).view(np.uint64)
+    rk = np.asarray(rkeys).view(np.uint64)
+    assert len(gk) == len(rk), f"G differs: {len(gk)} vs {len(rk)}"
+    gi, ri = np.argsort(gk, kind="stable"), np.argsort(rk, kind="stable")
+    assert np.array_equal(gk[gi], rk[ri]), "group key sets differ"
+    for spec, g, r in zip(aggs, gouts, routs):
+        g, r = np.asarray(g)[gi], np.asarray(r)[ri]
+        fp_in = spec["op"] != "count" and vals_dtypes[spec["a"]] == np.float64
+        if spec["op"] == "avg" or (spec["op"] == "sum" and fp_in):
+            assert np.all(np.abs(g - r) <= rtol * np.abs(r)), spec
+        else:
+            assert np.array_equal(g.view(np.uint64) if g.dtype != np.uint64 else g,
+                                  r.view(np.uint64) if r.dtype != np.uint64 else r), spec
