@@ -49,6 +49,9 @@ WORKLOADS = {
     "c3": dict(desc="C3: lineitem SF10, 60,000,000 rows; GROUP BY l_orderkey (15M groups, HBM hash table), "
                     "COUNT/SUM/MIN/MAX(l_quantity), clustered row order",
                rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000),
+    "c5": dict(desc="C5 sweep point: 2^28 rows, p i32 ~ U[0,1e6), key = hash(Zipf(s) rank over G), v i64; "
+                    "WHERE p < T GROUP BY key: COUNT, SUM, MIN, MAX(v)",
+               rows=1 << 28, seed=datagen.BASE_SEED + 5, kind="sweep", f64=False, groups=1 << 10),
 }
 
 
@@ -68,11 +71,32 @@ def workload_columns(wl, cols):
         return ([(cols["shipdate"], Q1_PRED)], [cols["returnflag"], cols["linestatus"]], [cols[x] for x in v],
                 aggs, 4 + 1 + 1 + 4 * 8)
     aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    if wl["kind"] == "sweep":
+        return [(cols["p"], {"hi": wl["threshold"] - 1})], [cols["key"]], [cols["v"]], aggs, 20
     return [], [cols["orderkey"]], [cols["quantity"]], aggs, 16
 
 
 def wl_fields(wl):
+    if wl["kind"] == "sweep":
+        return ("p", "key", "v")
     return q1_fields(wl["f64"]) if wl["kind"] == "q1" else ("orderkey", "quantity")
+
+
+def gen_device(wl, length, start, n, dev):
+    if wl["kind"] == "sweep":
+        return datagen.sweep_device(length, wl["seed"], wl["groups"], s=wl["zipf"], row0=start, device=dev)
+    return datagen.lineitem_device(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, device=dev)
+
+
+def gen_host(wl, length, start, n, out=None):
+    if wl["kind"] == "sweep":
+        h = datagen.sweep_host(length, wl["seed"], wl["groups"], s=wl["zipf"], row0=start)
+        if out is not None:
+            for f in out:
+                out[f][:] = h[f]
+            return out
+        return h
+    return datagen.lineitem_host(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, out=out)
 
 
 class ClockSampler:
@@ -167,7 +191,7 @@ def run_reference(args, wl, rank):
     if rank != 0:
         return
     sample = min(wl["rows"], args.ref_rows)
-    cols = datagen.lineitem_host(sample, wl["seed"], fields=wl_fields(wl), n_total=wl["rows"])
+    cols = gen_host(wl, sample, 0, wl["rows"])
     for _ in range(args.warmup):
         oracle_time(wl, cols, sample)
     ts = [oracle_time(wl, cols, sample) for _ in range(args.steps)]
@@ -197,8 +221,14 @@ def main():
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--tier", type=int, default=0)
+    ap.add_argument("--c5-groups", type=int, default=1 << 10, help="C5: key cardinality G")
+    ap.add_argument("--c5-zipf", type=float, default=0.0, help="C5: Zipf exponent s (0 = uniform)")
+    ap.add_argument("--c5-sel", type=float, default=1.0, help="C5: selectivity (0.01, 0.5, 1.0)")
     args = ap.parse_args()
-    wl = WORKLOADS[args.workload]
+    wl = dict(WORKLOADS[args.workload])
+    if wl["kind"] == "sweep":
+        wl.update(groups=args.c5_groups, zipf=args.c5_zipf, threshold=max(1, int(round(args.c5_sel * 10**6))))
+        wl["desc"] += f" [G={args.c5_groups}, zipf={args.c5_zipf}, selectivity={args.c5_sel}]"
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
@@ -215,7 +245,7 @@ def main():
 
     n = wl["rows"]
     start, length = shard_range(n, rank, world)
-    cols = datagen.lineitem_device(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, device=dev)
+    cols = gen_device(wl, length, start, n, dev)
     torch.cuda.synchronize()
     p, k, v, aggs, bpr = workload_columns(wl, cols)
     order = wl["kind"] == "q1"
@@ -276,8 +306,7 @@ def main():
     e2e = None
     if not args.no_e2e:
         host = {f: torch.empty(length, dtype=c.dtype, pin_memory=True) for f, c in cols.items()}
-        datagen.lineitem_host(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n,
-                              out={f: h.numpy() for f, h in host.items()})
+        gen_host(wl, length, start, n, out={f: h.numpy() for f, h in host.items()})
         hp, hk, hv, haggs, _ = workload_columns(wl, host)
         h2d = sum(h.numel() * h.element_size() for h in host.values())
         if world == 1:
@@ -323,7 +352,7 @@ def main():
     if rank == 0 and world == 1 and not args.no_cpu:
         sample = min(n, args.cpu_rows)
         hcols = {f: h.numpy()[:sample] for f, h in host.items()} if e2e is not None else \
-            datagen.lineitem_host(sample, wl["seed"], fields=wl_fields(wl), n_total=n)
+            gen_host(wl, sample, 0, n)
         dt = oracle_time(wl, hcols, sample)
         cpu = {"value": sample / dt, "unit": "rows/s", "cores": 1, "kind": "oracle",
                "sample": f"first {sample:,} rows of the same workload, oracle.sga (C++17, single thread), "

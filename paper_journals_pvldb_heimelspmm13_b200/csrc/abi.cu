@@ -283,6 +283,32 @@ ocl_status plan_preds(const ocl_column* pred_cols, const ocl_range* preds, int32
   return OCL_OK;
 }
 
+// Shared-memory budget of one register-tier CTA (private records + mid-G table).
+constexpr size_t kRegTierSmem = 200 * 1024;
+
+// Tiers: <= 4 expected groups -> private slots only; <= the CTA
+// table capacity -> private slots + per-CTA shared-memory hash table; else the
+// HBM table.  tier 1/3/4 force the register tier (4: with the shared table).
+bool use_reg_tier(const ocl_sga_args* a, const Plan& p) {
+  if (a->tier == 1 || a->tier == 3 || a->tier == 4) return true;
+  if (a->tier == 2) return false;
+  if (a->expected_groups <= reg_tier_slots()) return true;
+  return p.smem_cap > 0;
+}
+
+// CTA shared-table capacity for the register tier (0 = none).
+int32_t plan_smem_cap(const ocl_sga_args* a, const Plan& p) {
+  bool want = a->tier == 4 || (a->tier == 0 && a->expected_groups > reg_tier_slots());
+  if (!want) return 0;
+  size_t priv = (size_t)reg_tier_slots() * p.priv_rec * 256;
+  if (priv >= kRegTierSmem) return 0;
+  uint64_t cap = next_pow2((uint64_t)std::max<int64_t>(2 * a->expected_groups, 64));
+  uint64_t fit = (kRegTierSmem - priv) / (size_t)p.stride;
+  while (cap > fit) cap >>= 1;
+  if (a->tier == 0 && (int64_t)cap < 2 * a->expected_groups) return 0;   // would overflow: use the HBM tier
+  return (int32_t)(cap >= 64 ? cap : 0);
+}
+
 ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true) {
   if (!a) return fail(OCL_ERR_INVALID_ARG, "NULL args");
   memset(P, 0, sizeof(*P));
@@ -316,6 +342,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   P->table_bytes = align_up((P->cap + 1) * (size_t)p.stride, 256);
   p.status = a->dev_status;
   p.bitmap_out = a->bitmap_out;
+  p.smem_cap = plan_smem_cap(a, p);
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;
   f.keys_out = a->keys_out;
@@ -327,11 +354,6 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   return OCL_OK;
 }
 
-bool use_reg_tier(const ocl_sga_args* a) {
-  if (a->tier == 1 || a->tier == 3) return true;
-  if (a->tier == 2) return false;
-  return a->expected_groups <= reg_tier_slots();
-}
 
 int fused_grid(ocl_ctx* ctx, const Planned& P, bool reg) {
   return ctx->sms * fused_blocks_per_sm(P.plan, reg, P.values_f64);
@@ -350,11 +372,11 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   OCL_CUDA(cudaMemsetAsync(ws, 0, P.table_bytes, s), "table init");
   if (a->dev_status) OCL_CUDA(cudaMemsetAsync(a->dev_status, 0, sizeof(int32_t), s), "status init");
   if (P.plan.n > 0) {
-    bool reg = use_reg_tier(a);
+    bool reg = use_reg_tier(a, P.plan);
     if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, s), "profile event");
     cudaError_t err = cudaSuccess;
     int kind = 0;
-    if (!(reg && a->tier != 3 && launch_fused_spec(P.plan, ctx->sms, s, &err, &kind)))
+    if (!(reg && a->tier != 3 && P.plan.smem_cap == 0 && launch_fused_spec(P.plan, ctx->sms, s, &err, &kind)))
       err = launch_fused(P.plan, reg, P.values_f64, fused_grid(ctx, P, reg), s);
     OCL_CUDA(err, "fused kernel launch");
     ctx->last_kernel = kind;
@@ -795,7 +817,7 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
   p.table = table;
   p.status = d_status;
   p.bitmap_out = nullptr;
-  const bool reg = use_reg_tier(args);
+  const bool reg = use_reg_tier(args, P.plan);
   const int grid = fused_grid(ctx, P, reg);
   const int64_t n = P.plan.n;
   int64_t nchunks = (n + chunk_rows - 1) / chunk_rows;

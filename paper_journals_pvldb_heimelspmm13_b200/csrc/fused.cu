@@ -188,6 +188,65 @@ __device__ __forceinline__ void privg_add(const Plan& p, uint8_t* sm, int slot, 
   }
 }
 
+// Per-CTA shared-memory hash table (mid-G overflow of the private slots, P:L564-568
+// local-memory aggregation tables): linear probing with shared-memory atomicCAS,
+// at most kSmemProbes probes, then the row goes to the HBM table.
+constexpr int kSmemProbes = 32;
+
+__device__ __forceinline__ uint8_t* smem_find_or_insert(uint8_t* tab, uint32_t cap, int32_t stride, uint64_t key) {
+  const uint64_t sk = ~key;
+  uint32_t h = (uint32_t)fmix64(key) & (cap - 1);
+  for (int probe = 0; probe < kSmemProbes; ++probe) {
+    uint64_t* kp = (uint64_t*)(tab + (size_t)h * stride);
+    uint64_t cur = *(volatile uint64_t*)kp;
+    if (cur == sk) return (uint8_t*)kp;
+    if (cur == 0) {
+      uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
+      if (prev == 0 || prev == sk) return (uint8_t*)kp;
+    }
+    h = (h + 1) & (cap - 1);
+  }
+  return nullptr;
+}
+
+// Row contribution with atomics on an entry (shared or global) from fast-path values.
+template <int NV, bool F64>
+__device__ __forceinline__ void entry_add_fast(const Plan& p, uint8_t* e, const RowIn<NV, F64>& x) {
+  atomicAdd((unsigned long long*)(e + 8), 1ULL);
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (F64) {
+      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), x.vd[v]);
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(x.vd[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(x.vd[v]));
+    } else {
+      if (d.is_f64) continue;
+      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)x.vi[v], (uint64_t)(x.vi[v] >> 63));
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(x.vi[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(x.vi[v]));
+    }
+  }
+}
+
+// Merge a whole entry (shared-memory table or CTA block entry) into the HBM table.
+__device__ __forceinline__ void entry_merge_global(const Plan& p, uint64_t key, const uint8_t* src) {
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
+  if (!e) return;
+  atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(src + 8));
+  for (int v = 0; v < p.nvals; ++v) {
+    const DevValue& d = p.vals[v];
+    if (d.off_sum >= 0) {
+      if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(src + d.off_sum));
+      else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(src + d.off_sum),
+                           *(const uint64_t*)(src + d.off_sum + 8));
+    }
+    if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(src + d.off_min));
+    if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(src + d.off_max));
+  }
+}
+
 template <int NV, bool F64>
 __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t (&rk)[kRegSlots], uint8_t* sm, int tid,
                                           const RowIn<NV, F64>& x, int64_t r) {
@@ -205,8 +264,16 @@ __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t
       for (int s = 0; s < L; ++s) rk[s] = ~*(volatile uint64_t*)&dir[s];
       go = true;
     } else {
-      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
-      if (e) update_entry_slow(p, e, r);
+      uint8_t* e = nullptr;
+      if (p.smem_cap && x.fast && !special)     // mid-G: CTA shared-memory table
+        e = smem_find_or_insert(sm + (size_t)kRegSlots * p.priv_rec * kFusedThreads, (uint32_t)p.smem_cap, p.stride,
+                                x.key);
+      if (e) {
+        entry_add_fast<NV, F64>(p, e, x);
+      } else {
+        e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+        if (e) update_entry_slow(p, e, r);
+      }
     }
   }
   if (go) privg_add<NV, F64>(p, sm, slot, tid, x);
@@ -222,7 +289,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   const int tid = threadIdx.x, lane = tid & 31;
   {
     uint4* z = (uint4*)sm;
-    const int n16 = (int)((size_t)L * p.priv_rec * T / 16);
+    const int n16 = (int)(((size_t)L * p.priv_rec * T + (size_t)p.smem_cap * p.stride) / 16);
     for (int i = tid; i < n16; i += T) z[i] = make_uint4(0, 0, 0, 0);
   }
   for (int i = tid; i < L * 32; i += T) blk[i] = 0;
@@ -294,24 +361,16 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   __syncthreads();
   // one thread per slot pushes the block entry into the global table
   if (tid < L) {
-    const int s = tid;
-    uint64_t sk = dir[s];
-    if (sk != 0) {
-      const uint8_t* be = blkb + s * 256;
-      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
-      if (e) {
-        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(be + 8));
-        for (int v = 0; v < p.nvals; ++v) {
-          const DevValue& d = p.vals[v];
-          if (d.off_sum >= 0) {
-            if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(be + d.off_sum));
-            else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(be + d.off_sum),
-                                 *(const uint64_t*)(be + d.off_sum + 8));
-          }
-          if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(be + d.off_min));
-          if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(be + d.off_max));
-        }
-      }
+    const uint64_t sk = dir[tid];
+    if (sk != 0) entry_merge_global(p, ~sk, blkb + tid * 256);
+  }
+  // the CTA's shared-memory table (mid-G): one thread per occupied entry
+  if (p.smem_cap) {
+    const uint8_t* tab = sm + (size_t)L * p.priv_rec * T;
+    for (int i = tid; i < p.smem_cap; i += T) {
+      const uint8_t* e = tab + (size_t)i * p.stride;
+      const uint64_t sk = *(const uint64_t*)e;
+      if (sk != 0) entry_merge_global(p, ~sk, e);
     }
   }
 }
@@ -373,7 +432,9 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant
 // ------------------------------------------------------------------ dispatch
 constexpr int kUnits = 2;
 
-static size_t reg_smem(const Plan& p) { return (size_t)kRegSlots * p.priv_rec * kFusedThreads; }
+static size_t reg_smem(const Plan& p) {
+  return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.stride;
+}
 
 template <int NV, bool F64>
 static cudaError_t launch_reg_nv(const Plan& p, int grid, cudaStream_t s) {

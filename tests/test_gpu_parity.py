@@ -240,8 +240,20 @@ def test_fused_many_groups(G):
     preds = [(sw["p"], {"hi": 499999})]
     aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
             {"op": "avg", "a": 0}]
-    for tier in (1, 2):
+    for tier in (0, 1, 2, 3, 4):
         _check_sga(preds, [sw["key"]], [sw["v"]], aggs, expected_groups=G, tier=tier)
+
+
+@pytest.mark.parametrize("G,s,sel", [(16, 0.0, 10**6), (256, 1.5, 5 * 10**5), (4096, 1.0, 10**4), (1 << 16, 1.5, 10**6),
+                                     (1 << 20, 0.0, 5 * 10**5)])
+def test_fused_sweep_c5_shape(G, s, sel):
+    """C5 sweep points (scaled to 2^21 rows): count, sum, min, max of v (+ fp64 sum/avg of v/100), auto tier."""
+    n = 1 << 21
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, G, s=s, f64=True)
+    preds = [(sw["p"], {"hi": sel - 1})]
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
+            {"op": "sum", "a": 1}, {"op": "avg", "a": 1}]
+    _check_sga(preds, [sw["key"]], [sw["v"], sw["v_f"]], aggs, expected_groups=G)
 
 
 def test_fused_edge_cases():
