@@ -292,13 +292,12 @@ constexpr size_t kRegTierSmem = 200 * 1024;
 bool use_reg_tier(const ocl_sga_args* a, const Plan& p) {
   if (a->tier == 1 || a->tier == 3 || a->tier == 4) return true;
   if (a->tier == 2) return false;
-  if (a->expected_groups <= reg_tier_slots()) return true;
-  return p.smem_cap > 0;
+  return true;   // auto: private slots catch the hot keys, warp-aggregated HBM updates the rest
 }
 
 // CTA shared-table capacity for the register tier (0 = none).
 int32_t plan_smem_cap(const ocl_sga_args* a, const Plan& p) {
-  bool want = a->tier == 4 || (a->tier == 0 && a->expected_groups > reg_tier_slots());
+  bool want = a->tier == 4;   // 64-bit shared-memory atomics are CAS loops on sm_100: opt-in only
   if (!want) return 0;
   size_t priv = (size_t)reg_tier_slots() * p.priv_rec * 256;
   if (priv >= kRegTierSmem) return 0;

@@ -247,9 +247,74 @@ __device__ __forceinline__ void entry_merge_global(const Plan& p, uint64_t key, 
   }
 }
 
+// Per-warp staging of rows that miss the private slots: the warp groups them by key
+// (__match_any_sync) and one leader per distinct key applies the group's combined
+// contribution to the HBM table — hot keys of skewed (Zipf) inputs and runs of
+// clustered keys cost one atomic update per warp instead of one per row.
+template <int NV, bool F64>
+struct MissStage {
+  int64_t vi[F64 ? 1 : NV][32];
+  double vd[F64 ? NV : 1][32];
+};
+
+template <int NV, bool F64>
+__device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F64>& st, bool miss, const RowIn<NV, F64>& x,
+                                                 int lane) {
+  const unsigned mmask = __ballot_sync(0xffffffffu, miss);
+  if (mmask == 0) return;
+  if (miss) {
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if constexpr (F64) st.vd[v][lane] = x.vd[v];
+      else st.vi[v][lane] = x.vi[v];
+    }
+  }
+  __syncwarp();
+  if (miss) {
+    const unsigned peers = __match_any_sync(mmask, x.key);
+    if (lane == __ffs(peers) - 1) {
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+      if (e) {
+        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)__popc(peers));
+#pragma unroll
+        for (int v = 0; v < NV; ++v) {
+          if (v >= p.nvals) break;
+          const DevValue& d = p.vals[v];
+          if constexpr (F64) {
+            double sum = 0.0, mn = x.vd[v], mx = x.vd[v];
+            for (unsigned b = peers; b; b &= b - 1) {
+              const double y = st.vd[v][__ffs(b) - 1];
+              sum += y;
+              mn = fmin(mn, y);
+              mx = fmax(mx, y);
+            }
+            if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), sum);
+            if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mn));
+            if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mx));
+          } else {
+            if (d.is_f64) continue;
+            I128 sum{0, 0};
+            int64_t mn = x.vi[v], mx = x.vi[v];
+            for (unsigned b = peers; b; b &= b - 1) {
+              const int64_t y = st.vi[v][__ffs(b) - 1];
+              sum = i128_add(sum, i128_from_i64(y));
+              mn = min(mn, y);
+              mx = max(mx, y);
+            }
+            if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), sum.lo, sum.hi);
+            if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
+            if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
+          }
+        }
+      }
+    }
+  }
+  __syncwarp();
+}
+
 template <int NV, bool F64>
 __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t (&rk)[kRegSlots], uint8_t* sm, int tid,
-                                          const RowIn<NV, F64>& x, int64_t r) {
+                                          MissStage<NV, F64>& stage, const RowIn<NV, F64>& x, int64_t r) {
   constexpr int L = kRegSlots;
   int slot = -1;
 #pragma unroll
@@ -257,7 +322,8 @@ __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t
     if (x.key == rk[s]) slot = s;
   const bool special = x.key == ~0ULL;
   bool go = x.q && x.fast && slot >= 0 && !special;
-  if (x.q && !go) {                       // rare after warm-up: new key in this CTA, or slow value
+  bool miss = false;
+  if (x.q && !go) {                       // new key in this CTA, a slow value, or more keys than slots
     slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, x.key) : -1;
     if (slot >= 0) {
 #pragma unroll
@@ -265,11 +331,13 @@ __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t
       go = true;
     } else {
       uint8_t* e = nullptr;
-      if (p.smem_cap && x.fast && !special)     // mid-G: CTA shared-memory table
+      if (p.smem_cap && x.fast && !special)     // tier 4: CTA shared-memory table
         e = smem_find_or_insert(sm + (size_t)kRegSlots * p.priv_rec * kFusedThreads, (uint32_t)p.smem_cap, p.stride,
                                 x.key);
       if (e) {
         entry_add_fast<NV, F64>(p, e, x);
+      } else if (x.fast && !special) {
+        miss = true;                            // warp-aggregated HBM update below
       } else {
         e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
         if (e) update_entry_slow(p, e, r);
@@ -277,6 +345,7 @@ __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t
     }
   }
   if (go) privg_add<NV, F64>(p, sm, slot, tid, x);
+  warp_miss_update<NV, F64>(p, stage, miss, x, tid & 31);
 }
 
 template <int NV, bool F64, int U>
@@ -298,6 +367,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   uint64_t rk[L];
 #pragma unroll
   for (int s = 0; s < L; ++s) rk[s] = ~0ULL;   // ~0 never matches a slot (special key)
+  __shared__ MissStage<NV, F64> stages[kFusedThreads / 32];
+  MissStage<NV, F64>& stage = stages[tid >> 5];
 
   constexpr int kTile = 64 * U;
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
@@ -317,8 +388,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
         eval_row_scalar<NV, F64>(p, r + 1, x1);
       }
       if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-      privg_row<NV, F64>(p, dir, rk, sm, tid, x0, r);
-      privg_row<NV, F64>(p, dir, rk, sm, tid, x1, r + 1);
+      privg_row<NV, F64>(p, dir, rk, sm, tid, stage, x0, r);
+      privg_row<NV, F64>(p, dir, rk, sm, tid, stage, x1, r + 1);
     }
   }
 
@@ -402,35 +473,121 @@ __device__ __forceinline__ void glb_row(const Plan& p, const RowIn<NV, F64>& x, 
   }
 }
 
+// Warp-level run combining before the HBM atomics (many-groups tier).  Lanes own
+// consecutive rows, so runs of equal keys (clustered inputs such as lineitem
+// ordered by orderkey, or hot keys) are contiguous lane ranges: one segmented
+// shuffle reduction folds each run into its first lane, which alone touches the
+// table.  Rows that are not eligible (slow values, the key ~0) take the per-row path.
+template <int NV, bool F64>
+__device__ __forceinline__ void glb_unit(const Plan& p, const RowIn<NV, F64>& x, int64_t r, int lane) {
+  const bool ok = x.q && x.fast && x.key != ~0ULL;
+  const unsigned okmask = __ballot_sync(0xffffffffu, ok);
+  const uint64_t kprev = __shfl_up_sync(0xffffffffu, x.key, 1);
+  const bool cont = ok && lane > 0 && ((okmask >> (lane - 1)) & 1u) && kprev == x.key;
+  const unsigned contmask = __ballot_sync(0xffffffffu, cont);
+  if (contmask == 0) {                   // no run in this unit (shuffled / high-cardinality): per row
+    glb_row<NV, F64>(p, x, r);
+    return;
+  }
+  if (x.q && !ok) glb_row<NV, F64>(p, x, r);
+  const unsigned later = lane == 31 ? 0u : (~contmask & ~((2u << lane) - 1u));   // segment starts after me
+  const int seg_end = later ? __ffs(later) - 2 : 31;
+  uint32_t c = ok ? 1u : 0u;
+  I128 si[F64 ? 1 : NV];
+  double sd[F64 ? NV : 1], mnd[F64 ? NV : 1], mxd[F64 ? NV : 1];
+  int64_t mni[F64 ? 1 : NV], mxi[F64 ? 1 : NV];
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if constexpr (F64) {
+      sd[v] = ok ? x.vd[v] : 0.0;
+      mnd[v] = x.vd[v];
+      mxd[v] = x.vd[v];
+    } else {
+      si[v] = ok ? i128_from_i64(x.vi[v]) : I128{0, 0};
+      mni[v] = x.vi[v];
+      mxi[v] = x.vi[v];
+    }
+  }
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const bool take = lane + o <= seg_end;
+    c += take ? __shfl_down_sync(0xffffffffu, c, o) : 0u;
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if (v >= p.nvals) break;
+      const DevValue& d = p.vals[v];
+      if constexpr (F64) {
+        double y = __shfl_down_sync(0xffffffffu, sd[v], o);
+        if (take) sd[v] += y;
+        if (d.off_min >= 0) { double z = __shfl_down_sync(0xffffffffu, mnd[v], o); if (take) mnd[v] = fmin(mnd[v], z); }
+        if (d.off_max >= 0) { double z = __shfl_down_sync(0xffffffffu, mxd[v], o); if (take) mxd[v] = fmax(mxd[v], z); }
+      } else {
+        if (d.off_sum >= 0) {
+          I128 y;
+          y.lo = __shfl_down_sync(0xffffffffu, si[v].lo, o);
+          y.hi = __shfl_down_sync(0xffffffffu, si[v].hi, o);
+          if (take) si[v] = i128_add(si[v], y);
+        }
+        if (d.off_min >= 0) {
+          int64_t z = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mni[v], o);
+          if (take) mni[v] = min(mni[v], z);
+        }
+        if (d.off_max >= 0) {
+          int64_t z = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mxi[v], o);
+          if (take) mxi[v] = max(mxi[v], z);
+        }
+      }
+    }
+  }
+  if (!ok || cont) return;                // run heads only
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+  if (!e) return;
+  atomicAdd((unsigned long long*)(e + 8), (unsigned long long)c);
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if constexpr (F64) {
+      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), sd[v]);
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mnd[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mxd[v]));
+    } else {
+      if (d.is_f64) continue;
+      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), si[v].lo, si[v].hi);
+      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mni[v]));
+      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mxi[v]));
+    }
+  }
+}
+
 template <int NV, bool F64, int U>
 __global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant__ Plan p) {
   const int lane = threadIdx.x & 31;
-  constexpr int kTile = 64 * U;
+  constexpr int kTile = 32 * U;            // lane l owns rows base + 32u + l: consecutive rows across lanes
   const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
   const int64_t ntiles = (p.n + kTile - 1) / kTile;
   for (int64_t t = warp; t < ntiles; t += nwarps) {
     const int64_t base = t * kTile;
-    const bool vec = p.vec_ok && base + kTile <= p.n;
+    RowIn<NV, F64> x[U];
+#pragma unroll
+    for (int u = 0; u < U; ++u) eval_row_scalar<NV, F64>(p, base + 32 * u + lane, x[u]);
 #pragma unroll
     for (int u = 0; u < U; ++u) {
-      const int64_t r = base + 64 * u + 2 * lane;
-      RowIn<NV, F64> x0, x1;
-      if (vec) {
-        eval_pair_vec<NV, F64>(p, r, x0, x1);
-      } else {
-        eval_row_scalar<NV, F64>(p, r, x0);
-        eval_row_scalar<NV, F64>(p, r + 1, x1);
+      const int64_t r = base + 32 * u + lane;
+      if (p.bitmap_out) {
+        const uint32_t w = __ballot_sync(0xffffffffu, x[u].q);
+        const int64_t wi = r >> 5;
+        if (lane == 0 && wi < ((p.n + 31) >> 5)) p.bitmap_out[wi] = w;
       }
-      if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-      glb_row<NV, F64>(p, x0, r);
-      glb_row<NV, F64>(p, x1, r + 1);
+      glb_unit<NV, F64>(p, x[u], r, lane);
     }
   }
 }
 
 // ------------------------------------------------------------------ dispatch
 constexpr int kUnits = 2;
+constexpr int kGlbUnits = 4;
 
 static size_t reg_smem(const Plan& p) {
   return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.stride;
@@ -458,10 +615,10 @@ static cudaError_t launch_reg_f(const Plan& p, int grid, cudaStream_t s) {
 template <bool F64>
 static cudaError_t launch_glb_f(const Plan& p, int grid, cudaStream_t s) {
   count_launch();
-  if (p.nvals <= 1) k_sga_glb<1, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else if (p.nvals <= 2) k_sga_glb<2, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else if (p.nvals <= 4) k_sga_glb<4, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else k_sga_glb<6, F64, kUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  if (p.nvals <= 1) k_sga_glb<1, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 2) k_sga_glb<2, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 4) k_sga_glb<4, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  else k_sga_glb<6, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
   return cudaGetLastError();
 }
 
@@ -470,7 +627,7 @@ int reg_tier_slots() { return kRegSlots; }
 template <int NV, bool F64>
 static const void* reg_kernel_ptr() { return (const void*)k_sga_reg<NV, F64, kUnits>; }
 template <int NV, bool F64>
-static const void* glb_kernel_ptr() { return (const void*)k_sga_glb<NV, F64, kUnits>; }
+static const void* glb_kernel_ptr() { return (const void*)k_sga_glb<NV, F64, kGlbUnits>; }
 
 // Resident CTAs per SM of the instantiation launch_fused would pick (persistent grid sizing).
 int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64) {
