@@ -295,17 +295,19 @@ bool use_reg_tier(const ocl_sga_args* a, const Plan& p) {
   return true;   // auto: private slots catch the hot keys, warp-aggregated HBM updates the rest
 }
 
-// CTA shared-table capacity for the register tier (0 = none).
+// CTA shared-table capacity for the register tier (0 = none).  Eligible plans:
+// every value an integer column (its fast path is int32, the table's field width).
 int32_t plan_smem_cap(const ocl_sga_args* a, const Plan& p) {
-  bool want = a->tier == 4;   // 64-bit shared-memory atomics are CAS loops on sm_100: opt-in only
-  if (!want) return 0;
-  size_t priv = (size_t)reg_tier_slots() * p.priv_rec * 256;
+  if (a->tier == 2 || a->tier == 3) return 0;
+  for (int v = 0; v < p.nvals; ++v)
+    if (p.vals[v].is_f64 || p.vals[v].expr != OCL_EXPR_COL) return 0;
+  const size_t priv = (size_t)reg_tier_slots() * p.priv_rec * 256;
   if (priv >= kRegTierSmem) return 0;
-  uint64_t cap = next_pow2((uint64_t)std::max<int64_t>(2 * a->expected_groups, 64));
-  uint64_t fit = (kRegTierSmem - priv) / (size_t)p.stride;
-  while (cap > fit) cap >>= 1;
-  if (a->tier == 0 && (int64_t)cap < 2 * a->expected_groups) return 0;   // would overflow: use the HBM tier
-  return (int32_t)(cap >= 64 ? cap : 0);
+  const uint64_t fit = next_pow2((kRegTierSmem - priv) / (size_t)p.cta_stride + 1) / 2;   // largest pow2 that fits
+  if (a->tier == 4) return (int32_t)std::min<uint64_t>(fit, 1u << 14);
+  if (a->expected_groups <= reg_tier_slots()) return 0;
+  const uint64_t cap = next_pow2((uint64_t)std::max<int64_t>(2 * a->expected_groups, 64));
+  return cap <= fit ? (int32_t)cap : 0;     // too many groups for shared memory: HBM table
 }
 
 ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true) {
@@ -341,6 +343,17 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   P->table_bytes = align_up((P->cap + 1) * (size_t)p.stride, 256);
   p.status = a->dev_status;
   p.bitmap_out = a->bitmap_out;
+  {   // CTA-table entry layout: [~key u64][count u32] per value [lo16 sum][hi16 sum][min][max]
+    int co = 12;
+    for (int v = 0; v < p.nvals; ++v) {
+      DevValue& d = p.vals[v];
+      d.co_lo = d.co_hi = d.co_min = d.co_max = -1;
+      if (d.off_sum >= 0) { d.co_lo = co; d.co_hi = co + 4; co += 8; }
+      if (d.off_min >= 0) { d.co_min = co; co += 4; }
+      if (d.off_max >= 0) { d.co_max = co; co += 4; }
+    }
+    p.cta_stride = (int)align_up((size_t)co, 8);
+  }
   p.smem_cap = plan_smem_cap(a, p);
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;

@@ -135,6 +135,7 @@ struct DevValue {
   int32_t is_f64;
   int32_t off_sum, off_min, off_max;  // entry byte offsets, -1 if that state is not needed
   int32_t po_sum, po_hi, po_min, po_max;  // private-accumulator field offsets (bytes per thread), -1 if absent
+  int32_t co_lo, co_hi, co_min, co_max;   // CTA-table 32-bit field offsets (bytes in the entry), -1 if absent
   int64_t S;                          // 10^scale
   double Sf;
 };
@@ -153,6 +154,7 @@ struct Plan {
   int32_t has_minmax;
   int32_t priv_rec;     // private accumulator record: bytes per thread per group slot
   int32_t smem_cap;     // register tier: per-CTA shared-memory hash table entries (0 = none; power of two)
+  int32_t cta_stride;   // bytes per CTA-table entry
   int32_t* status;      // device status word (may be null)
   uint32_t* bitmap_out; // optional selection bitmap
   const int32_t* gids;  // unfused aggregate: direct group ids (table indexed by gid)

@@ -188,10 +188,17 @@ __device__ __forceinline__ void privg_add(const Plan& p, uint8_t* sm, int slot, 
   }
 }
 
-// Per-CTA shared-memory hash table (mid-G overflow of the private slots, P:L564-568
-// local-memory aggregation tables): linear probing with shared-memory atomicCAS,
-// at most kSmemProbes probes, then the row goes to the HBM table.
-constexpr int kSmemProbes = 32;
+// Per-CTA shared-memory hash table (mid G: more distinct keys than private slots;
+// the paper's per-work-group local-memory aggregation tables).
+// sm_100 has no native 64-bit shared-memory atomic add/max (they lower to CAS
+// loops), so the table uses 32-bit fields and native 32-bit atomics only:
+//   [~key u64][count u32] per value: [sum of low 16 bits u32][sum of high 16 bits s32]
+//   [min u32][max u32] (order-preserving encodings, 0 = identity).
+// Values are int32 on this path (fast-path COL values), so each field absorbs 2^16
+// updates exactly; the CTA flushes the table into the HBM table every 2^16 rows.
+// Linear probing with 64-bit shared atomicCAS on the key, at most kSmemProbes probes.
+constexpr int kSmemProbes = 16;
+constexpr int kCtaFlushRounds = 64;   // rounds of (warps x tile) rows = 64 x 8 x 128 = 65,536 rows
 
 __device__ __forceinline__ uint8_t* smem_find_or_insert(uint8_t* tab, uint32_t cap, int32_t stride, uint64_t key) {
   const uint64_t sk = ~key;
@@ -209,25 +216,53 @@ __device__ __forceinline__ uint8_t* smem_find_or_insert(uint8_t* tab, uint32_t c
   return nullptr;
 }
 
-// Row contribution with atomics on an entry (shared or global) from fast-path values.
+__device__ __forceinline__ uint32_t enc32_max(int32_t v) { return (uint32_t)v ^ 0x80000000u; }
+__device__ __forceinline__ uint32_t enc32_min(int32_t v) { return ~enc32_max(v); }
+
 template <int NV, bool F64>
-__device__ __forceinline__ void entry_add_fast(const Plan& p, uint8_t* e, const RowIn<NV, F64>& x) {
-  atomicAdd((unsigned long long*)(e + 8), 1ULL);
+__device__ __forceinline__ void cta_add(const Plan& p, uint8_t* e, const RowIn<NV, F64>& x) {
+  atomicAdd((unsigned int*)(e + 8), 1u);
+  if constexpr (!F64) {
 #pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (F64) {
-      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), x.vd[v]);
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(x.vd[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(x.vd[v]));
-    } else {
-      if (d.is_f64) continue;
-      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)x.vi[v], (uint64_t)(x.vi[v] >> 63));
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(x.vi[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(x.vi[v]));
+    for (int v = 0; v < NV; ++v) {
+      if (v >= p.nvals) break;
+      const DevValue& d = p.vals[v];
+      const int32_t w = (int32_t)x.vi[v];
+      if (d.co_lo >= 0) {
+        atomicAdd((unsigned int*)(e + d.co_lo), (unsigned int)w & 0xFFFFu);
+        atomicAdd((int*)(e + d.co_hi), w >> 16);
+      }
+      if (d.co_min >= 0) atomicMax((unsigned int*)(e + d.co_min), enc32_min(w));
+      if (d.co_max >= 0) atomicMax((unsigned int*)(e + d.co_max), enc32_max(w));
     }
   }
+}
+
+// Fold one CTA-table entry into the HBM table and reset its accumulators (key kept).
+__device__ __forceinline__ void cta_flush_entry(const Plan& p, uint8_t* ce) {
+  const uint64_t sk = *(const uint64_t*)ce;
+  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+  if (sk == 0 || cnt == 0) return;
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
+  if (e) {
+    atomicAdd((unsigned long long*)(e + 8), (unsigned long long)cnt);
+    for (int v = 0; v < p.nvals; ++v) {
+      const DevValue& d = p.vals[v];
+      if (d.co_lo >= 0) {
+        const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
+        atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)sum, (uint64_t)(sum >> 63));
+      }
+      if (d.co_min >= 0) {
+        const int32_t mn = (int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u);
+        atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
+      }
+      if (d.co_max >= 0) {
+        const int32_t mx = (int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u);
+        atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
+      }
+    }
+  }
+  for (int w = 8; w < p.cta_stride; w += 4) *(uint32_t*)(ce + w) = 0;
 }
 
 // Merge a whole entry (shared-memory table or CTA block entry) into the HBM table.
@@ -331,11 +366,11 @@ __device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t
       go = true;
     } else {
       uint8_t* e = nullptr;
-      if (p.smem_cap && x.fast && !special)     // tier 4: CTA shared-memory table
-        e = smem_find_or_insert(sm + (size_t)kRegSlots * p.priv_rec * kFusedThreads, (uint32_t)p.smem_cap, p.stride,
-                                x.key);
+      if (p.smem_cap && x.fast && !special)     // mid G: CTA shared-memory table
+        e = smem_find_or_insert(sm + (size_t)kRegSlots * p.priv_rec * kFusedThreads, (uint32_t)p.smem_cap,
+                                p.cta_stride, x.key);
       if (e) {
-        entry_add_fast<NV, F64>(p, e, x);
+        cta_add<NV, F64>(p, e, x);
       } else if (x.fast && !special) {
         miss = true;                            // warp-aggregated HBM update below
       } else {
@@ -358,7 +393,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   const int tid = threadIdx.x, lane = tid & 31;
   {
     uint4* z = (uint4*)sm;
-    const int n16 = (int)(((size_t)L * p.priv_rec * T + (size_t)p.smem_cap * p.stride) / 16);
+    const int n16 = (int)(((size_t)L * p.priv_rec * T + (size_t)p.smem_cap * p.cta_stride) / 16);
     for (int i = tid; i < n16; i += T) z[i] = make_uint4(0, 0, 0, 0);
   }
   for (int i = tid; i < L * 32; i += T) blk[i] = 0;
@@ -374,7 +409,19 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
   const int64_t ntiles = (p.n + kTile - 1) / kTile;
-  for (int64_t t = warp; t < ntiles; t += nwarps) {
+  // CTA-uniform round count (warp 0 of the CTA has the most tiles) so the whole CTA
+  // can meet at the periodic CTA-table flushes
+  const int64_t first = (int64_t)blockIdx.x * (T / 32);
+  const int64_t rounds = ntiles > first ? (ntiles - first + nwarps - 1) / nwarps : 0;
+  uint8_t* cta_tab = sm + (size_t)L * p.priv_rec * T;
+  for (int64_t round = 0; round < rounds; ++round) {
+    if (p.smem_cap && round > 0 && round % kCtaFlushRounds == 0) {
+      __syncthreads();
+      for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
+      __syncthreads();
+    }
+    const int64_t t = warp + round * nwarps;
+    if (t >= ntiles) continue;
     const int64_t base = t * kTile;
     const bool vec = p.vec_ok && base + kTile <= p.n;
 #pragma unroll
@@ -436,14 +483,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
     if (sk != 0) entry_merge_global(p, ~sk, blkb + tid * 256);
   }
   // the CTA's shared-memory table (mid-G): one thread per occupied entry
-  if (p.smem_cap) {
-    const uint8_t* tab = sm + (size_t)L * p.priv_rec * T;
-    for (int i = tid; i < p.smem_cap; i += T) {
-      const uint8_t* e = tab + (size_t)i * p.stride;
-      const uint64_t sk = *(const uint64_t*)e;
-      if (sk != 0) entry_merge_global(p, ~sk, e);
-    }
-  }
+  if (p.smem_cap)
+    for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
 }
 
 // ------------------------------------------------------------------ global tier
@@ -511,7 +552,8 @@ __device__ __forceinline__ void glb_unit(const Plan& p, const RowIn<NV, F64>& x,
 #pragma unroll
   for (int o = 1; o < 32; o <<= 1) {
     const bool take = lane + o <= seg_end;
-    c += take ? __shfl_down_sync(0xffffffffu, c, o) : 0u;
+    const uint32_t cy = __shfl_down_sync(0xffffffffu, c, o);   // every lane shuffles; `take` selects
+    if (take) c += cy;
 #pragma unroll
     for (int v = 0; v < NV; ++v) {
       if (v >= p.nvals) break;
@@ -590,7 +632,7 @@ constexpr int kUnits = 2;
 constexpr int kGlbUnits = 4;
 
 static size_t reg_smem(const Plan& p) {
-  return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.stride;
+  return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.cta_stride;
 }
 
 template <int NV, bool F64>
