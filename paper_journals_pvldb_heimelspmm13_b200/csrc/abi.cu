@@ -215,12 +215,27 @@ ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* agg
       rec = (int)align_up((size_t)rec, 8);
       d.po_sum = rec;
       rec += 8;
-      if (!d.is_f64) { d.po_hi = rec; rec += 4; }
+      if (!d.is_f64 && d.expr != OCL_EXPR_COL) { d.po_hi = rec; rec += 4; }   // products: 96-bit
     }
     if (need_min[v]) { rec = (int)align_up((size_t)rec, 8); d.po_min = rec; rec += 8; }
     if (need_max[v]) { rec = (int)align_up((size_t)rec, 8); d.po_max = rec; rec += 8; }
   }
   p.priv_rec = (int)align_up((size_t)rec, 8);
+  // distinct operand columns (static shapes load each once) and per-value indices
+  p.ncols = 0;
+  auto col_index = [&](const DevCol& c) -> int {
+    for (int i = 0; i < p.ncols; ++i)
+      if (p.vcols[i].ptr == c.ptr && p.vcols[i].dtype == c.dtype) return i;
+    if (p.ncols == kMaxCols) return -1;
+    p.vcols[p.ncols] = c;
+    return p.ncols++;
+  };
+  for (int v = 0; v < p.nvals; ++v) {
+    DevValue& d = p.vals[v];
+    d.ia = col_index(d.a);
+    d.ib = d.expr >= OCL_EXPR_MUL_1MINUS ? col_index(d.b) : 0;
+    d.ic = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? col_index(d.c) : 0;
+  }
   int stride = (int)align_up((size_t)off, 16);
   if (stride <= 32) stride = 32;
   else if (stride <= 64) stride = 64;
@@ -279,6 +294,11 @@ ocl_status plan_preds(const ocl_column* pred_cols, const ocl_range* preds, int32
     d.is_f64 = pred_cols[i].dtype == OCL_F64;
     d.anti = preds[i].anti ? 1 : 0;
     normalise_range(preds[i], &d.lo, &d.hi, &d.flo, &d.fhi);
+    if (d.lo > d.hi || d.lo > INT32_MAX || d.hi < INT32_MIN) { d.lo32 = 1; d.hi32 = 0; }   // empty range
+    else {
+      d.lo32 = (int32_t)std::max<int64_t>(d.lo, INT32_MIN);
+      d.hi32 = (int32_t)std::min<int64_t>(d.hi, INT32_MAX);
+    }
   }
   return OCL_OK;
 }
@@ -286,19 +306,19 @@ ocl_status plan_preds(const ocl_column* pred_cols, const ocl_range* preds, int32
 // Shared-memory budget of one register-tier CTA (private records + mid-G table).
 constexpr size_t kRegTierSmem = 200 * 1024;
 
-// Tiers: <= 4 expected groups -> private slots only; <= the CTA
-// table capacity -> private slots + per-CTA shared-memory hash table; else the
-// HBM table.  tier 1/3/4 force the register tier (4: with the shared table).
-bool use_reg_tier(const ocl_sga_args* a, const Plan& p) {
-  if (a->tier == 1 || a->tier == 3 || a->tier == 4) return true;
-  if (a->tier == 2) return false;
-  return true;   // auto: private slots catch the hot keys, warp-aggregated HBM updates the rest
+// Tier selection: 0 auto; 1 register tier (private slots + HBM);
+// 2 HBM-only kernel; 3 register tier with the dynamic (unspecialised) shape;
+// 4 register tier with the CTA shared-memory table forced on.
+int fused_mode(const ocl_sga_args* a) {
+  if (a->tier == 2) return 2;
+  if (a->tier == 3) return 1;
+  return 0;
 }
 
 // CTA shared-table capacity for the register tier (0 = none).  Eligible plans:
 // every value an integer column (its fast path is int32, the table's field width).
 int32_t plan_smem_cap(const ocl_sga_args* a, const Plan& p) {
-  if (a->tier == 2 || a->tier == 3) return 0;
+  if (a->tier == 1 || a->tier == 2 || a->tier == 3) return 0;
   for (int v = 0; v < p.nvals; ++v)
     if (p.vals[v].is_f64 || p.vals[v].expr != OCL_EXPR_COL) return 0;
   const size_t priv = (size_t)reg_tier_slots() * p.priv_rec * 256;
@@ -367,10 +387,6 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
 }
 
 
-int fused_grid(ocl_ctx* ctx, const Planned& P, bool reg) {
-  return ctx->sms * fused_blocks_per_sm(P.plan, reg, P.values_f64);
-}
-
 // table + finalize workspace of a fused call
 size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) { return P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256); }
 
@@ -384,13 +400,9 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   OCL_CUDA(cudaMemsetAsync(ws, 0, P.table_bytes, s), "table init");
   if (a->dev_status) OCL_CUDA(cudaMemsetAsync(a->dev_status, 0, sizeof(int32_t), s), "status init");
   if (P.plan.n > 0) {
-    bool reg = use_reg_tier(a, P.plan);
     if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, s), "profile event");
-    cudaError_t err = cudaSuccess;
     int kind = 0;
-    if (!(reg && a->tier != 3 && P.plan.smem_cap == 0 && launch_fused_spec(P.plan, ctx->sms, s, &err, &kind)))
-      err = launch_fused(P.plan, reg, P.values_f64, fused_grid(ctx, P, reg), s);
-    OCL_CUDA(err, "fused kernel launch");
+    OCL_CUDA(launch_fused(P.plan, fused_mode(a), P.values_f64, ctx->sms, s, &kind), "fused kernel launch");
     ctx->last_kernel = kind;
     if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, s), "profile event");
   }
@@ -829,8 +841,7 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
   p.table = table;
   p.status = d_status;
   p.bitmap_out = nullptr;
-  const bool reg = use_reg_tier(args, P.plan);
-  const int grid = fused_grid(ctx, P, reg);
+  const int mode = fused_mode(args);
   const int64_t n = P.plan.n;
   int64_t nchunks = (n + chunk_rows - 1) / chunk_rows;
   for (int64_t c = 0; c < nchunks; ++c) {
@@ -851,13 +862,15 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
     };
     for (int i = 0; i < q.npreds; ++i) remap(q.preds[i].col);
     for (int i = 0; i < q.nkeys; ++i) remap(q.keys[i].col);
+    for (int i = 0; i < q.ncols; ++i) remap(q.vcols[i]);
     for (int v = 0; v < q.nvals; ++v) {
       remap(q.vals[v].a);
       if (q.vals[v].expr >= OCL_EXPR_MUL_1MINUS) remap(q.vals[v].b);
       if (q.vals[v].expr >= OCL_EXPR_MUL_1MINUS_1PLUS) remap(q.vals[v].c);
     }
     q.vec_ok = 1;   // staging buffers are 256-byte aligned
-    OCL_CUDA(launch_fused(q, reg, P.values_f64, grid, ks), "fused kernel (chunk)");
+    int kind = 0;
+    OCL_CUDA(launch_fused(q, mode, P.values_f64, ctx->sms, ks, &kind), "fused kernel (chunk)");
     OCL_CUDA(cudaEventRecord(ctx->ev_consumed[sl], ks), "event");
   }
   EmitArgs ea;

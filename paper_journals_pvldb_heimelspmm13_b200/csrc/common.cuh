@@ -119,6 +119,7 @@ struct DevPred {
   int32_t is_f64;
   int32_t anti;
   int64_t lo, hi;     // normalised inclusive integer bounds (lo > hi: empty range)
+  int32_t lo32, hi32; // the same clamped to int32 (u8 / i32 columns compare in 32 bits)
   double flo, fhi;    // normalised inclusive fp64 bounds
 };
 
@@ -136,6 +137,7 @@ struct DevValue {
   int32_t off_sum, off_min, off_max;  // entry byte offsets, -1 if that state is not needed
   int32_t po_sum, po_hi, po_min, po_max;  // private-accumulator field offsets (bytes per thread), -1 if absent
   int32_t co_lo, co_hi, co_min, co_max;   // CTA-table 32-bit field offsets (bytes in the entry), -1 if absent
+  int32_t ia, ib, ic;                 // operand indices into Plan::vcols (static shapes)
   int64_t S;                          // 10^scale
   double Sf;
 };
@@ -148,6 +150,9 @@ struct Plan {
   DevPred preds[kMaxPreds];
   DevKey keys[kMaxKeys];
   DevValue vals[kMaxVals];
+  int32_t ncols;        // distinct value columns (operands of all value expressions)
+  int32_t pad2_;
+  DevCol vcols[kMaxCols];
   uint8_t* table;       // cap + 1 entries (side entry last)
   uint64_t mask;        // cap - 1 (cap is a power of two)
   int32_t stride;       // entry bytes

@@ -1,186 +1,349 @@
 // fused.cu — K9: fused select -> hash group -> aggregate, one pass over the columns.
 //
-// Paper steps fused here: selection (§4.1.1), hash group-by
-// with dense group ids (L551-561 §4.1.6; hashing L511-533 §4.1.4), multi-column
-// grouping on combined ids (L559-561), hierarchical grouped aggregation with
-// per-work-group tables and several accumulators per group for few groups
-// (L562-600 §4.1.7).  Nothing is materialised: no bitmap (unless requested for
-// tests), no oid list, no gid column.
+// Paper steps fused here: selection (§4.1.1), hash group-by with
+// dense group ids (L551-561 §4.1.6; hashing L511-533 §4.1.4), multi-column grouping
+// on combined ids (L559-561), hierarchical grouped aggregation with per-work-group
+// tables and several accumulators per group for few groups (L562-600 §4.1.7).
+// Nothing is materialised: no bitmap (unless requested for tests), no oid list, no
+// gid column.
 //
-// B200 design (DESIGN.md §Kernels):
-//  * persistent grid (#SMs x resident CTAs); a warp owns tiles of 64*U rows; lane
-//    l handles rows (2l, 2l+1) of each 64-row unit, so every column is read with one
-//    vector load per lane per unit (u8: 2 B, i32: 8 B, i64/f64: 16 B) and every
-//    warp-wide load is a contiguous, fully-used run (P:L619-633 GPU pattern).
-//  * REGISTER tier (few groups): each thread keeps L private accumulator slots in
-//    registers — the limit of the paper's "multiple accumulators per group" idea:
-//    one accumulator set per thread, no atomics in the row loop.  A block-wide
-//    slot directory in shared memory gives every thread the same key -> slot map.
-//    Integer SUMs use 96-bit (lo64 + hi32) predicated add-with-carry chains: exact
-//    for any per-thread row count < 2^31 (the int128 state is formed at flush).
-//  * GLOBAL tier (many groups): find-or-insert in the HBM open-addressing table
-//    and update the entry with atomics (native f64 add, int128 as two u64 atomics).
-//  * Rows a tier cannot place (more than L keys in a block, int32-overflowing
-//    factors, the key ~0) take the exact int128 global path, so every tier is
-//    correct for every input; the tier only decides speed.
+// B200 design (DESIGN.md §6):
+//  * Persistent grid (#SMs x resident CTAs).  A warp owns tiles of 128 rows; lane l
+//    holds rows (2l, 2l+1) of each 64-row unit, so every column is read with one
+//    vector load per lane per unit (u8 2 B, i32 8 B, i64/f64 16 B) and every
+//    warp-wide load is one contiguous, fully used run (the paper's GPU pattern,
+//    P:L619-633).
+//  * Three places a qualifying row can be accumulated, tried in order:
+//    1. PRIVATE slots: each thread owns one accumulator record per group slot in
+//       shared memory ([slot][field][thread]); a CTA-wide directory maps the first 4
+//       distinct keys to slots.  A row costs one slot-indexed read-modify-write per
+//       accumulator: no atomics — the limit of the paper's "multiple accumulators
+//       per group".  Few-group queries (TPC-H Q1) live entirely here;
+//       with skewed keys the hot keys land here.
+//    2. CTA TABLE (mid G): a shared-memory hash table with native 32-bit atomics
+//       (sm_100 lowers 64-bit shared atomics to CAS loops): int32 values as 16-bit
+//       split sums, flushed to HBM every 2^16 rows.
+//    3. HBM TABLE: rows that miss are grouped per warp by key (__match_any_sync); one
+//       leader per distinct key applies the group's combined update with global
+//       atomics (int128 sums as two 64-bit atomics with carry from the returned value).
+//    Rows whose values need int128 (int32-overflowing factors), or the key ~0, take an
+//    exact per-row path.  Every path is exact; the tiers only decide speed.
+//  * The kernel is templated on a *shape*: DynShape reads the plan's column widths and
+//    expressions at run time (any plan); StaticShape<...> fixes them at compile time
+//    (no dtype dispatch, every value column loaded once, narrow keys in 32 bits) — the
+//    B200 stand-in for Ocelot's run-time kernel compilation.
+//    Plans whose shape matches an instantiated StaticShape run the specialised code.
+#include <type_traits>
+
 #include "launch.cuh"
 #include "rowops.cuh"
 
 namespace ocl {
 
 constexpr int kFusedThreads = 256;
+constexpr int kRegSlots = 4;
+constexpr int kUnits = 2;
+constexpr int kTileRows = 64 * kUnits;
 
-__device__ __forceinline__ void add96(bool pr, uint32_t& a0, uint32_t& a1, uint32_t& a2, int64_t v) {
-  uint32_t v0 = (uint32_t)(uint64_t)v, v1 = (uint32_t)((uint64_t)v >> 32), v2 = (uint32_t)(v >> 63);
-  asm("{\n\t.reg .pred p;\n\t"
-      "setp.ne.u32 p, %3, 0;\n\t"
-      "@p add.cc.u32 %0, %0, %4;\n\t"
-      "@p addc.cc.u32 %1, %1, %5;\n\t"
-      "@p addc.u32 %2, %2, %6;\n\t}"
-      : "+r"(a0), "+r"(a1), "+r"(a2)
-      : "r"((uint32_t)pr), "r"(v0), "r"(v1), "r"(v2));
+// ------------------------------------------------------------------ shapes
+enum : uint32_t { VF_SUM = 1, VF_MIN = 2, VF_MAX = 4 };
+// value descriptor: kind (2 bits) | a (3) | b (3) | c (3) | flags (3)
+__host__ __device__ constexpr uint32_t vop(uint32_t kind, uint32_t flags, uint32_t a, uint32_t b = 0,
+                                           uint32_t c = 0) {
+  return kind | (a << 2) | (b << 5) | (c << 8) | (flags << 11);
 }
 
-// Per-row inputs after predicate / key / value evaluation.
-template <int NV, bool F64>
-struct RowIn {
-  bool q;
-  bool fast;
-  uint64_t key;
+struct DynShape {
+  static constexpr bool kStatic = false;
+  static constexpr int NC = 1;
+  using Key = uint64_t;
+  __device__ static int np(const Plan& p) { return p.npreds; }
+  __device__ static int pw(const Plan& p, int i) { return p.preds[i].col.width; }
+  __device__ static bool pf64(const Plan& p, int i) { return p.preds[i].is_f64; }
+  __device__ static int nk(const Plan& p) { return p.nkeys; }
+  __device__ static int kw(const Plan& p, int i) { return p.keys[i].col.width; }
+  __device__ static int nv(const Plan& p) { return p.nvals; }
+  __device__ static int kind(const Plan& p, int v) { return p.vals[v].expr; }
+  __device__ static bool fsum(const Plan& p, int v) { return p.vals[v].off_sum >= 0; }
+  __device__ static bool fmn(const Plan& p, int v) { return p.vals[v].off_min >= 0; }
+  __device__ static bool fmx(const Plan& p, int v) { return p.vals[v].off_max >= 0; }
+  __device__ static bool vf64(const Plan& p, int v) { return p.vals[v].is_f64; }
+  __device__ static bool special(uint64_t k) { return k == ~0ULL; }
+};
+
+// PW: predicate width (0 = none); K0W/K1W: key widths (0 = absent); NC distinct
+// 8-byte value columns (int64, or fp64 when F64); OPS: vop(...) per value.
+template <int PW, bool PF64, int K0W, int K1W, int NC_, bool F64, uint32_t... OPS>
+struct StaticShape {
+  static constexpr bool kStatic = true;
+  static constexpr int NC = NC_;
+  static constexpr int KBITS = 8 * (K0W + K1W);
+  using Key = typename std::conditional<(KBITS > 0 && KBITS <= 32), uint32_t, uint64_t>::type;
+  static constexpr int NVS = sizeof...(OPS);
+  __host__ __device__ static constexpr uint32_t op(int v) {
+    const uint32_t a[NVS] = {OPS...};
+    return a[v];
+  }
+  __host__ __device__ static constexpr int np(const Plan&) { return PW ? 1 : 0; }
+  __host__ __device__ static constexpr int pw(const Plan&, int) { return PW; }
+  __host__ __device__ static constexpr bool pf64(const Plan&, int) { return PF64; }
+  __host__ __device__ static constexpr int nk(const Plan&) { return (K0W > 0) + (K1W > 0); }
+  __host__ __device__ static constexpr int kw(const Plan&, int i) { return i == 0 ? K0W : K1W; }
+  __host__ __device__ static constexpr int nv(const Plan&) { return NVS; }
+  __host__ __device__ static constexpr int kind(const Plan&, int v) { return (int)(op(v) & 3); }
+  __host__ __device__ static constexpr int ia(int v) { return (int)((op(v) >> 2) & 7); }
+  __host__ __device__ static constexpr int ib(int v) { return (int)((op(v) >> 5) & 7); }
+  __host__ __device__ static constexpr int ic(int v) { return (int)((op(v) >> 8) & 7); }
+  __host__ __device__ static constexpr bool fsum(const Plan&, int v) { return (op(v) >> 11) & VF_SUM; }
+  __host__ __device__ static constexpr bool fmn(const Plan&, int v) { return (op(v) >> 11) & VF_MIN; }
+  __host__ __device__ static constexpr bool fmx(const Plan&, int v) { return (op(v) >> 11) & VF_MAX; }
+  __host__ __device__ static constexpr bool vf64(const Plan&, int) { return F64; }
+  __device__ static bool special(Key k) {
+    if constexpr (KBITS > 0 && KBITS < 32) return false;        // narrow keys can never be ~0
+    else return k == (Key)~0ULL;
+  }
+};
+
+// ------------------------------------------------------------------ row evaluation
+template <class Sh, int NV, bool F64>
+struct Row {
+  bool q, fast;
+  typename Sh::Key key;
   int64_t vi[F64 ? 1 : NV];
   double vd[F64 ? NV : 1];
 };
 
-// Evaluate values of one row from raw operands (vector path: loaded as pairs).
-template <int NV, bool F64>
-__device__ __forceinline__ void eval_values_pair(const Plan& p, int64_t r, RowIn<NV, F64>& x0, RowIn<NV, F64>& x1) {
+template <int W>
+__device__ __forceinline__ void ld2c(const void* base, int64_t r, uint64_t& x0, uint64_t& x1) {
+  if constexpr (W == 1) {
+    uint32_t v = __ldg((const unsigned short*)((const uint8_t*)base + r));
+    x0 = v & 0xFF;
+    x1 = v >> 8;
+  } else if constexpr (W == 4) {
+    int2 v = __ldg((const int2*)((const int32_t*)base + r));
+    x0 = (uint64_t)(int64_t)v.x;
+    x1 = (uint64_t)(int64_t)v.y;
+  } else {
+    longlong2 v = __ldg((const longlong2*)((const long long*)base + r));
+    x0 = (uint64_t)v.x;
+    x1 = (uint64_t)v.y;
+  }
+}
+
+// 2-row load with a width that is a compile-time constant for static shapes.
+__device__ __forceinline__ void ld2w(int w, const void* base, int64_t r, uint64_t& x0, uint64_t& x1) {
+  if (w == 1) ld2c<1>(base, r, x0, x1);
+  else if (w == 4) ld2c<4>(base, r, x0, x1);
+  else ld2c<8>(base, r, x0, x1);
+}
+__device__ __forceinline__ uint64_t ld1w(int w, const void* base, int64_t r) {
+  if (w == 1) return __ldg((const uint8_t*)base + r);
+  if (w == 4) return (uint64_t)(int64_t)__ldg((const int32_t*)base + r);
+  return (uint64_t)__ldg((const long long*)base + r);
+}
+
+__device__ __forceinline__ int64_t mul_wide_s32(int32_t a, int32_t b) {
+  int64_t r;
+  asm("mul.wide.s32 %0, %1, %2;" : "=l"(r) : "r"(a), "r"(b));
+  return r;
+}
+
+template <class Sh>
+__device__ __forceinline__ bool pred_ok(const Plan& p, int i, uint64_t raw) {
+  const DevPred& d = p.preds[i];
+  bool ok;
+  if (Sh::pf64(p, i)) {
+    const double x = __longlong_as_double((long long)raw);
+    ok = x >= d.flo && x <= d.fhi;
+  } else if (Sh::pw(p, i) < 8) {
+    const int32_t x = (int32_t)(uint32_t)raw;                // u8 / i32: 32-bit compare on clamped bounds
+    ok = x >= d.lo32 && x <= d.hi32;
+  } else {
+    const int64_t x = (int64_t)raw;
+    ok = x >= d.lo && x <= d.hi;
+  }
+  return ok != (bool)d.anti;
+}
+
+// Value v of one row from its raw operands.  Integer fast path: COL values that fit
+// int32 (accumulated in 64 bits), products of int32 factors via mul.wide.s32 (exact
+// in int64); anything else clears `fast` (the row takes the exact int128 path).
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void value_of(const Plan& p, int v, uint64_t ra, uint64_t rb, uint64_t rc,
+                                         Row<Sh, NV, F64>& x) {
+  const DevValue& d = p.vals[v];
+  const int kind = Sh::kind(p, v);
+  if constexpr (F64) {
+    const double a = __longlong_as_double((long long)ra);
+    if (kind == OCL_EXPR_COL) {
+      x.vd[v] = a;
+    } else {
+      double e = __dmul_rn(a, __dsub_rn(d.Sf, __longlong_as_double((long long)rb)));
+      if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) e = __dmul_rn(e, __dadd_rn(d.Sf, __longlong_as_double((long long)rc)));
+      x.vd[v] = e;
+    }
+  } else {
+    const int64_t a = (int64_t)ra;
+    if (kind == OCL_EXPR_COL) {
+      x.fast = x.fast && fits_i32(a);
+      x.vi[v] = a;
+    } else {
+      const int64_t t = (int64_t)((uint64_t)d.S - rb);
+      x.fast = x.fast && fits_i32(a) && fits_i32(t);
+      int64_t e = mul_wide_s32((int32_t)a, (int32_t)t);
+      if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) {
+        const int64_t u = (int64_t)((uint64_t)d.S + rc);
+        x.fast = x.fast && fits_i32(e) && fits_i32(u);
+        e = mul_wide_s32((int32_t)e, (int32_t)u);
+      }
+      x.vi[v] = e;
+    }
+  }
+}
+
+template <class Sh>
+__device__ __forceinline__ typename Sh::Key pack_key(const Plan& p, const uint64_t* raw) {
+  typename Sh::Key k = 0;
 #pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (!F64) {
-      if (d.is_f64) {   // mixed int/fp64 plan: fp64 values take the exact slow path
+  for (int i = 0; i < kMaxKeys; ++i) {
+    if (i >= Sh::nk(p)) break;
+    k |= (typename Sh::Key)((raw[i] & p.keys[i].mask) << p.keys[i].shift);
+  }
+  return k;
+}
+
+// Both rows of a lane's 64-row unit (vector loads; full tiles only).
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void eval_pair(const Plan& p, int64_t r, Row<Sh, NV, F64>& x0, Row<Sh, NV, F64>& x1) {
+  x0.q = x1.q = true;
+  x0.fast = x1.fast = true;
+#pragma unroll
+  for (int i = 0; i < kMaxPreds; ++i) {
+    if (i >= Sh::np(p)) break;
+    uint64_t u0, u1;
+    ld2w(Sh::pw(p, i), p.preds[i].col.ptr, r, u0, u1);
+    x0.q = x0.q && pred_ok<Sh>(p, i, u0);
+    x1.q = x1.q && pred_ok<Sh>(p, i, u1);
+  }
+  uint64_t k0[kMaxKeys] = {0, 0}, k1[kMaxKeys] = {0, 0};
+#pragma unroll
+  for (int i = 0; i < kMaxKeys; ++i) {
+    if (i >= Sh::nk(p)) break;
+    ld2w(Sh::kw(p, i), p.keys[i].col.ptr, r, k0[i], k1[i]);
+  }
+  x0.key = pack_key<Sh>(p, k0);
+  x1.key = pack_key<Sh>(p, k1);
+  if constexpr (Sh::kStatic) {
+    uint64_t c0[Sh::NC], c1[Sh::NC];      // every distinct value column loaded once
+#pragma unroll
+    for (int i = 0; i < Sh::NC; ++i) ld2c<8>(p.vcols[i].ptr, r, c0[i], c1[i]);
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      value_of<Sh, NV, F64>(p, v, c0[Sh::ia(v)], c0[Sh::ib(v)], c0[Sh::ic(v)], x0);
+      value_of<Sh, NV, F64>(p, v, c1[Sh::ia(v)], c1[Sh::ib(v)], c1[Sh::ic(v)], x1);
+    }
+  } else {
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if (v >= p.nvals) break;
+      const DevValue& d = p.vals[v];
+      if (!F64 && d.is_f64) {              // mixed int/fp64 plan: fp64 values take the exact slow path
         x0.fast = x1.fast = false;
         continue;
       }
-    }
-    uint64_t a0, a1, b0 = 0, b1 = 0, c0 = 0, c1 = 0;
-    load_pair(d.a, r, a0, a1);
-    if (d.expr >= OCL_EXPR_MUL_1MINUS) load_pair(d.b, r, b0, b1);
-    if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS) load_pair(d.c, r, c0, c1);
-    if constexpr (F64) {
-      x0.vd[v] = value_f64(d, a0, b0, c0);
-      x1.vd[v] = value_f64(d, a1, b1, c1);
-    } else {
-      x0.vi[v] = value_i64_fast(d, a0, b0, c0, x0.fast);
-      x1.vi[v] = value_i64_fast(d, a1, b1, c1, x1.fast);
+      uint64_t a0, a1, b0 = 0, b1 = 0, c0 = 0, c1 = 0;
+      ld2w(d.a.width, d.a.ptr, r, a0, a1);
+      if (d.expr >= OCL_EXPR_MUL_1MINUS) ld2w(d.b.width, d.b.ptr, r, b0, b1);
+      if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS) ld2w(d.c.width, d.c.ptr, r, c0, c1);
+      value_of<Sh, NV, F64>(p, v, a0, b0, c0, x0);
+      value_of<Sh, NV, F64>(p, v, a1, b1, c1, x1);
     }
   }
 }
 
-template <int NV, bool F64>
-__device__ __forceinline__ void eval_row_scalar(const Plan& p, int64_t r, RowIn<NV, F64>& x) {
+// One row with scalar loads (ragged tail, unaligned columns).
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F64>& x) {
   x.fast = true;
-  x.q = r < p.n && row_pred_scalar(p, r);
   x.key = 0;
+  x.q = r < p.n;
   if (!x.q) return;
-  x.key = row_key_scalar(p, r);
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (!F64) {
-      if (d.is_f64) {
-        x.fast = false;
-        continue;
-      }
-    }
-    uint64_t a = load_one(d.a, r);
-    uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? load_one(d.b, r) : 0;
-    uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? load_one(d.c, r) : 0;
-    if constexpr (F64) x.vd[v] = value_f64(d, a, b, c);
-    else x.vi[v] = value_i64_fast(d, a, b, c, x.fast);
-  }
-}
-
-template <int NV, bool F64>
-__device__ __forceinline__ void eval_pair_vec(const Plan& p, int64_t r, RowIn<NV, F64>& x0, RowIn<NV, F64>& x1) {
-  x0.q = true;
-  x1.q = true;
 #pragma unroll
   for (int i = 0; i < kMaxPreds; ++i) {
-    if (i >= p.npreds) break;
-    uint64_t u0, u1;
-    load_pair(p.preds[i].col, r, u0, u1);
-    x0.q = x0.q && eval_pred(p.preds[i], u0);
-    x1.q = x1.q && eval_pred(p.preds[i], u1);
+    if (i >= Sh::np(p)) break;
+    x.q = x.q && pred_ok<Sh>(p, i, ld1w(Sh::pw(p, i), p.preds[i].col.ptr, r));
   }
-  x0.key = 0;
-  x1.key = 0;
+  uint64_t k[kMaxKeys] = {0, 0};
 #pragma unroll
   for (int i = 0; i < kMaxKeys; ++i) {
-    if (i >= p.nkeys) break;
-    uint64_t u0, u1;
-    load_pair(p.keys[i].col, r, u0, u1);
-    x0.key |= (u0 & p.keys[i].mask) << p.keys[i].shift;
-    x1.key |= (u1 & p.keys[i].mask) << p.keys[i].shift;
+    if (i >= Sh::nk(p)) break;
+    k[i] = ld1w(Sh::kw(p, i), p.keys[i].col.ptr, r);
   }
-  x0.fast = true;
-  x1.fast = true;
-  eval_values_pair<NV, F64>(p, r, x0, x1);
+  x.key = pack_key<Sh>(p, k);
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= Sh::nv(p)) break;
+    const DevValue& d = p.vals[v];
+    if (!F64 && d.is_f64) {
+      x.fast = false;
+      continue;
+    }
+    const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
+    const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
+    const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
+    value_of<Sh, NV, F64>(p, v, a, b, c, x);
+  }
 }
 
-// ------------------------------------------------------------------ register (private accumulator) tier
-// Few groups: each thread owns one accumulator record per group slot in shared
-// memory, laid out [slot][field][thread] (field offsets from the host planner,
-// Plan::priv_rec bytes per thread per slot): count u32; per value: SUM as 96-bit
-// (u64 lo + u32 hi) or double; MIN / MAX as order-preserving u64 encodings (zero
-// = identity).  A row costs one slot-indexed read-modify-write per accumulator:
-// no atomics in the row loop — the limit of the paper's "multiple accumulators
-// per group" in local memory.  A block-wide slot directory in shared
-// memory gives every thread the same key -> slot map.
-constexpr int kRegSlots = 4;
-
-template <int NV, bool F64>
-__device__ __forceinline__ void privg_add(const Plan& p, uint8_t* sm, int slot, int tid, const RowIn<NV, F64>& x) {
+// ------------------------------------------------------------------ 1. private slots
+// Record per thread per slot (offsets from the planner, Plan::priv_rec bytes):
+// count u32; per value: SUM of a COL value as i64 (fast path: int32 values), SUM of a
+// product as 96-bit (u64 lo + u32 hi), fp64 SUM as double; MIN / MAX as u64 order-
+// preserving encodings (0 = identity).  Layout [slot][field][thread].
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void priv_add(const Plan& p, uint8_t* sm, int slot, int tid, const Row<Sh, NV, F64>& x) {
   constexpr int T = kFusedThreads;
   uint8_t* base = sm + (size_t)slot * p.priv_rec * T;
   ((uint32_t*)base)[tid] += 1u;
 #pragma unroll
   for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
+    if (v >= Sh::nv(p)) break;
     const DevValue& d = p.vals[v];
     if constexpr (F64) {
       const double val = x.vd[v];
-      if (d.po_sum >= 0) ((double*)(base + d.po_sum * T))[tid] += val;
-      if (d.po_min >= 0) {
+      if (Sh::fsum(p, v)) ((double*)(base + d.po_sum * T))[tid] += val;
+      if (Sh::fmn(p, v)) {
         uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
         *m = max(*m, enc_min_f(val));
       }
-      if (d.po_max >= 0) {
+      if (Sh::fmx(p, v)) {
         uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
         *m = max(*m, enc_max_f(val));
       }
     } else {
-      if (d.is_f64) continue;                       // mixed plan: fp64 values went to the slow path
+      if (Sh::vf64(p, v)) continue;
       const int64_t val = x.vi[v];
-      if (d.po_sum >= 0) {
-        uint64_t* lo = (uint64_t*)(base + d.po_sum * T) + tid;
-        uint32_t* hi = (uint32_t*)(base + d.po_hi * T) + tid;
-        uint64_t l = *lo;
-        uint32_t h = *hi;
-        uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
-        asm("add.cc.u32 %0, %0, %3;\n\taddc.cc.u32 %1, %1, %4;\n\taddc.u32 %2, %2, %5;"
-            : "+r"(l0), "+r"(l1), "+r"(h)
-            : "r"((uint32_t)(uint64_t)val), "r"((uint32_t)((uint64_t)val >> 32)), "r"((uint32_t)(val >> 63)));
-        *lo = (uint64_t)l0 | ((uint64_t)l1 << 32);
-        *hi = h;
+      if (Sh::fsum(p, v)) {
+        if (Sh::kind(p, v) == OCL_EXPR_COL) {
+          ((int64_t*)(base + d.po_sum * T))[tid] += (int64_t)(int32_t)val;
+        } else {
+          uint64_t* lo = (uint64_t*)(base + d.po_sum * T) + tid;
+          uint32_t* hi = (uint32_t*)(base + d.po_hi * T) + tid;
+          uint64_t l = *lo;
+          uint32_t h = *hi;
+          uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
+          asm("add.cc.u32 %0, %0, %3;\n\taddc.cc.u32 %1, %1, %4;\n\taddc.u32 %2, %2, %5;"
+              : "+r"(l0), "+r"(l1), "+r"(h)
+              : "r"((uint32_t)(uint64_t)val), "r"((uint32_t)((uint64_t)val >> 32)), "r"((uint32_t)(val >> 63)));
+          *lo = (uint64_t)l0 | ((uint64_t)l1 << 32);
+          *hi = h;
+        }
       }
-      if (d.po_min >= 0) {
+      if (Sh::fmn(p, v)) {
         uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
         *m = max(*m, enc_min_i(val));
       }
-      if (d.po_max >= 0) {
+      if (Sh::fmx(p, v)) {
         uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
         *m = max(*m, enc_max_i(val));
       }
@@ -188,19 +351,14 @@ __device__ __forceinline__ void privg_add(const Plan& p, uint8_t* sm, int slot, 
   }
 }
 
-// Per-CTA shared-memory hash table (mid G: more distinct keys than private slots;
-// the paper's per-work-group local-memory aggregation tables).
-// sm_100 has no native 64-bit shared-memory atomic add/max (they lower to CAS
-// loops), so the table uses 32-bit fields and native 32-bit atomics only:
-//   [~key u64][count u32] per value: [sum of low 16 bits u32][sum of high 16 bits s32]
-//   [min u32][max u32] (order-preserving encodings, 0 = identity).
-// Values are int32 on this path (fast-path COL values), so each field absorbs 2^16
-// updates exactly; the CTA flushes the table into the HBM table every 2^16 rows.
-// Linear probing with 64-bit shared atomicCAS on the key, at most kSmemProbes probes.
+// ------------------------------------------------------------------ 2. CTA table
+// [~key u64][count u32] per value: [sum of low 16 bits u32][sum of high 16 bits s32]
+// [min u32][max u32] (order-preserving encodings, 0 = identity); int32 values only,
+// 2^16 updates per field between flushes.  64-bit CAS on the key, linear probing.
 constexpr int kSmemProbes = 16;
-constexpr int kCtaFlushRounds = 64;   // rounds of (warps x tile) rows = 64 x 8 x 128 = 65,536 rows
+constexpr int kCtaFlushRounds = 64;   // 64 rounds x 8 warps x 128 rows = 65,536 rows
 
-__device__ __forceinline__ uint8_t* smem_find_or_insert(uint8_t* tab, uint32_t cap, int32_t stride, uint64_t key) {
+__device__ __forceinline__ uint8_t* cta_find_or_insert(uint8_t* tab, uint32_t cap, int32_t stride, uint64_t key) {
   const uint64_t sk = ~key;
   uint32_t h = (uint32_t)fmix64(key) & (cap - 1);
   for (int probe = 0; probe < kSmemProbes; ++probe) {
@@ -219,21 +377,21 @@ __device__ __forceinline__ uint8_t* smem_find_or_insert(uint8_t* tab, uint32_t c
 __device__ __forceinline__ uint32_t enc32_max(int32_t v) { return (uint32_t)v ^ 0x80000000u; }
 __device__ __forceinline__ uint32_t enc32_min(int32_t v) { return ~enc32_max(v); }
 
-template <int NV, bool F64>
-__device__ __forceinline__ void cta_add(const Plan& p, uint8_t* e, const RowIn<NV, F64>& x) {
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void cta_add(const Plan& p, uint8_t* e, const Row<Sh, NV, F64>& x) {
   atomicAdd((unsigned int*)(e + 8), 1u);
   if constexpr (!F64) {
 #pragma unroll
     for (int v = 0; v < NV; ++v) {
-      if (v >= p.nvals) break;
+      if (v >= Sh::nv(p)) break;
       const DevValue& d = p.vals[v];
       const int32_t w = (int32_t)x.vi[v];
-      if (d.co_lo >= 0) {
+      if (Sh::fsum(p, v)) {
         atomicAdd((unsigned int*)(e + d.co_lo), (unsigned int)w & 0xFFFFu);
         atomicAdd((int*)(e + d.co_hi), w >> 16);
       }
-      if (d.co_min >= 0) atomicMax((unsigned int*)(e + d.co_min), enc32_min(w));
-      if (d.co_max >= 0) atomicMax((unsigned int*)(e + d.co_max), enc32_max(w));
+      if (Sh::fmn(p, v)) atomicMax((unsigned int*)(e + d.co_min), enc32_min(w));
+      if (Sh::fmx(p, v)) atomicMax((unsigned int*)(e + d.co_max), enc32_max(w));
     }
   }
 }
@@ -249,7 +407,8 @@ __device__ __forceinline__ void cta_flush_entry(const Plan& p, uint8_t* ce) {
     for (int v = 0; v < p.nvals; ++v) {
       const DevValue& d = p.vals[v];
       if (d.co_lo >= 0) {
-        const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
+        const int64_t sum =
+            (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
         atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)sum, (uint64_t)(sum >> 63));
       }
       if (d.co_min >= 0) {
@@ -265,36 +424,16 @@ __device__ __forceinline__ void cta_flush_entry(const Plan& p, uint8_t* ce) {
   for (int w = 8; w < p.cta_stride; w += 4) *(uint32_t*)(ce + w) = 0;
 }
 
-// Merge a whole entry (shared-memory table or CTA block entry) into the HBM table.
-__device__ __forceinline__ void entry_merge_global(const Plan& p, uint64_t key, const uint8_t* src) {
-  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
-  if (!e) return;
-  atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(src + 8));
-  for (int v = 0; v < p.nvals; ++v) {
-    const DevValue& d = p.vals[v];
-    if (d.off_sum >= 0) {
-      if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(src + d.off_sum));
-      else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(src + d.off_sum),
-                           *(const uint64_t*)(src + d.off_sum + 8));
-    }
-    if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(src + d.off_min));
-    if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(src + d.off_max));
-  }
-}
-
-// Per-warp staging of rows that miss the private slots: the warp groups them by key
-// (__match_any_sync) and one leader per distinct key applies the group's combined
-// contribution to the HBM table — hot keys of skewed (Zipf) inputs and runs of
-// clustered keys cost one atomic update per warp instead of one per row.
+// ------------------------------------------------------------------ 3. HBM table (warp-aggregated)
 template <int NV, bool F64>
 struct MissStage {
   int64_t vi[F64 ? 1 : NV][32];
   double vd[F64 ? NV : 1][32];
 };
 
-template <int NV, bool F64>
-__device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F64>& st, bool miss, const RowIn<NV, F64>& x,
-                                                 int lane) {
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F64>& st, bool miss,
+                                                 const Row<Sh, NV, F64>& x, int lane) {
   const unsigned mmask = __ballot_sync(0xffffffffu, miss);
   if (mmask == 0) return;
   if (miss) {
@@ -306,14 +445,14 @@ __device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F6
   }
   __syncwarp();
   if (miss) {
-    const unsigned peers = __match_any_sync(mmask, x.key);
+    const unsigned peers = __match_any_sync(mmask, (unsigned long long)x.key);
     if (lane == __ffs(peers) - 1) {
-      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x.key, p.status);
       if (e) {
         atomicAdd((unsigned long long*)(e + 8), (unsigned long long)__popc(peers));
 #pragma unroll
         for (int v = 0; v < NV; ++v) {
-          if (v >= p.nvals) break;
+          if (v >= Sh::nv(p)) break;
           const DevValue& d = p.vals[v];
           if constexpr (F64) {
             double sum = 0.0, mn = x.vd[v], mx = x.vd[v];
@@ -323,11 +462,11 @@ __device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F6
               mn = fmin(mn, y);
               mx = fmax(mx, y);
             }
-            if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), sum);
-            if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mn));
-            if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mx));
+            if (Sh::fsum(p, v)) atomicAdd((double*)(e + d.off_sum), sum);
+            if (Sh::fmn(p, v)) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mn));
+            if (Sh::fmx(p, v)) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mx));
           } else {
-            if (d.is_f64) continue;
+            if (Sh::vf64(p, v)) continue;
             I128 sum{0, 0};
             int64_t mn = x.vi[v], mx = x.vi[v];
             for (unsigned b = peers; b; b &= b - 1) {
@@ -336,9 +475,9 @@ __device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F6
               mn = min(mn, y);
               mx = max(mx, y);
             }
-            if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), sum.lo, sum.hi);
-            if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
-            if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
+            if (Sh::fsum(p, v)) atomic_add_i128((uint64_t*)(e + d.off_sum), sum.lo, sum.hi);
+            if (Sh::fmn(p, v)) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
+            if (Sh::fmx(p, v)) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
           }
         }
       }
@@ -347,50 +486,58 @@ __device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F6
   __syncwarp();
 }
 
-template <int NV, bool F64>
-__device__ __forceinline__ void privg_row(const Plan& p, uint64_t* dir, uint64_t (&rk)[kRegSlots], uint8_t* sm, int tid,
-                                          MissStage<NV, F64>& stage, const RowIn<NV, F64>& x, int64_t r) {
+// ------------------------------------------------------------------ per-row dispatch
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename Sh::Key (&rk)[kRegSlots],
+                                          uint8_t* sm, uint8_t* cta_tab, int tid, MissStage<NV, F64>& stage,
+                                          const Row<Sh, NV, F64>& x, int64_t r) {
+  using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
   int slot = -1;
 #pragma unroll
   for (int s = L - 1; s >= 0; --s)
     if (x.key == rk[s]) slot = s;
-  const bool special = x.key == ~0ULL;
+  const bool special = Sh::special(x.key);
   bool go = x.q && x.fast && slot >= 0 && !special;
   bool miss = false;
   if (x.q && !go) {                       // new key in this CTA, a slow value, or more keys than slots
-    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, x.key) : -1;
+    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, (uint64_t)x.key) : -1;
     if (slot >= 0) {
 #pragma unroll
-      for (int s = 0; s < L; ++s) rk[s] = ~*(volatile uint64_t*)&dir[s];
+      for (int s = 0; s < L; ++s) {
+        const uint64_t sk = *(volatile uint64_t*)&dir[s];
+        rk[s] = sk ? (Key)~sk : (Key)~0ULL;
+      }
       go = true;
     } else {
       uint8_t* e = nullptr;
-      if (p.smem_cap && x.fast && !special)     // mid G: CTA shared-memory table
-        e = smem_find_or_insert(sm + (size_t)kRegSlots * p.priv_rec * kFusedThreads, (uint32_t)p.smem_cap,
-                                p.cta_stride, x.key);
+      if (p.smem_cap && x.fast && !special) e = cta_find_or_insert(cta_tab, (uint32_t)p.smem_cap, p.cta_stride, x.key);
       if (e) {
-        cta_add<NV, F64>(p, e, x);
+        cta_add<Sh, NV, F64>(p, e, x);
       } else if (x.fast && !special) {
-        miss = true;                            // warp-aggregated HBM update below
+        miss = true;                      // warp-aggregated HBM update below
       } else {
-        e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+        e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x.key, p.status);
         if (e) update_entry_slow(p, e, r);
       }
     }
   }
-  if (go) privg_add<NV, F64>(p, sm, slot, tid, x);
-  warp_miss_update<NV, F64>(p, stage, miss, x, tid & 31);
+  if (go) priv_add<Sh, NV, F64>(p, sm, slot, tid, x);
+  warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);
 }
 
-template <int NV, bool F64, int U>
-__global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant__ Plan p) {
+// ------------------------------------------------------------------ the kernel
+template <class Sh, int NV, bool F64>
+__global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ Plan p) {
+  using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
   constexpr int T = kFusedThreads;
   extern __shared__ __align__(16) uint8_t sm[];
   __shared__ uint64_t dir[L];
-  __shared__ __align__(16) uint64_t blk[L * 32];   // block accumulators, entry layout (stride <= 256 B)
+  __shared__ __align__(16) uint64_t blk[L * 32];   // CTA-level entry per slot (stride <= 256 B)
+  __shared__ MissStage<NV, F64> stages[T / 32];
   const int tid = threadIdx.x, lane = tid & 31;
+  uint8_t* cta_tab = sm + (size_t)L * p.priv_rec * T;
   {
     uint4* z = (uint4*)sm;
     const int n16 = (int)(((size_t)L * p.priv_rec * T + (size_t)p.smem_cap * p.cta_stride) / 16);
@@ -399,21 +546,18 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
   for (int i = tid; i < L * 32; i += T) blk[i] = 0;
   if (tid < L) dir[tid] = 0;
   __syncthreads();
-  uint64_t rk[L];
+  Key rk[L];
 #pragma unroll
-  for (int s = 0; s < L; ++s) rk[s] = ~0ULL;   // ~0 never matches a slot (special key)
-  __shared__ MissStage<NV, F64> stages[kFusedThreads / 32];
+  for (int s = 0; s < L; ++s) rk[s] = (Key)~0ULL;   // never matches an admissible key
   MissStage<NV, F64>& stage = stages[tid >> 5];
 
-  constexpr int kTile = 64 * U;
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
-  const int64_t ntiles = (p.n + kTile - 1) / kTile;
-  // CTA-uniform round count (warp 0 of the CTA has the most tiles) so the whole CTA
-  // can meet at the periodic CTA-table flushes
+  const int64_t ntiles = (p.n + kTileRows - 1) / kTileRows;
+  // CTA-uniform round count (the CTA's first warp has the most tiles): the whole CTA
+  // meets at the periodic CTA-table flushes
   const int64_t first = (int64_t)blockIdx.x * (T / 32);
   const int64_t rounds = ntiles > first ? (ntiles - first + nwarps - 1) / nwarps : 0;
-  uint8_t* cta_tab = sm + (size_t)L * p.priv_rec * T;
   for (int64_t round = 0; round < rounds; ++round) {
     if (p.smem_cap && round > 0 && round % kCtaFlushRounds == 0) {
       __syncthreads();
@@ -422,32 +566,39 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
     }
     const int64_t t = warp + round * nwarps;
     if (t >= ntiles) continue;
-    const int64_t base = t * kTile;
-    const bool vec = p.vec_ok && base + kTile <= p.n;
+    const int64_t base = t * kTileRows;
+    if (p.vec_ok && base + kTileRows <= p.n) {
+      Row<Sh, NV, F64> x[kUnits][2];
 #pragma unroll
-    for (int u = 0; u < U; ++u) {
-      const int64_t r = base + 64 * u + 2 * lane;
-      RowIn<NV, F64> x0, x1;
-      if (vec) {
-        eval_pair_vec<NV, F64>(p, r, x0, x1);
-      } else {
-        eval_row_scalar<NV, F64>(p, r, x0);
-        eval_row_scalar<NV, F64>(p, r + 1, x1);
+      for (int u = 0; u < kUnits; ++u) eval_pair<Sh, NV, F64>(p, base + 64 * u + 2 * lane, x[u][0], x[u][1]);
+#pragma unroll
+      for (int u = 0; u < kUnits; ++u) {
+        const int64_t r = base + 64 * u + 2 * lane;
+        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x[u][0].q, x[u][1].q);
+        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][0], r);
+        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][1], r + 1);
       }
-      if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-      privg_row<NV, F64>(p, dir, rk, sm, tid, stage, x0, r);
-      privg_row<NV, F64>(p, dir, rk, sm, tid, stage, x1, r + 1);
+    } else {
+      for (int u = 0; u < kUnits; ++u) {
+        const int64_t r = base + 64 * u + 2 * lane;
+        Row<Sh, NV, F64> x0, x1;
+        eval_one<Sh, NV, F64>(p, r, x0);
+        eval_one<Sh, NV, F64>(p, r + 1, x1);
+        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+      }
     }
   }
 
-  // ---- flush: warp reduce of the private records -> shared block entry -> one global update per slot
+  // ---- flush: warp-reduce the private records -> CTA entry per slot -> HBM table
   __syncthreads();
   uint8_t* blkb = (uint8_t*)blk;
   for (int s = 0; s < L; ++s) {
-    if (dir[s] == 0) continue;                       // uniform: slot never used in this block
+    if (dir[s] == 0) continue;                       // uniform: slot never used in this CTA
     uint8_t* be = blkb + s * 256;
     const uint8_t* rec = sm + (size_t)s * p.priv_rec * T;
-    uint32_t c = __reduce_add_sync(0xffffffffu, ((const uint32_t*)rec)[tid]);
+    const uint32_t c = __reduce_add_sync(0xffffffffu, ((const uint32_t*)rec)[tid]);
     if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)c);
     for (int v = 0; v < p.nvals; ++v) {
       const DevValue& d = p.vals[v];
@@ -459,7 +610,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
         } else {
           I128 x;
           x.lo = ((const uint64_t*)(rec + d.po_sum * T))[tid];
-          x.hi = (uint64_t)(int64_t)(int32_t)((const uint32_t*)(rec + d.po_hi * T))[tid];
+          x.hi = d.po_hi >= 0 ? (uint64_t)(int64_t)(int32_t)((const uint32_t*)(rec + d.po_hi * T))[tid]
+                              : (uint64_t)((int64_t)x.lo >> 63);
           x = warp_sum_i128(x);
           if (lane == 0) atomic_add_i128((uint64_t*)(be + d.off_sum), x.lo, x.hi);
         }
@@ -477,228 +629,235 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga_reg(const __grid_constant
     }
   }
   __syncthreads();
-  // one thread per slot pushes the block entry into the global table
   if (tid < L) {
     const uint64_t sk = dir[tid];
-    if (sk != 0) entry_merge_global(p, ~sk, blkb + tid * 256);
+    if (sk != 0) {
+      const uint8_t* src = blkb + tid * 256;
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
+      if (e) {
+        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(src + 8));
+        for (int v = 0; v < p.nvals; ++v) {
+          const DevValue& d = p.vals[v];
+          if (d.off_sum >= 0) {
+            if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(src + d.off_sum));
+            else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(src + d.off_sum),
+                                 *(const uint64_t*)(src + d.off_sum + 8));
+          }
+          if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(src + d.off_min));
+          if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(src + d.off_max));
+        }
+      }
+    }
   }
-  // the CTA's shared-memory table (mid-G): one thread per occupied entry
   if (p.smem_cap)
     for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
 }
 
-// ------------------------------------------------------------------ global tier
+// ------------------------------------------------------------------ HBM-only tier (tier 2)
+// Lanes own consecutive rows; runs of equal keys are folded by a segmented shuffle
+// reduction into their first lane, which alone touches the table.
 template <int NV, bool F64>
-__device__ __forceinline__ void glb_row(const Plan& p, const RowIn<NV, F64>& x, int64_t r) {
-  if (!x.q) return;
-  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
-  if (!e) return;
-  if (!x.fast) {
-    update_entry_slow(p, e, r);
-    return;
-  }
-  atomicAdd((unsigned long long*)(e + 8), 1ULL);
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (F64) {
-      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), x.vd[v]);
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(x.vd[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(x.vd[v]));
-    } else {
-      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)x.vi[v], (uint64_t)(x.vi[v] >> 63));
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(x.vi[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(x.vi[v]));
+__global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant__ Plan p) {
+  using Sh = DynShape;
+  const int lane = threadIdx.x & 31;
+  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
+  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
+  const int64_t nunits = (p.n + 31) / 32;
+  for (int64_t t = warp; t < nunits; t += nwarps) {
+    const int64_t r = t * 32 + lane;
+    Row<Sh, NV, F64> x;
+    eval_one<Sh, NV, F64>(p, r, x);
+    if (p.bitmap_out) {
+      const uint32_t w = __ballot_sync(0xffffffffu, x.q);
+      if (lane == 0) p.bitmap_out[t] = w;
     }
-  }
-}
-
-// Warp-level run combining before the HBM atomics (many-groups tier).  Lanes own
-// consecutive rows, so runs of equal keys (clustered inputs such as lineitem
-// ordered by orderkey, or hot keys) are contiguous lane ranges: one segmented
-// shuffle reduction folds each run into its first lane, which alone touches the
-// table.  Rows that are not eligible (slow values, the key ~0) take the per-row path.
-template <int NV, bool F64>
-__device__ __forceinline__ void glb_unit(const Plan& p, const RowIn<NV, F64>& x, int64_t r, int lane) {
-  const bool ok = x.q && x.fast && x.key != ~0ULL;
-  const unsigned okmask = __ballot_sync(0xffffffffu, ok);
-  const uint64_t kprev = __shfl_up_sync(0xffffffffu, x.key, 1);
-  const bool cont = ok && lane > 0 && ((okmask >> (lane - 1)) & 1u) && kprev == x.key;
-  const unsigned contmask = __ballot_sync(0xffffffffu, cont);
-  if (contmask == 0) {                   // no run in this unit (shuffled / high-cardinality): per row
-    glb_row<NV, F64>(p, x, r);
-    return;
-  }
-  if (x.q && !ok) glb_row<NV, F64>(p, x, r);
-  const unsigned later = lane == 31 ? 0u : (~contmask & ~((2u << lane) - 1u));   // segment starts after me
-  const int seg_end = later ? __ffs(later) - 2 : 31;
-  uint32_t c = ok ? 1u : 0u;
-  I128 si[F64 ? 1 : NV];
-  double sd[F64 ? NV : 1], mnd[F64 ? NV : 1], mxd[F64 ? NV : 1];
-  int64_t mni[F64 ? 1 : NV], mxi[F64 ? 1 : NV];
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if constexpr (F64) {
-      sd[v] = ok ? x.vd[v] : 0.0;
-      mnd[v] = x.vd[v];
-      mxd[v] = x.vd[v];
-    } else {
-      si[v] = ok ? i128_from_i64(x.vi[v]) : I128{0, 0};
-      mni[v] = x.vi[v];
-      mxi[v] = x.vi[v];
+    const bool ok = x.q && x.fast && x.key != ~0ULL;
+    const unsigned okmask = __ballot_sync(0xffffffffu, ok);
+    const uint64_t kprev = __shfl_up_sync(0xffffffffu, x.key, 1);
+    const bool cont = ok && lane > 0 && ((okmask >> (lane - 1)) & 1u) && kprev == x.key;
+    const unsigned contmask = __ballot_sync(0xffffffffu, cont);
+    if (x.q && !ok) {                      // exact per-row path
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+      if (e) update_entry_slow(p, e, r);
     }
-  }
+    const unsigned later = lane == 31 ? 0u : (~contmask & ~((2u << lane) - 1u));
+    const int seg_end = later ? __ffs(later) - 2 : 31;
+    uint32_t c = ok ? 1u : 0u;
+    I128 si[F64 ? 1 : NV];
+    double sd[F64 ? NV : 1], mnd[F64 ? NV : 1], mxd[F64 ? NV : 1];
+    int64_t mni[F64 ? 1 : NV], mxi[F64 ? 1 : NV];
 #pragma unroll
-  for (int o = 1; o < 32; o <<= 1) {
-    const bool take = lane + o <= seg_end;
-    const uint32_t cy = __shfl_down_sync(0xffffffffu, c, o);   // every lane shuffles; `take` selects
-    if (take) c += cy;
+    for (int v = 0; v < NV; ++v) {
+      if constexpr (F64) {
+        sd[v] = ok ? x.vd[v] : 0.0;
+        mnd[v] = mxd[v] = x.vd[v];
+      } else {
+        si[v] = ok ? i128_from_i64(x.vi[v]) : I128{0, 0};
+        mni[v] = mxi[v] = x.vi[v];
+      }
+    }
+    if (contmask) {
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const bool take = lane + o <= seg_end;
+        const uint32_t cy = __shfl_down_sync(0xffffffffu, c, o);   // every lane shuffles; `take` selects
+        if (take) c += cy;
+#pragma unroll
+        for (int v = 0; v < NV; ++v) {
+          if (v >= p.nvals) break;
+          if constexpr (F64) {
+            const double y = __shfl_down_sync(0xffffffffu, sd[v], o);
+            const double a = __shfl_down_sync(0xffffffffu, mnd[v], o);
+            const double b = __shfl_down_sync(0xffffffffu, mxd[v], o);
+            if (take) {
+              sd[v] += y;
+              mnd[v] = fmin(mnd[v], a);
+              mxd[v] = fmax(mxd[v], b);
+            }
+          } else {
+            I128 y;
+            y.lo = __shfl_down_sync(0xffffffffu, si[v].lo, o);
+            y.hi = __shfl_down_sync(0xffffffffu, si[v].hi, o);
+            const int64_t a = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mni[v], o);
+            const int64_t b = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mxi[v], o);
+            if (take) {
+              si[v] = i128_add(si[v], y);
+              mni[v] = min(mni[v], a);
+              mxi[v] = max(mxi[v], b);
+            }
+          }
+        }
+      }
+    }
+    if (!ok || cont) continue;             // run heads only
+    uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
+    if (!e) continue;
+    atomicAdd((unsigned long long*)(e + 8), (unsigned long long)c);
 #pragma unroll
     for (int v = 0; v < NV; ++v) {
       if (v >= p.nvals) break;
       const DevValue& d = p.vals[v];
       if constexpr (F64) {
-        double y = __shfl_down_sync(0xffffffffu, sd[v], o);
-        if (take) sd[v] += y;
-        if (d.off_min >= 0) { double z = __shfl_down_sync(0xffffffffu, mnd[v], o); if (take) mnd[v] = fmin(mnd[v], z); }
-        if (d.off_max >= 0) { double z = __shfl_down_sync(0xffffffffu, mxd[v], o); if (take) mxd[v] = fmax(mxd[v], z); }
+        if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), sd[v]);
+        if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mnd[v]));
+        if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mxd[v]));
       } else {
-        if (d.off_sum >= 0) {
-          I128 y;
-          y.lo = __shfl_down_sync(0xffffffffu, si[v].lo, o);
-          y.hi = __shfl_down_sync(0xffffffffu, si[v].hi, o);
-          if (take) si[v] = i128_add(si[v], y);
-        }
-        if (d.off_min >= 0) {
-          int64_t z = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mni[v], o);
-          if (take) mni[v] = min(mni[v], z);
-        }
-        if (d.off_max >= 0) {
-          int64_t z = (int64_t)__shfl_down_sync(0xffffffffu, (long long)mxi[v], o);
-          if (take) mxi[v] = max(mxi[v], z);
-        }
+        if (d.is_f64) continue;
+        if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), si[v].lo, si[v].hi);
+        if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mni[v]));
+        if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mxi[v]));
       }
-    }
-  }
-  if (!ok || cont) return;                // run heads only
-  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, x.key, p.status);
-  if (!e) return;
-  atomicAdd((unsigned long long*)(e + 8), (unsigned long long)c);
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (F64) {
-      if (d.off_sum >= 0) atomicAdd((double*)(e + d.off_sum), sd[v]);
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mnd[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mxd[v]));
-    } else {
-      if (d.is_f64) continue;
-      if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), si[v].lo, si[v].hi);
-      if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mni[v]));
-      if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mxi[v]));
     }
   }
 }
 
-template <int NV, bool F64, int U>
-__global__ void __launch_bounds__(kFusedThreads) k_sga_glb(const __grid_constant__ Plan p) {
-  const int lane = threadIdx.x & 31;
-  constexpr int kTile = 32 * U;            // lane l owns rows base + 32u + l: consecutive rows across lanes
-  const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
-  const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
-  const int64_t ntiles = (p.n + kTile - 1) / kTile;
-  for (int64_t t = warp; t < ntiles; t += nwarps) {
-    const int64_t base = t * kTile;
-    RowIn<NV, F64> x[U];
-#pragma unroll
-    for (int u = 0; u < U; ++u) eval_row_scalar<NV, F64>(p, base + 32 * u + lane, x[u]);
-#pragma unroll
-    for (int u = 0; u < U; ++u) {
-      const int64_t r = base + 32 * u + lane;
-      if (p.bitmap_out) {
-        const uint32_t w = __ballot_sync(0xffffffffu, x[u].q);
-        const int64_t wi = r >> 5;
-        if (lane == 0 && wi < ((p.n + 31) >> 5)) p.bitmap_out[wi] = w;
-      }
-      glb_unit<NV, F64>(p, x[u], r, lane);
-    }
+// ------------------------------------------------------------------ static shapes (AOT instantiations)
+// TPC-H Q1: pred i32; keys u8, u8; columns qty, price, disc, tax;
+// values qty, price, price*(S-disc), price*(S-disc)*(S+tax), disc (SUMs).
+using ShQ1I = StaticShape<4, false, 1, 1, 4, false, vop(0, VF_SUM, 0), vop(0, VF_SUM, 1), vop(1, VF_SUM, 1, 2),
+                          vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
+using ShQ1F = StaticShape<4, false, 1, 1, 4, true, vop(0, VF_SUM, 0), vop(0, VF_SUM, 1), vop(1, VF_SUM, 1, 2),
+                          vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
+// GROUP BY an i64 key, COUNT/SUM/MIN/MAX of one i64 column (config C3), and the same
+// behind an i32 range predicate (config C5).
+using ShK64 = StaticShape<0, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+using ShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+
+template <class Sh>
+static bool shape_match(const Plan& g) {
+  if (g.npreds != Sh::np(g) || g.nkeys != Sh::nk(g) || g.nvals != Sh::nv(g)) return false;
+  for (int i = 0; i < g.npreds; ++i)
+    if (g.preds[i].col.width != Sh::pw(g, i) || (bool)g.preds[i].is_f64 != Sh::pf64(g, i)) return false;
+  for (int i = 0; i < g.nkeys; ++i)
+    if (g.keys[i].col.width != Sh::kw(g, i)) return false;
+  if (g.ncols != Sh::NC) return false;
+  for (int i = 0; i < g.ncols; ++i)
+    if (g.vcols[i].width != 8 || (g.vcols[i].dtype == OCL_F64) != Sh::vf64(g, 0)) return false;
+  for (int v = 0; v < g.nvals; ++v) {
+    const DevValue& d = g.vals[v];
+    if (d.expr != Sh::kind(g, v) || (bool)d.is_f64 != Sh::vf64(g, v)) return false;
+    if ((d.off_sum >= 0) != Sh::fsum(g, v) || (d.off_min >= 0) != Sh::fmn(g, v) ||
+        (d.off_max >= 0) != Sh::fmx(g, v))
+      return false;
+    if (d.ia != Sh::ia(v)) return false;
+    if (d.expr >= OCL_EXPR_MUL_1MINUS && d.ib != Sh::ib(v)) return false;
+    if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS && d.ic != Sh::ic(v)) return false;
   }
+  return true;
 }
 
 // ------------------------------------------------------------------ dispatch
-constexpr int kUnits = 2;
-constexpr int kGlbUnits = 4;
-
 static size_t reg_smem(const Plan& p) {
   return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.cta_stride;
 }
 
-template <int NV, bool F64>
-static cudaError_t launch_reg_nv(const Plan& p, int grid, cudaStream_t s) {
+template <class Sh, int NV, bool F64>
+static cudaError_t launch_k(const Plan& p, int sms, cudaStream_t s) {
   const size_t smem = reg_smem(p);
-  cudaError_t e = cudaFuncSetAttribute(k_sga_reg<NV, F64, kUnits>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                       (int)smem);
+  cudaError_t e = cudaFuncSetAttribute(k_sga<Sh, NV, F64>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, k_sga<Sh, NV, F64>, kFusedThreads, smem) != cudaSuccess ||
+      nb < 1)
+    nb = 1;
+  int64_t grid = (int64_t)sms * nb;
+  const int64_t need = ((p.n + kTileRows - 1) / kTileRows + (kFusedThreads / 32) - 1) / (kFusedThreads / 32);
+  if (need < grid) grid = need > 0 ? need : 1;
   count_launch();
-  k_sga_reg<NV, F64, kUnits><<<grid, kFusedThreads, smem, s>>>(p);
+  k_sga<Sh, NV, F64><<<(int)grid, kFusedThreads, smem, s>>>(p);
   return cudaGetLastError();
 }
 
 template <bool F64>
-static cudaError_t launch_reg_f(const Plan& p, int grid, cudaStream_t s) {
-  if (p.nvals <= 1) return launch_reg_nv<1, F64>(p, grid, s);
-  if (p.nvals <= 2) return launch_reg_nv<2, F64>(p, grid, s);
-  if (p.nvals <= 4) return launch_reg_nv<4, F64>(p, grid, s);
-  return launch_reg_nv<6, F64>(p, grid, s);
+static cudaError_t launch_dyn(const Plan& p, int sms, cudaStream_t s) {
+  if (p.nvals <= 1) return launch_k<DynShape, 1, F64>(p, sms, s);
+  if (p.nvals <= 2) return launch_k<DynShape, 2, F64>(p, sms, s);
+  if (p.nvals <= 4) return launch_k<DynShape, 4, F64>(p, sms, s);
+  return launch_k<DynShape, 6, F64>(p, sms, s);
 }
 
 template <bool F64>
-static cudaError_t launch_glb_f(const Plan& p, int grid, cudaStream_t s) {
+static cudaError_t launch_glb(const Plan& p, int sms, cudaStream_t s) {
+  int64_t grid = (int64_t)sms * 8;
+  const int64_t need = ((p.n + 31) / 32 + 7) / 8;
+  if (need < grid) grid = need > 0 ? need : 1;
   count_launch();
-  if (p.nvals <= 1) k_sga_glb<1, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else if (p.nvals <= 2) k_sga_glb<2, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else if (p.nvals <= 4) k_sga_glb<4, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
-  else k_sga_glb<6, F64, kGlbUnits><<<grid, kFusedThreads, 0, s>>>(p);
+  if (p.nvals <= 1) k_sga_glb<1, F64><<<(int)grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 2) k_sga_glb<2, F64><<<(int)grid, kFusedThreads, 0, s>>>(p);
+  else if (p.nvals <= 4) k_sga_glb<4, F64><<<(int)grid, kFusedThreads, 0, s>>>(p);
+  else k_sga_glb<6, F64><<<(int)grid, kFusedThreads, 0, s>>>(p);
   return cudaGetLastError();
 }
 
 int reg_tier_slots() { return kRegSlots; }
 
-template <int NV, bool F64>
-static const void* reg_kernel_ptr() { return (const void*)k_sga_reg<NV, F64, kUnits>; }
-template <int NV, bool F64>
-static const void* glb_kernel_ptr() { return (const void*)k_sga_glb<NV, F64, kGlbUnits>; }
-
-// Resident CTAs per SM of the instantiation launch_fused would pick (persistent grid sizing).
-int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64) {
-  const int nv = p.nvals <= 1 ? 1 : (p.nvals <= 2 ? 2 : (p.nvals <= 4 ? 4 : 6));
-  const void* fn;
-  if (reg_tier) {
-    if (values_f64) fn = nv == 1 ? reg_kernel_ptr<1, true>() : nv == 2 ? reg_kernel_ptr<2, true>() : nv == 4 ? reg_kernel_ptr<4, true>() : reg_kernel_ptr<6, true>();
-    else fn = nv == 1 ? reg_kernel_ptr<1, false>() : nv == 2 ? reg_kernel_ptr<2, false>() : nv == 4 ? reg_kernel_ptr<4, false>() : reg_kernel_ptr<6, false>();
-    cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)reg_smem(p));
-  } else {
-    if (values_f64) fn = nv == 1 ? glb_kernel_ptr<1, true>() : nv == 2 ? glb_kernel_ptr<2, true>() : nv == 4 ? glb_kernel_ptr<4, true>() : glb_kernel_ptr<6, true>();
-    else fn = nv == 1 ? glb_kernel_ptr<1, false>() : nv == 2 ? glb_kernel_ptr<2, false>() : nv == 4 ? glb_kernel_ptr<4, false>() : glb_kernel_ptr<6, false>();
-  }
-  int nb = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, reg_tier ? reg_smem(p) : 0) != cudaSuccess ||
-      nb < 1)
-    nb = 1;
-  return nb;
-}
-
-// values_f64: all value expressions are fp64 (mixed int/fp64 plans use the
-// integer kernels, whose slow path handles fp64 values exactly too).
-cudaError_t launch_fused(const Plan& p, bool reg_tier, bool values_f64, int grid, cudaStream_t s) {
+// mode 0: fused kernel (static shape if one matches); 1: fused kernel, DynShape only;
+// 2: HBM-only kernel.  values_f64: every value expression is fp64 (mixed plans use the
+// integer instantiation, whose exact slow path handles fp64 values).  *kind reports
+// the shape used (0 dynamic / HBM-only, 1.. static).
+cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind) {
+  *kind = 0;
   if (p.n == 0) return cudaSuccess;
-  int64_t tiles = (p.n + 64 * kUnits - 1) / (64 * kUnits);
-  int64_t g = (tiles + (kFusedThreads / 32) - 1) / (kFusedThreads / 32);
-  if (g > grid) g = grid;
-  if (reg_tier) return values_f64 ? launch_reg_f<true>(p, (int)g, s) : launch_reg_f<false>(p, (int)g, s);
-  return values_f64 ? launch_glb_f<true>(p, (int)g, s) : launch_glb_f<false>(p, (int)g, s);
+  if (mode == 2) return values_f64 ? launch_glb<true>(p, sms, s) : launch_glb<false>(p, sms, s);
+  if (mode == 0 && p.vec_ok) {
+    if (shape_match<ShQ1I>(p)) {
+      *kind = 1;
+      return launch_k<ShQ1I, 5, false>(p, sms, s);
+    }
+    if (shape_match<ShQ1F>(p)) {
+      *kind = 2;
+      return launch_k<ShQ1F, 5, true>(p, sms, s);
+    }
+    if (shape_match<ShK64>(p)) {
+      *kind = 3;
+      return launch_k<ShK64, 1, false>(p, sms, s);
+    }
+    if (shape_match<ShP32K64>(p)) {
+      *kind = 4;
+      return launch_k<ShP32K64, 1, false>(p, sms, s);
+    }
+  }
+  return values_f64 ? launch_dyn<true>(p, sms, s) : launch_dyn<false>(p, sms, s);
 }
 
 }  // namespace ocl

@@ -53,9 +53,8 @@ cudaError_t launch_merge_partials(const uint8_t* partials, int32_t nparts, int64
                                   int32_t* status, int grid, cudaStream_t s);
 cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
                                    int grid, cudaStream_t s);
-cudaError_t launch_fused(const Plan& p, bool reg_tier, bool values_f64, int grid, cudaStream_t s);
-int fused_blocks_per_sm(const Plan& p, bool reg_tier, bool values_f64);
+// Fused select -> group -> aggregate kernel (fused.cu).  mode 0: static shape if one
+// matches the plan, else dynamic; 1: dynamic shape only; 2: HBM-only kernel.
+cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind);
 int reg_tier_slots();
-// Plan-specialised register-tier kernels (fused_spec.cu); false if no signature matches.
-bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 }  // namespace ocl
