@@ -221,6 +221,17 @@ ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* agg
     if (need_max[v]) { rec = (int)align_up((size_t)rec, 8); d.po_max = rec; rec += 8; }
   }
   p.priv_rec = (int)align_up((size_t)rec, 8);
+  {   // CTA-table entry layout: [~key u64][count u32] per value [lo16 sum][hi16 sum][min][max]
+    int co = 12;
+    for (int v = 0; v < p.nvals; ++v) {
+      DevValue& d = p.vals[v];
+      d.co_lo = d.co_hi = d.co_min = d.co_max = -1;
+      if (d.off_sum >= 0) { d.co_lo = co; d.co_hi = co + 4; co += 8; }
+      if (d.off_min >= 0) { d.co_min = co; co += 4; }
+      if (d.off_max >= 0) { d.co_max = co; co += 4; }
+    }
+    p.cta_stride = (int)align_up((size_t)co, 8);
+  }
   // distinct operand columns (static shapes load each once) and per-value indices
   p.ncols = 0;
   auto col_index = [&](const DevCol& c) -> int {
@@ -363,17 +374,6 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   P->table_bytes = align_up((P->cap + 1) * (size_t)p.stride, 256);
   p.status = a->dev_status;
   p.bitmap_out = a->bitmap_out;
-  {   // CTA-table entry layout: [~key u64][count u32] per value [lo16 sum][hi16 sum][min][max]
-    int co = 12;
-    for (int v = 0; v < p.nvals; ++v) {
-      DevValue& d = p.vals[v];
-      d.co_lo = d.co_hi = d.co_min = d.co_max = -1;
-      if (d.off_sum >= 0) { d.co_lo = co; d.co_hi = co + 4; co += 8; }
-      if (d.off_min >= 0) { d.co_min = co; co += 4; }
-      if (d.off_max >= 0) { d.co_max = co; co += 4; }
-    }
-    p.cta_stride = (int)align_up((size_t)co, 8);
-  }
   p.smem_cap = plan_smem_cap(a, p);
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;
@@ -631,7 +631,9 @@ ocl_status ocl_group_aggregate(ocl_ctx* ctx, const int32_t* gids, const uint32_t
   p.n = max_rows;
   if (max_groups == 0) return OCL_OK;
   OCL_CUDA(cudaMemsetAsync(ws, 0, (size_t)max_groups * p.stride, st), "state init");
-  OCL_CUDA(launch_group_aggregate(p, max_rows, ngroups_dev, max_groups, ctx->grid, st), "group_aggregate launch");
+  p.direct = 1;
+  OCL_CUDA(launch_group_aggregate(p, max_rows, ngroups_dev, max_groups, P.values_f64, ctx->sms, st),
+           "group_aggregate launch");
   P.fin.out_capacity = max_groups;
   OCL_CUDA(launch_finalize_dense(p.table, p.stride, ngroups_dev, max_groups, P.fin, ctx->grid, st), "finalize");
   return OCL_OK;

@@ -1,112 +1,150 @@
 // aggregate.cu — K8: grouped aggregation over a dense group-id column (unfused chain).
 //
 // Paper (§4.1.7): work-groups on disjoint partitions build
-// intermediate aggregation tables with atomics in local memory; for few groups
-// each group is spread over several accumulators ("the number of accumulators
-// per group being chosen inversely proportional to the number of groups") to
-// cut same-address contention; tables that do not fit local memory fall back to
-// the same scheme in global memory.  Then one thread per group finalises.
+// intermediate aggregation tables with atomics in local memory; for few groups each
+// group is spread over several accumulators ("the number of accumulators per group
+// being chosen inversely proportional to the number of groups") to cut same-address
+// contention; tables that do not fit local memory fall back to the same scheme in
+// global memory.  Then one thread per group finalises (k_finalize_dense).
 //
-// B200 design: SMEM tier — R replicas of the G-entry state table in shared memory
-// (R = largest power of two <= 32 with R*G*stride <= the smem budget, lane picks
-// replica lane % R), shared-memory atomics (native 64-bit add / max, fp64 add),
-// then one flush of the CTA's non-empty entries into the HBM table.  GLOBAL tier
-// when G*stride exceeds shared memory: the same updates on the HBM table.
-// Values are read at row oids[j] (fused gather), integer expressions in int128.
-#include "launch.cuh"
-#include "rowops.cuh"
+// B200 design: the same three tiers as the fused kernel (sga_device.cuh), indexed by
+// the group id instead of a hashed key:
+//   PRIVATE  (G small): one accumulator record per group per thread in shared memory
+//            ([g][field][thread]) — the paper's multiple accumulators taken to one per
+//            thread: no atomics at all in the row loop;
+//   CTA      (G fits shared memory, integer COL values): a direct-indexed array of
+//            32-bit-field entries updated with native shared-memory atomics, flushed to
+//            HBM every 2^16 rows;
+//   HBM      otherwise: warp-aggregated (__match_any_sync on the gid) global atomics.
+// Values are read at row oids[j] (a fused gather).  Rows whose values need int128 go
+// through the exact per-row path.
+#include "sga_device.cuh"
 
 namespace ocl {
 
-__device__ __forceinline__ void agg_update_row(const Plan& p, uint8_t* e, int64_t r) {
-  atomicAdd((unsigned long long*)(e + 8), 1ULL);
-  for (int i = 0; i < p.nvals; ++i) {
-    const DevValue& v = p.vals[i];
-    uint64_t ra = load_one(v.a, r);
-    uint64_t rb = v.expr >= OCL_EXPR_MUL_1MINUS ? load_one(v.b, r) : 0;
-    uint64_t rc = v.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? load_one(v.c, r) : 0;
-    if (v.is_f64) {
-      double d = value_f64(v, ra, rb, rc);
-      if (v.off_sum >= 0) atomicAdd((double*)(e + v.off_sum), d);
-      if (v.off_min >= 0) atomicMax((unsigned long long*)(e + v.off_min), (unsigned long long)enc_min_f(d));
-      if (v.off_max >= 0) atomicMax((unsigned long long*)(e + v.off_max), (unsigned long long)enc_max_f(d));
-    } else {
-      bool fast = true;
-      int64_t x = value_i64_fast(v, ra, rb, rc, fast);
-      I128 y = fast ? i128_from_i64(x) : value_i128(v, ra, rb, rc);
-      if (v.off_sum >= 0) atomic_add_i128((uint64_t*)(e + v.off_sum), y.lo, y.hi);
-      if (v.off_min >= 0) atomicMax((unsigned long long*)(e + v.off_min), (unsigned long long)enc_min_i((int64_t)y.lo));
-      if (v.off_max >= 0) atomicMax((unsigned long long*)(e + v.off_max), (unsigned long long)enc_max_i((int64_t)y.lo));
+constexpr size_t kAggSmemBudget = 160 * 1024;
+enum AggMode { AGG_PRIV = 0, AGG_CTA = 1, AGG_HBM = 2 };
+
+template <int NV, bool F64>
+__device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<DynShape, NV, F64>& x) {
+  x.q = true;
+  x.fast = true;
+  x.key = (uint64_t)(uint32_t)g;
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= p.nvals) break;
+    const DevValue& d = p.vals[v];
+    if (!F64 && d.is_f64) {
+      x.fast = false;
+      continue;
     }
+    const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
+    const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
+    const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
+    value_of<DynShape, NV, F64>(p, v, a, b, c, x);
   }
 }
 
-template <bool SMEM>
-__global__ void __launch_bounds__(256) k_group_aggregate(const __grid_constant__ Plan p, int64_t max_rows,
-                                                         const int64_t* ngroups_dev, int64_t max_groups,
-                                                         int32_t replicas) {
-  extern __shared__ __align__(16) uint64_t sm[];
+template <int NV, bool F64, int MODE>
+__global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_constant__ Plan p, int64_t max_rows,
+                                                                   const int64_t* ngroups_dev, int64_t max_groups) {
+  constexpr int T = kFusedThreads;
+  extern __shared__ __align__(16) uint8_t sm[];
+  __shared__ MissStage<NV, F64> stages[T / 32];
+  const int tid = threadIdx.x;
   int64_t G = ngroups_dev ? *ngroups_dev : max_groups;
   if (G > max_groups) G = max_groups;
   const int64_t m = p.m_dev ? *p.m_dev : max_rows;
-  const int64_t words = SMEM ? (int64_t)replicas * G * p.stride / 8 : 0;
-  if constexpr (SMEM) {
-    for (int64_t i = threadIdx.x; i < words; i += blockDim.x) sm[i] = 0;
+  if constexpr (MODE != AGG_HBM) {
+    const size_t bytes = MODE == AGG_PRIV ? (size_t)G * p.priv_rec * T : (size_t)G * p.cta_stride;
+    uint4* z = (uint4*)sm;
+    for (int64_t i = tid; i < (int64_t)(bytes / 16); i += T) z[i] = make_uint4(0, 0, 0, 0);
     __syncthreads();
   }
-  const int rep = (threadIdx.x & 31) & (replicas - 1);
-  for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
-    int32_t g = __ldg(p.gids + j);
-    if (g < 0 || g >= G) continue;
-    int64_t r = p.oids ? (int64_t)__ldg(p.oids + j) : j;
-    uint8_t* e = SMEM ? (uint8_t*)sm + ((int64_t)rep * G + g) * p.stride : p.table + (int64_t)g * p.stride;
-    agg_update_row(p, e, r);
-  }
-  if constexpr (SMEM) {
-    __syncthreads();
-    // flush: one thread per (group, replica) entry with a non-zero count
-    for (int64_t i = threadIdx.x; i < (int64_t)replicas * G; i += blockDim.x) {
-      const uint8_t* se = (const uint8_t*)sm + i * p.stride;
-      uint64_t c = *(const uint64_t*)(se + 8);
-      if (c == 0) continue;
-      uint8_t* e = p.table + (i % G) * p.stride;
-      atomicAdd((unsigned long long*)(e + 8), (unsigned long long)c);
-      for (int v = 0; v < p.nvals; ++v) {
-        const DevValue& d = p.vals[v];
-        if (d.off_sum >= 0) {
-          if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(se + d.off_sum));
-          else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(se + d.off_sum),
-                               *(const uint64_t*)(se + d.off_sum + 8));
-        }
-        if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(se + d.off_min));
-        if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(se + d.off_max));
-      }
+  MissStage<NV, F64>& stage = stages[tid >> 5];
+  const int64_t per_round = (int64_t)gridDim.x * T;
+  const int64_t rounds = (m + per_round - 1) / per_round;    // uniform across the grid
+  for (int64_t round = 0; round < rounds; ++round) {
+    if (MODE == AGG_CTA && round > 0 && round % 256 == 0) {   // 256 rounds x 256 threads = 2^16 rows per CTA
+      __syncthreads();
+      for (int64_t g = tid; g < G; g += T) cta_flush_entry(p, sm + g * p.cta_stride, g);
+      __syncthreads();
     }
+    const int64_t j = round * per_round + (int64_t)blockIdx.x * T + tid;
+    Row<DynShape, NV, F64> x;
+    const int32_t g = j < m ? __ldg(p.gids + j) : -1;
+    const bool valid = g >= 0 && g < G;
+    const int64_t r = valid ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : 0;
+    if (valid) {
+      agg_eval<NV, F64>(p, r, g, x);
+    } else {
+      x.q = false;
+      x.fast = true;
+      x.key = 0;
+    }
+    bool miss = false;
+    if (valid) {
+      if (!x.fast) update_entry_slow(p, p.table + (int64_t)g * p.stride, r);
+      else if (MODE == AGG_PRIV) priv_add<DynShape, NV, F64>(p, sm, g, tid, x);
+      else if (MODE == AGG_CTA) cta_add<DynShape, NV, F64>(p, sm + (int64_t)g * p.cta_stride, x);
+      else miss = true;
+    }
+    if (MODE == AGG_HBM) warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);
+  }
+  if constexpr (MODE == AGG_PRIV) {
+    __syncthreads();
+    for (int64_t g = 0; g < G; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);
+  } else if constexpr (MODE == AGG_CTA) {
+    __syncthreads();
+    for (int64_t g = tid; g < G; g += T) cta_flush_entry(p, sm + g * p.cta_stride, g);
   }
 }
 
-constexpr size_t kAggSmemBudget = 96 * 1024;
+template <int NV, bool F64, int MODE>
+static cudaError_t launch_agg_mode(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
+                                   size_t smem, int sms, cudaStream_t s) {
+  auto fn = k_group_aggregate<NV, F64, MODE>;
+  if (smem) {
+    cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    if (e != cudaSuccess) return e;
+  }
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, smem) != cudaSuccess || nb < 1) nb = 1;
+  int64_t grid = (int64_t)sms * nb;
+  const int64_t need = (max_rows + kFusedThreads - 1) / kFusedThreads;
+  if (need < grid) grid = need > 0 ? need : 1;
+  count_launch();
+  fn<<<(int)grid, kFusedThreads, smem, s>>>(p, max_rows, ngroups_dev, max_groups);
+  return cudaGetLastError();
+}
+
+template <int NV, bool F64>
+static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
+                                 int sms, cudaStream_t s) {
+  const size_t priv = (size_t)max_groups * p.priv_rec * kFusedThreads;
+  const size_t cta = (size_t)max_groups * p.cta_stride;
+  bool int_cols = true;
+  for (int v = 0; v < p.nvals; ++v) int_cols = int_cols && !p.vals[v].is_f64 && p.vals[v].expr == OCL_EXPR_COL;
+  if (priv <= 96 * 1024) return launch_agg_mode<NV, F64, AGG_PRIV>(p, max_rows, ngroups_dev, max_groups, priv, sms, s);
+  if (int_cols && !F64 && cta <= kAggSmemBudget)
+    return launch_agg_mode<NV, F64, AGG_CTA>(p, max_rows, ngroups_dev, max_groups, cta, sms, s);
+  return launch_agg_mode<NV, F64, AGG_HBM>(p, max_rows, ngroups_dev, max_groups, 0, sms, s);
+}
+
+template <bool F64>
+static cudaError_t launch_agg_f(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
+                                int sms, cudaStream_t s) {
+  if (p.nvals <= 1) return launch_agg_nv<1, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (p.nvals <= 2) return launch_agg_nv<2, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (p.nvals <= 4) return launch_agg_nv<4, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  return launch_agg_nv<6, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+}
 
 cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
-                                   int grid, cudaStream_t s) {
+                                   bool values_f64, int sms, cudaStream_t s) {
   if (max_rows == 0 || max_groups == 0) return cudaSuccess;
-  int64_t g = (max_rows + 255) / 256;
-  if (g > grid) g = grid;
-  size_t one = (size_t)max_groups * p.stride;
-  if (one <= kAggSmemBudget) {
-    int R = 32;
-    while (R > 1 && (size_t)R * one > kAggSmemBudget) R >>= 1;
-    size_t bytes = (size_t)R * one;
-    cudaError_t e = cudaFuncSetAttribute(k_group_aggregate<true>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                                         (int)kAggSmemBudget);
-    if (e != cudaSuccess) return e;
-    count_launch();
-    k_group_aggregate<true><<<(int)g, 256, bytes, s>>>(p, max_rows, ngroups_dev, max_groups, R);
-  } else {
-    count_launch();
-    k_group_aggregate<false><<<(int)g, 256, 0, s>>>(p, max_rows, ngroups_dev, max_groups, 1);
-  }
-  return cudaGetLastError();
+  return values_f64 ? launch_agg_f<true>(p, max_rows, ngroups_dev, max_groups, sms, s)
+                    : launch_agg_f<false>(p, max_rows, ngroups_dev, max_groups, sms, s);
 }
 
 }  // namespace ocl

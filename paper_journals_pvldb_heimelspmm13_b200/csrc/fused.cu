@@ -33,502 +33,13 @@
 //    (no dtype dispatch, every value column loaded once, narrow keys in 32 bits) — the
 //    B200 stand-in for Ocelot's run-time kernel compilation.
 //    Plans whose shape matches an instantiated StaticShape run the specialised code.
-#include <type_traits>
-
-#include "launch.cuh"
-#include "rowops.cuh"
+#include "sga_device.cuh"
 
 namespace ocl {
 
-constexpr int kFusedThreads = 256;
-constexpr int kRegSlots = 4;
-constexpr int kUnits = 2;
-constexpr int kTileRows = 64 * kUnits;
-
-// ------------------------------------------------------------------ shapes
-enum : uint32_t { VF_SUM = 1, VF_MIN = 2, VF_MAX = 4 };
-// value descriptor: kind (2 bits) | a (3) | b (3) | c (3) | flags (3)
-__host__ __device__ constexpr uint32_t vop(uint32_t kind, uint32_t flags, uint32_t a, uint32_t b = 0,
-                                           uint32_t c = 0) {
-  return kind | (a << 2) | (b << 5) | (c << 8) | (flags << 11);
-}
-
-struct DynShape {
-  static constexpr bool kStatic = false;
-  static constexpr int NC = 1;
-  using Key = uint64_t;
-  __device__ static int np(const Plan& p) { return p.npreds; }
-  __device__ static int pw(const Plan& p, int i) { return p.preds[i].col.width; }
-  __device__ static bool pf64(const Plan& p, int i) { return p.preds[i].is_f64; }
-  __device__ static int nk(const Plan& p) { return p.nkeys; }
-  __device__ static int kw(const Plan& p, int i) { return p.keys[i].col.width; }
-  __device__ static int nv(const Plan& p) { return p.nvals; }
-  __device__ static int kind(const Plan& p, int v) { return p.vals[v].expr; }
-  __device__ static bool fsum(const Plan& p, int v) { return p.vals[v].off_sum >= 0; }
-  __device__ static bool fmn(const Plan& p, int v) { return p.vals[v].off_min >= 0; }
-  __device__ static bool fmx(const Plan& p, int v) { return p.vals[v].off_max >= 0; }
-  __device__ static bool vf64(const Plan& p, int v) { return p.vals[v].is_f64; }
-  __device__ static bool special(uint64_t k) { return k == ~0ULL; }
-};
-
-// PW: predicate width (0 = none); K0W/K1W: key widths (0 = absent); NC distinct
-// 8-byte value columns (int64, or fp64 when F64); OPS: vop(...) per value.
-template <int PW, bool PF64, int K0W, int K1W, int NC_, bool F64, uint32_t... OPS>
-struct StaticShape {
-  static constexpr bool kStatic = true;
-  static constexpr int NC = NC_;
-  static constexpr int KBITS = 8 * (K0W + K1W);
-  using Key = typename std::conditional<(KBITS > 0 && KBITS <= 32), uint32_t, uint64_t>::type;
-  static constexpr int NVS = sizeof...(OPS);
-  __host__ __device__ static constexpr uint32_t op(int v) {
-    const uint32_t a[NVS] = {OPS...};
-    return a[v];
-  }
-  __host__ __device__ static constexpr int np(const Plan&) { return PW ? 1 : 0; }
-  __host__ __device__ static constexpr int pw(const Plan&, int) { return PW; }
-  __host__ __device__ static constexpr bool pf64(const Plan&, int) { return PF64; }
-  __host__ __device__ static constexpr int nk(const Plan&) { return (K0W > 0) + (K1W > 0); }
-  __host__ __device__ static constexpr int kw(const Plan&, int i) { return i == 0 ? K0W : K1W; }
-  __host__ __device__ static constexpr int nv(const Plan&) { return NVS; }
-  __host__ __device__ static constexpr int kind(const Plan&, int v) { return (int)(op(v) & 3); }
-  __host__ __device__ static constexpr int ia(int v) { return (int)((op(v) >> 2) & 7); }
-  __host__ __device__ static constexpr int ib(int v) { return (int)((op(v) >> 5) & 7); }
-  __host__ __device__ static constexpr int ic(int v) { return (int)((op(v) >> 8) & 7); }
-  __host__ __device__ static constexpr bool fsum(const Plan&, int v) { return (op(v) >> 11) & VF_SUM; }
-  __host__ __device__ static constexpr bool fmn(const Plan&, int v) { return (op(v) >> 11) & VF_MIN; }
-  __host__ __device__ static constexpr bool fmx(const Plan&, int v) { return (op(v) >> 11) & VF_MAX; }
-  __host__ __device__ static constexpr bool vf64(const Plan&, int) { return F64; }
-  __device__ static bool special(Key k) {
-    if constexpr (KBITS > 0 && KBITS < 32) return false;        // narrow keys can never be ~0
-    else return k == (Key)~0ULL;
-  }
-};
-
-// ------------------------------------------------------------------ row evaluation
-template <class Sh, int NV, bool F64>
-struct Row {
-  bool q, fast;
-  typename Sh::Key key;
-  int64_t vi[F64 ? 1 : NV];
-  double vd[F64 ? NV : 1];
-};
-
-template <int W>
-__device__ __forceinline__ void ld2c(const void* base, int64_t r, uint64_t& x0, uint64_t& x1) {
-  if constexpr (W == 1) {
-    uint32_t v = __ldg((const unsigned short*)((const uint8_t*)base + r));
-    x0 = v & 0xFF;
-    x1 = v >> 8;
-  } else if constexpr (W == 4) {
-    int2 v = __ldg((const int2*)((const int32_t*)base + r));
-    x0 = (uint64_t)(int64_t)v.x;
-    x1 = (uint64_t)(int64_t)v.y;
-  } else {
-    longlong2 v = __ldg((const longlong2*)((const long long*)base + r));
-    x0 = (uint64_t)v.x;
-    x1 = (uint64_t)v.y;
-  }
-}
-
-// 2-row load with a width that is a compile-time constant for static shapes.
-__device__ __forceinline__ void ld2w(int w, const void* base, int64_t r, uint64_t& x0, uint64_t& x1) {
-  if (w == 1) ld2c<1>(base, r, x0, x1);
-  else if (w == 4) ld2c<4>(base, r, x0, x1);
-  else ld2c<8>(base, r, x0, x1);
-}
-__device__ __forceinline__ uint64_t ld1w(int w, const void* base, int64_t r) {
-  if (w == 1) return __ldg((const uint8_t*)base + r);
-  if (w == 4) return (uint64_t)(int64_t)__ldg((const int32_t*)base + r);
-  return (uint64_t)__ldg((const long long*)base + r);
-}
-
-__device__ __forceinline__ int64_t mul_wide_s32(int32_t a, int32_t b) {
-  int64_t r;
-  asm("mul.wide.s32 %0, %1, %2;" : "=l"(r) : "r"(a), "r"(b));
-  return r;
-}
-
-template <class Sh>
-__device__ __forceinline__ bool pred_ok(const Plan& p, int i, uint64_t raw) {
-  const DevPred& d = p.preds[i];
-  bool ok;
-  if (Sh::pf64(p, i)) {
-    const double x = __longlong_as_double((long long)raw);
-    ok = x >= d.flo && x <= d.fhi;
-  } else if (Sh::pw(p, i) < 8) {
-    const int32_t x = (int32_t)(uint32_t)raw;                // u8 / i32: 32-bit compare on clamped bounds
-    ok = x >= d.lo32 && x <= d.hi32;
-  } else {
-    const int64_t x = (int64_t)raw;
-    ok = x >= d.lo && x <= d.hi;
-  }
-  return ok != (bool)d.anti;
-}
-
-// Value v of one row from its raw operands.  Integer fast path: COL values that fit
-// int32 (accumulated in 64 bits), products of int32 factors via mul.wide.s32 (exact
-// in int64); anything else clears `fast` (the row takes the exact int128 path).
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void value_of(const Plan& p, int v, uint64_t ra, uint64_t rb, uint64_t rc,
-                                         Row<Sh, NV, F64>& x) {
-  const DevValue& d = p.vals[v];
-  const int kind = Sh::kind(p, v);
-  if constexpr (F64) {
-    const double a = __longlong_as_double((long long)ra);
-    if (kind == OCL_EXPR_COL) {
-      x.vd[v] = a;
-    } else {
-      double e = __dmul_rn(a, __dsub_rn(d.Sf, __longlong_as_double((long long)rb)));
-      if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) e = __dmul_rn(e, __dadd_rn(d.Sf, __longlong_as_double((long long)rc)));
-      x.vd[v] = e;
-    }
-  } else {
-    const int64_t a = (int64_t)ra;
-    if (kind == OCL_EXPR_COL) {
-      x.fast = x.fast && fits_i32(a);
-      x.vi[v] = a;
-    } else {
-      const int64_t t = (int64_t)((uint64_t)d.S - rb);
-      x.fast = x.fast && fits_i32(a) && fits_i32(t);
-      int64_t e = mul_wide_s32((int32_t)a, (int32_t)t);
-      if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) {
-        const int64_t u = (int64_t)((uint64_t)d.S + rc);
-        x.fast = x.fast && fits_i32(e) && fits_i32(u);
-        e = mul_wide_s32((int32_t)e, (int32_t)u);
-      }
-      x.vi[v] = e;
-    }
-  }
-}
-
-template <class Sh>
-__device__ __forceinline__ typename Sh::Key pack_key(const Plan& p, const uint64_t* raw) {
-  typename Sh::Key k = 0;
-#pragma unroll
-  for (int i = 0; i < kMaxKeys; ++i) {
-    if (i >= Sh::nk(p)) break;
-    k |= (typename Sh::Key)((raw[i] & p.keys[i].mask) << p.keys[i].shift);
-  }
-  return k;
-}
-
-// Both rows of a lane's 64-row unit (vector loads; full tiles only).
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void eval_pair(const Plan& p, int64_t r, Row<Sh, NV, F64>& x0, Row<Sh, NV, F64>& x1) {
-  x0.q = x1.q = true;
-  x0.fast = x1.fast = true;
-#pragma unroll
-  for (int i = 0; i < kMaxPreds; ++i) {
-    if (i >= Sh::np(p)) break;
-    uint64_t u0, u1;
-    ld2w(Sh::pw(p, i), p.preds[i].col.ptr, r, u0, u1);
-    x0.q = x0.q && pred_ok<Sh>(p, i, u0);
-    x1.q = x1.q && pred_ok<Sh>(p, i, u1);
-  }
-  uint64_t k0[kMaxKeys] = {0, 0}, k1[kMaxKeys] = {0, 0};
-#pragma unroll
-  for (int i = 0; i < kMaxKeys; ++i) {
-    if (i >= Sh::nk(p)) break;
-    ld2w(Sh::kw(p, i), p.keys[i].col.ptr, r, k0[i], k1[i]);
-  }
-  x0.key = pack_key<Sh>(p, k0);
-  x1.key = pack_key<Sh>(p, k1);
-  if constexpr (Sh::kStatic) {
-    uint64_t c0[Sh::NC], c1[Sh::NC];      // every distinct value column loaded once
-#pragma unroll
-    for (int i = 0; i < Sh::NC; ++i) ld2c<8>(p.vcols[i].ptr, r, c0[i], c1[i]);
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      value_of<Sh, NV, F64>(p, v, c0[Sh::ia(v)], c0[Sh::ib(v)], c0[Sh::ic(v)], x0);
-      value_of<Sh, NV, F64>(p, v, c1[Sh::ia(v)], c1[Sh::ib(v)], c1[Sh::ic(v)], x1);
-    }
-  } else {
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if (v >= p.nvals) break;
-      const DevValue& d = p.vals[v];
-      if (!F64 && d.is_f64) {              // mixed int/fp64 plan: fp64 values take the exact slow path
-        x0.fast = x1.fast = false;
-        continue;
-      }
-      uint64_t a0, a1, b0 = 0, b1 = 0, c0 = 0, c1 = 0;
-      ld2w(d.a.width, d.a.ptr, r, a0, a1);
-      if (d.expr >= OCL_EXPR_MUL_1MINUS) ld2w(d.b.width, d.b.ptr, r, b0, b1);
-      if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS) ld2w(d.c.width, d.c.ptr, r, c0, c1);
-      value_of<Sh, NV, F64>(p, v, a0, b0, c0, x0);
-      value_of<Sh, NV, F64>(p, v, a1, b1, c1, x1);
-    }
-  }
-}
-
-// One row with scalar loads (ragged tail, unaligned columns).
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F64>& x) {
-  x.fast = true;
-  x.key = 0;
-  x.q = r < p.n;
-  if (!x.q) return;
-#pragma unroll
-  for (int i = 0; i < kMaxPreds; ++i) {
-    if (i >= Sh::np(p)) break;
-    x.q = x.q && pred_ok<Sh>(p, i, ld1w(Sh::pw(p, i), p.preds[i].col.ptr, r));
-  }
-  uint64_t k[kMaxKeys] = {0, 0};
-#pragma unroll
-  for (int i = 0; i < kMaxKeys; ++i) {
-    if (i >= Sh::nk(p)) break;
-    k[i] = ld1w(Sh::kw(p, i), p.keys[i].col.ptr, r);
-  }
-  x.key = pack_key<Sh>(p, k);
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= Sh::nv(p)) break;
-    const DevValue& d = p.vals[v];
-    if (!F64 && d.is_f64) {
-      x.fast = false;
-      continue;
-    }
-    const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
-    const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
-    const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
-    value_of<Sh, NV, F64>(p, v, a, b, c, x);
-  }
-}
-
-// ------------------------------------------------------------------ 1. private slots
-// Record per thread per slot (offsets from the planner, Plan::priv_rec bytes):
-// count u32; per value: SUM of a COL value as i64 (fast path: int32 values), SUM of a
-// product as 96-bit (u64 lo + u32 hi), fp64 SUM as double; MIN / MAX as u64 order-
-// preserving encodings (0 = identity).  Layout [slot][field][thread].
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void priv_add(const Plan& p, uint8_t* sm, int slot, int tid, const Row<Sh, NV, F64>& x) {
-  constexpr int T = kFusedThreads;
-  uint8_t* base = sm + (size_t)slot * p.priv_rec * T;
-  ((uint32_t*)base)[tid] += 1u;
-#pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= Sh::nv(p)) break;
-    const DevValue& d = p.vals[v];
-    if constexpr (F64) {
-      const double val = x.vd[v];
-      if (Sh::fsum(p, v)) ((double*)(base + d.po_sum * T))[tid] += val;
-      if (Sh::fmn(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
-        *m = max(*m, enc_min_f(val));
-      }
-      if (Sh::fmx(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
-        *m = max(*m, enc_max_f(val));
-      }
-    } else {
-      if (Sh::vf64(p, v)) continue;
-      const int64_t val = x.vi[v];
-      if (Sh::fsum(p, v)) {
-        if (Sh::kind(p, v) == OCL_EXPR_COL) {
-          ((int64_t*)(base + d.po_sum * T))[tid] += (int64_t)(int32_t)val;
-        } else {
-          uint64_t* lo = (uint64_t*)(base + d.po_sum * T) + tid;
-          uint32_t* hi = (uint32_t*)(base + d.po_hi * T) + tid;
-          uint64_t l = *lo;
-          uint32_t h = *hi;
-          uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
-          asm("add.cc.u32 %0, %0, %3;\n\taddc.cc.u32 %1, %1, %4;\n\taddc.u32 %2, %2, %5;"
-              : "+r"(l0), "+r"(l1), "+r"(h)
-              : "r"((uint32_t)(uint64_t)val), "r"((uint32_t)((uint64_t)val >> 32)), "r"((uint32_t)(val >> 63)));
-          *lo = (uint64_t)l0 | ((uint64_t)l1 << 32);
-          *hi = h;
-        }
-      }
-      if (Sh::fmn(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
-        *m = max(*m, enc_min_i(val));
-      }
-      if (Sh::fmx(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
-        *m = max(*m, enc_max_i(val));
-      }
-    }
-  }
-}
-
-// ------------------------------------------------------------------ 2. CTA table
-// [~key u64][count u32] per value: [sum of low 16 bits u32][sum of high 16 bits s32]
-// [min u32][max u32] (order-preserving encodings, 0 = identity); int32 values only,
-// 2^16 updates per field between flushes.  64-bit CAS on the key, linear probing.
-constexpr int kSmemProbes = 16;
-constexpr int kCtaFlushRounds = 64;   // 64 rounds x 8 warps x 128 rows = 65,536 rows
-
-__device__ __forceinline__ uint8_t* cta_find_or_insert(uint8_t* tab, uint32_t cap, int32_t stride, uint64_t key) {
-  const uint64_t sk = ~key;
-  uint32_t h = (uint32_t)fmix64(key) & (cap - 1);
-  for (int probe = 0; probe < kSmemProbes; ++probe) {
-    uint64_t* kp = (uint64_t*)(tab + (size_t)h * stride);
-    uint64_t cur = *(volatile uint64_t*)kp;
-    if (cur == sk) return (uint8_t*)kp;
-    if (cur == 0) {
-      uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
-      if (prev == 0 || prev == sk) return (uint8_t*)kp;
-    }
-    h = (h + 1) & (cap - 1);
-  }
-  return nullptr;
-}
-
-__device__ __forceinline__ uint32_t enc32_max(int32_t v) { return (uint32_t)v ^ 0x80000000u; }
-__device__ __forceinline__ uint32_t enc32_min(int32_t v) { return ~enc32_max(v); }
-
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void cta_add(const Plan& p, uint8_t* e, const Row<Sh, NV, F64>& x) {
-  atomicAdd((unsigned int*)(e + 8), 1u);
-  if constexpr (!F64) {
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if (v >= Sh::nv(p)) break;
-      const DevValue& d = p.vals[v];
-      const int32_t w = (int32_t)x.vi[v];
-      if (Sh::fsum(p, v)) {
-        atomicAdd((unsigned int*)(e + d.co_lo), (unsigned int)w & 0xFFFFu);
-        atomicAdd((int*)(e + d.co_hi), w >> 16);
-      }
-      if (Sh::fmn(p, v)) atomicMax((unsigned int*)(e + d.co_min), enc32_min(w));
-      if (Sh::fmx(p, v)) atomicMax((unsigned int*)(e + d.co_max), enc32_max(w));
-    }
-  }
-}
-
-// Fold one CTA-table entry into the HBM table and reset its accumulators (key kept).
-__device__ __forceinline__ void cta_flush_entry(const Plan& p, uint8_t* ce) {
-  const uint64_t sk = *(const uint64_t*)ce;
-  const uint32_t cnt = *(const uint32_t*)(ce + 8);
-  if (sk == 0 || cnt == 0) return;
-  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
-  if (e) {
-    atomicAdd((unsigned long long*)(e + 8), (unsigned long long)cnt);
-    for (int v = 0; v < p.nvals; ++v) {
-      const DevValue& d = p.vals[v];
-      if (d.co_lo >= 0) {
-        const int64_t sum =
-            (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
-        atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)sum, (uint64_t)(sum >> 63));
-      }
-      if (d.co_min >= 0) {
-        const int32_t mn = (int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u);
-        atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
-      }
-      if (d.co_max >= 0) {
-        const int32_t mx = (int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u);
-        atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
-      }
-    }
-  }
-  for (int w = 8; w < p.cta_stride; w += 4) *(uint32_t*)(ce + w) = 0;
-}
-
-// ------------------------------------------------------------------ 3. HBM table (warp-aggregated)
-template <int NV, bool F64>
-struct MissStage {
-  int64_t vi[F64 ? 1 : NV][32];
-  double vd[F64 ? NV : 1][32];
-};
-
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F64>& st, bool miss,
-                                                 const Row<Sh, NV, F64>& x, int lane) {
-  const unsigned mmask = __ballot_sync(0xffffffffu, miss);
-  if (mmask == 0) return;
-  if (miss) {
-#pragma unroll
-    for (int v = 0; v < NV; ++v) {
-      if constexpr (F64) st.vd[v][lane] = x.vd[v];
-      else st.vi[v][lane] = x.vi[v];
-    }
-  }
-  __syncwarp();
-  if (miss) {
-    const unsigned peers = __match_any_sync(mmask, (unsigned long long)x.key);
-    if (lane == __ffs(peers) - 1) {
-      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x.key, p.status);
-      if (e) {
-        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)__popc(peers));
-#pragma unroll
-        for (int v = 0; v < NV; ++v) {
-          if (v >= Sh::nv(p)) break;
-          const DevValue& d = p.vals[v];
-          if constexpr (F64) {
-            double sum = 0.0, mn = x.vd[v], mx = x.vd[v];
-            for (unsigned b = peers; b; b &= b - 1) {
-              const double y = st.vd[v][__ffs(b) - 1];
-              sum += y;
-              mn = fmin(mn, y);
-              mx = fmax(mx, y);
-            }
-            if (Sh::fsum(p, v)) atomicAdd((double*)(e + d.off_sum), sum);
-            if (Sh::fmn(p, v)) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_f(mn));
-            if (Sh::fmx(p, v)) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_f(mx));
-          } else {
-            if (Sh::vf64(p, v)) continue;
-            I128 sum{0, 0};
-            int64_t mn = x.vi[v], mx = x.vi[v];
-            for (unsigned b = peers; b; b &= b - 1) {
-              const int64_t y = st.vi[v][__ffs(b) - 1];
-              sum = i128_add(sum, i128_from_i64(y));
-              mn = min(mn, y);
-              mx = max(mx, y);
-            }
-            if (Sh::fsum(p, v)) atomic_add_i128((uint64_t*)(e + d.off_sum), sum.lo, sum.hi);
-            if (Sh::fmn(p, v)) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(mn));
-            if (Sh::fmx(p, v)) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(mx));
-          }
-        }
-      }
-    }
-  }
-  __syncwarp();
-}
-
-// ------------------------------------------------------------------ per-row dispatch
-template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename Sh::Key (&rk)[kRegSlots],
-                                          uint8_t* sm, uint8_t* cta_tab, int tid, MissStage<NV, F64>& stage,
-                                          const Row<Sh, NV, F64>& x, int64_t r) {
-  using Key = typename Sh::Key;
-  constexpr int L = kRegSlots;
-  int slot = -1;
-#pragma unroll
-  for (int s = L - 1; s >= 0; --s)
-    if (x.key == rk[s]) slot = s;
-  const bool special = Sh::special(x.key);
-  bool go = x.q && x.fast && slot >= 0 && !special;
-  bool miss = false;
-  if (x.q && !go) {                       // new key in this CTA, a slow value, or more keys than slots
-    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, (uint64_t)x.key) : -1;
-    if (slot >= 0) {
-#pragma unroll
-      for (int s = 0; s < L; ++s) {
-        const uint64_t sk = *(volatile uint64_t*)&dir[s];
-        rk[s] = sk ? (Key)~sk : (Key)~0ULL;
-      }
-      go = true;
-    } else {
-      uint8_t* e = nullptr;
-      if (p.smem_cap && x.fast && !special) e = cta_find_or_insert(cta_tab, (uint32_t)p.smem_cap, p.cta_stride, x.key);
-      if (e) {
-        cta_add<Sh, NV, F64>(p, e, x);
-      } else if (x.fast && !special) {
-        miss = true;                      // warp-aggregated HBM update below
-      } else {
-        e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x.key, p.status);
-        if (e) update_entry_slow(p, e, r);
-      }
-    }
-  }
-  if (go) priv_add<Sh, NV, F64>(p, sm, slot, tid, x);
-  warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);
-}
-
 // ------------------------------------------------------------------ the kernel
 template <class Sh, int NV, bool F64>
-__global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ Plan p) {
+__global__ void __launch_bounds__(kFusedThreads, Sh::kStatic ? 3 : 1) k_sga(const __grid_constant__ Plan p) {
   using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
   constexpr int T = kFusedThreads;
@@ -596,57 +107,14 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
   uint8_t* blkb = (uint8_t*)blk;
   for (int s = 0; s < L; ++s) {
     if (dir[s] == 0) continue;                       // uniform: slot never used in this CTA
-    uint8_t* be = blkb + s * 256;
-    const uint8_t* rec = sm + (size_t)s * p.priv_rec * T;
-    const uint32_t c = __reduce_add_sync(0xffffffffu, ((const uint32_t*)rec)[tid]);
-    if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)c);
-    for (int v = 0; v < p.nvals; ++v) {
-      const DevValue& d = p.vals[v];
-      if (d.po_sum >= 0) {
-        if (d.is_f64) {
-          double sum = ((const double*)(rec + d.po_sum * T))[tid];
-          for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
-          if (lane == 0) atomicAdd((double*)(be + d.off_sum), sum);
-        } else {
-          I128 x;
-          x.lo = ((const uint64_t*)(rec + d.po_sum * T))[tid];
-          x.hi = d.po_hi >= 0 ? (uint64_t)(int64_t)(int32_t)((const uint32_t*)(rec + d.po_hi * T))[tid]
-                              : (uint64_t)((int64_t)x.lo >> 63);
-          x = warp_sum_i128(x);
-          if (lane == 0) atomic_add_i128((uint64_t*)(be + d.off_sum), x.lo, x.hi);
-        }
-      }
-      if (d.po_min >= 0) {
-        unsigned long long m = ((const uint64_t*)(rec + d.po_min * T))[tid];
-        for (int o = 16; o > 0; o >>= 1) m = max(m, __shfl_xor_sync(0xffffffffu, m, o));
-        if (lane == 0 && m) atomicMax((unsigned long long*)(be + d.off_min), m);
-      }
-      if (d.po_max >= 0) {
-        unsigned long long m = ((const uint64_t*)(rec + d.po_max * T))[tid];
-        for (int o = 16; o > 0; o >>= 1) m = max(m, __shfl_xor_sync(0xffffffffu, m, o));
-        if (lane == 0 && m) atomicMax((unsigned long long*)(be + d.off_max), m);
-      }
-    }
+    priv_flush_warp(p, sm + (size_t)s * p.priv_rec * T, tid, blkb + s * 256);
   }
   __syncthreads();
   if (tid < L) {
     const uint64_t sk = dir[tid];
     if (sk != 0) {
-      const uint8_t* src = blkb + tid * 256;
       uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
-      if (e) {
-        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(src + 8));
-        for (int v = 0; v < p.nvals; ++v) {
-          const DevValue& d = p.vals[v];
-          if (d.off_sum >= 0) {
-            if (d.is_f64) atomicAdd((double*)(e + d.off_sum), *(const double*)(src + d.off_sum));
-            else atomic_add_i128((uint64_t*)(e + d.off_sum), *(const uint64_t*)(src + d.off_sum),
-                                 *(const uint64_t*)(src + d.off_sum + 8));
-          }
-          if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), *(const unsigned long long*)(src + d.off_min));
-          if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), *(const unsigned long long*)(src + d.off_max));
-        }
-      }
+      if (e) entry_merge(p, blkb + tid * 256, e);
     }
   }
   if (p.smem_cap)

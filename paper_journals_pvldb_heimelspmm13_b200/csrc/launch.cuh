@@ -52,7 +52,7 @@ cudaError_t launch_merge_partials(const uint8_t* partials, int32_t nparts, int64
                                   const int64_t* part_counts, const FinPlan& f, uint8_t* table, uint64_t mask,
                                   int32_t* status, int grid, cudaStream_t s);
 cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
-                                   int grid, cudaStream_t s);
+                                   bool values_f64, int sms, cudaStream_t s);
 // Fused select -> group -> aggregate kernel (fused.cu).  mode 0: static shape if one
 // matches the plan, else dynamic; 1: dynamic shape only; 2: HBM-only kernel.
 cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind);

@@ -209,25 +209,52 @@ __global__ void k_finalize_dense(const uint8_t* table, int32_t stride, const int
 }
 
 // ------------------------------------------------------------------ group build (K6/K7)
-__global__ void k_group_insert(const __grid_constant__ Plan p, int32_t* gid_out, int64_t max_rows) {
+// Group build (K6): per row, the packed key's table slot.  A CTA-level direct-mapped
+// cache in shared memory (key -> slot, 256 lines, filled first-come) answers repeated
+// keys without touching HBM — for few groups every row after warm-up; misses probe
+// the HBM table once per distinct key per warp (__match_any_sync) with atomicCAS.
+constexpr int kGroupCache = 256;
+
+__global__ void __launch_bounds__(256) k_group_insert(const __grid_constant__ Plan p, int32_t* gid_out,
+                                                      int64_t max_rows) {
+  __shared__ unsigned long long ck[kGroupCache];
+  __shared__ unsigned int cs[kGroupCache];
+  for (int i = threadIdx.x; i < kGroupCache; i += blockDim.x) {
+    ck[i] = 0;
+    cs[i] = 0xFFFFFFFFu;
+  }
+  __syncthreads();
+  const int lane = threadIdx.x & 31;
   const int64_t m = p.m_dev ? *p.m_dev : max_rows;
   for (int64_t j0 = blockIdx.x * (int64_t)blockDim.x; j0 < m; j0 += (int64_t)gridDim.x * blockDim.x) {
-    int64_t j = j0 + threadIdx.x;
-    bool act = j < m;
-    unsigned amask = __ballot_sync(0xffffffffu, act);
-    if (!act) continue;
-    int64_t r = p.oids ? (int64_t)p.oids[j] : j;
-    uint64_t key = row_key_scalar(p, r);
-    // warp-aggregated insert: one probe per distinct key per warp
-    unsigned peers = __match_any_sync(amask, key);
-    int leader = __ffs(peers) - 1;
-    int64_t slot = -1;
-    if ((threadIdx.x & 31) == leader) {
-      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
-      slot = e ? (int64_t)((e - p.table) / p.stride) : -1;
+    const int64_t j = j0 + threadIdx.x;
+    const bool act = j < m;
+    uint64_t key = 0;
+    uint32_t slot = 0xFFFFFFFFu;
+    int h = 0;
+    if (act) {
+      const int64_t r = p.oids ? (int64_t)__ldg(p.oids + j) : j;
+      key = row_key_scalar(p, r);
+      h = (int)(fmix64(key) & (kGroupCache - 1));
+      if (*(volatile unsigned long long*)&ck[h] == ~key && key != ~0ULL) slot = *(volatile unsigned int*)&cs[h];
     }
-    slot = __shfl_sync(amask, slot, leader);
-    gid_out[j] = (int32_t)slot;
+    const bool miss = act && slot == 0xFFFFFFFFu;
+    const unsigned mmask = __ballot_sync(0xffffffffu, miss);
+    if (miss) {
+      const unsigned peers = __match_any_sync(mmask, key);
+      const int leader = __ffs(peers) - 1;
+      uint32_t s = 0xFFFFFFFFu;
+      if (lane == leader) {
+        uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
+        if (e) {
+          s = (uint32_t)((e - p.table) / p.stride);
+          if (key != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key) == 0ULL)
+            *(volatile unsigned int*)&cs[h] = s;
+        }
+      }
+      slot = __shfl_sync(peers, s, leader);
+    }
+    if (act) gid_out[j] = (int32_t)slot;   // slot index; remapped to the dense id by k_group_lookup
   }
 }
 
@@ -235,8 +262,8 @@ __global__ void k_group_lookup(const uint8_t* table, int32_t stride, const int64
                                int32_t* gid_out) {
   const int64_t m = m_dev ? *m_dev : max_rows;
   for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
-    int32_t s = gid_out[j];
-    gid_out[j] = s >= 0 ? (int32_t)*(const int64_t*)(table + (int64_t)s * stride + 8) : -1;
+    const uint32_t s = (uint32_t)gid_out[j];
+    gid_out[j] = s != 0xFFFFFFFFu ? (int32_t)*(const int64_t*)(table + (int64_t)s * stride + 8) : -1;
   }
 }
 
