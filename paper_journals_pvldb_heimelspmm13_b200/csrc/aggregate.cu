@@ -18,12 +18,13 @@
 //   HBM      otherwise: warp-aggregated (__match_any_sync on the gid) global atomics.
 // Values are read at row oids[j] (a fused gather).  Rows whose values need int128 go
 // through the exact per-row path.
+#include <algorithm>
+
 #include "sga_device.cuh"
 
 namespace ocl {
 
 constexpr size_t kAggSmemBudget = 160 * 1024;
-enum AggMode { AGG_PRIV = 0, AGG_CTA = 1, AGG_HBM = 2 };
 
 template <int NV, bool F64>
 __device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<DynShape, NV, F64>& x) {
@@ -45,9 +46,12 @@ __device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Ro
   }
 }
 
-template <int NV, bool F64, int MODE>
+// Group g goes to the private records when g < npriv, else to the CTA array when
+// g < ncta (integer COL values), else to the warp-aggregated HBM update.
+template <int NV, bool F64>
 __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_constant__ Plan p, int64_t max_rows,
-                                                                   const int64_t* ngroups_dev, int64_t max_groups) {
+                                                                   const int64_t* ngroups_dev, int64_t max_groups,
+                                                                   int32_t npriv, int32_t ncta) {
   constexpr int T = kFusedThreads;
   extern __shared__ __align__(16) uint8_t sm[];
   __shared__ MissStage<NV, F64> stages[T / 32];
@@ -55,19 +59,24 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
   int64_t G = ngroups_dev ? *ngroups_dev : max_groups;
   if (G > max_groups) G = max_groups;
   const int64_t m = p.m_dev ? *p.m_dev : max_rows;
-  if constexpr (MODE != AGG_HBM) {
-    const size_t bytes = MODE == AGG_PRIV ? (size_t)G * p.priv_rec * T : (size_t)G * p.cta_stride;
+  const int64_t np_ = npriv < G ? npriv : G;
+  const int64_t nc_ = ncta < G ? ncta : G;
+  uint8_t* cta = sm + (size_t)npriv * p.priv_rec * T;
+  {
+    const size_t bytes = (size_t)np_ * p.priv_rec * T;
     uint4* z = (uint4*)sm;
     for (int64_t i = tid; i < (int64_t)(bytes / 16); i += T) z[i] = make_uint4(0, 0, 0, 0);
+    uint4* zc = (uint4*)cta;
+    for (int64_t i = tid; i < (int64_t)((size_t)nc_ * p.cta_stride / 16); i += T) zc[i] = make_uint4(0, 0, 0, 0);
     __syncthreads();
   }
   MissStage<NV, F64>& stage = stages[tid >> 5];
   const int64_t per_round = (int64_t)gridDim.x * T;
   const int64_t rounds = (m + per_round - 1) / per_round;    // uniform across the grid
   for (int64_t round = 0; round < rounds; ++round) {
-    if (MODE == AGG_CTA && round > 0 && round % 256 == 0) {   // 256 rounds x 256 threads = 2^16 rows per CTA
+    if (nc_ > np_ && round > 0 && round % 256 == 0) {          // 256 rounds x 256 threads = 2^16 rows per CTA
       __syncthreads();
-      for (int64_t g = tid; g < G; g += T) cta_flush_entry(p, sm + g * p.cta_stride, g);
+      for (int64_t g = np_ + tid; g < nc_; g += T) cta_flush_entry(p, cta + g * p.cta_stride, g);
       __syncthreads();
     }
     const int64_t j = round * per_round + (int64_t)blockIdx.x * T + tid;
@@ -85,50 +94,40 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
     bool miss = false;
     if (valid) {
       if (!x.fast) update_entry_slow(p, p.table + (int64_t)g * p.stride, r);
-      else if (MODE == AGG_PRIV) priv_add<DynShape, NV, F64>(p, sm, g, tid, x);
-      else if (MODE == AGG_CTA) cta_add<DynShape, NV, F64>(p, sm + (int64_t)g * p.cta_stride, x);
+      else if (g < np_) priv_add<DynShape, NV, F64>(p, sm, g, tid, x);
+      else if (g < nc_) cta_add<DynShape, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
       else miss = true;
     }
-    if (MODE == AGG_HBM) warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);
+    warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);
   }
-  if constexpr (MODE == AGG_PRIV) {
-    __syncthreads();
-    for (int64_t g = 0; g < G; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);
-  } else if constexpr (MODE == AGG_CTA) {
-    __syncthreads();
-    for (int64_t g = tid; g < G; g += T) cta_flush_entry(p, sm + g * p.cta_stride, g);
-  }
+  __syncthreads();
+  for (int64_t g = 0; g < np_; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);
+  for (int64_t g = np_ + tid; g < nc_; g += T) cta_flush_entry(p, cta + g * p.cta_stride, g);
 }
 
-template <int NV, bool F64, int MODE>
-static cudaError_t launch_agg_mode(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
-                                   size_t smem, int sms, cudaStream_t s) {
-  auto fn = k_group_aggregate<NV, F64, MODE>;
-  if (smem) {
-    cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-    if (e != cudaSuccess) return e;
-  }
+template <int NV, bool F64>
+static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
+                                 int sms, cudaStream_t s) {
+  // private records for the first groups (up to 96 KB), then a CTA array for integer COL plans
+  int64_t npriv = std::min<int64_t>(max_groups, (int64_t)(96 * 1024 / ((size_t)p.priv_rec * kFusedThreads)));
+  bool int_cols = true;
+  for (int v = 0; v < p.nvals; ++v) int_cols = int_cols && !p.vals[v].is_f64 && p.vals[v].expr == OCL_EXPR_COL;
+  int64_t ncta = npriv;
+  if (int_cols && !F64)
+    ncta = std::min<int64_t>(max_groups, npriv + (int64_t)((kAggSmemBudget - (size_t)npriv * p.priv_rec * kFusedThreads) /
+                                                            (size_t)p.cta_stride));
+  const size_t smem = (size_t)npriv * p.priv_rec * kFusedThreads + (size_t)ncta * p.cta_stride;
+  auto fn = k_group_aggregate<NV, F64>;
+  cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  if (e != cudaSuccess) return e;
   int nb = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, smem) != cudaSuccess || nb < 1) nb = 1;
   int64_t grid = (int64_t)sms * nb;
   const int64_t need = (max_rows + kFusedThreads - 1) / kFusedThreads;
   if (need < grid) grid = need > 0 ? need : 1;
   count_launch();
-  fn<<<(int)grid, kFusedThreads, smem, s>>>(p, max_rows, ngroups_dev, max_groups);
+  fn<<<(int)grid, kFusedThreads, smem, s>>>(p, max_rows, ngroups_dev, max_groups, (int32_t)npriv, (int32_t)ncta);
   return cudaGetLastError();
-}
-
-template <int NV, bool F64>
-static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
-                                 int sms, cudaStream_t s) {
-  const size_t priv = (size_t)max_groups * p.priv_rec * kFusedThreads;
-  const size_t cta = (size_t)max_groups * p.cta_stride;
-  bool int_cols = true;
-  for (int v = 0; v < p.nvals; ++v) int_cols = int_cols && !p.vals[v].is_f64 && p.vals[v].expr == OCL_EXPR_COL;
-  if (priv <= 96 * 1024) return launch_agg_mode<NV, F64, AGG_PRIV>(p, max_rows, ngroups_dev, max_groups, priv, sms, s);
-  if (int_cols && !F64 && cta <= kAggSmemBudget)
-    return launch_agg_mode<NV, F64, AGG_CTA>(p, max_rows, ngroups_dev, max_groups, cta, sms, s);
-  return launch_agg_mode<NV, F64, AGG_HBM>(p, max_rows, ngroups_dev, max_groups, 0, sms, s);
 }
 
 template <bool F64>

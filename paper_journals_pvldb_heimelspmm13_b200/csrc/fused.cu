@@ -39,7 +39,7 @@ namespace ocl {
 
 // ------------------------------------------------------------------ the kernel
 template <class Sh, int NV, bool F64>
-__global__ void __launch_bounds__(kFusedThreads, Sh::kStatic ? 3 : 1) k_sga(const __grid_constant__ Plan p) {
+__global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ Plan p) {
   using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
   constexpr int T = kFusedThreads;
@@ -79,15 +79,31 @@ __global__ void __launch_bounds__(kFusedThreads, Sh::kStatic ? 3 : 1) k_sga(cons
     if (t >= ntiles) continue;
     const int64_t base = t * kTileRows;
     if (p.vec_ok && base + kTileRows <= p.n) {
-      Row<Sh, NV, F64> x[kUnits][2];
+      if constexpr (Sh::kStatic) {
+        RawUnit<Sh> raw[kUnits];
 #pragma unroll
-      for (int u = 0; u < kUnits; ++u) eval_pair<Sh, NV, F64>(p, base + 64 * u + 2 * lane, x[u][0], x[u][1]);
+        for (int u = 0; u < kUnits; ++u) load_unit<Sh>(p, base + 64 * u + 2 * lane, raw[u]);
 #pragma unroll
-      for (int u = 0; u < kUnits; ++u) {
-        const int64_t r = base + 64 * u + 2 * lane;
-        if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x[u][0].q, x[u][1].q);
-        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][0], r);
-        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][1], r + 1);
+        for (int u = 0; u < kUnits; ++u) {
+          const int64_t r = base + 64 * u + 2 * lane;
+          Row<Sh, NV, F64> x0, x1;
+          eval_unit<Sh, NV, F64>(p, raw[u], 0, x0);
+          eval_unit<Sh, NV, F64>(p, raw[u], 1, x1);
+          if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+        }
+      } else {
+        Row<Sh, NV, F64> x[kUnits][2];
+#pragma unroll
+        for (int u = 0; u < kUnits; ++u) eval_pair<Sh, NV, F64>(p, base + 64 * u + 2 * lane, x[u][0], x[u][1]);
+#pragma unroll
+        for (int u = 0; u < kUnits; ++u) {
+          const int64_t r = base + 64 * u + 2 * lane;
+          if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x[u][0].q, x[u][1].q);
+          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][0], r);
+          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][1], r + 1);
+        }
       }
     } else {
       for (int u = 0; u < kUnits; ++u) {

@@ -232,6 +232,47 @@ __device__ __forceinline__ void eval_pair(const Plan& p, int64_t r, Row<Sh, NV, 
   }
 }
 
+// Static shapes: raw column words of one 64-row unit (both rows of the lane), loaded
+// for every unit of a tile before any row is evaluated (loads in flight, few live
+// registers: values are computed per unit just before they are placed).
+template <class Sh>
+struct RawUnit {
+  uint64_t pr[2];
+  uint64_t k[2][kMaxKeys];
+  uint64_t c[2][Sh::NC];
+};
+
+template <class Sh>
+__device__ __forceinline__ void load_unit(const Plan& p, int64_t r, RawUnit<Sh>& u) {
+  if constexpr (Sh::kStatic) {
+    if (Sh::np(p) > 0) ld2w(Sh::pw(p, 0), p.preds[0].col.ptr, r, u.pr[0], u.pr[1]);
+#pragma unroll
+    for (int i = 0; i < kMaxKeys; ++i) {
+      if (i >= Sh::nk(p)) break;
+      ld2w(Sh::kw(p, i), p.keys[i].col.ptr, r, u.k[0][i], u.k[1][i]);
+    }
+#pragma unroll
+    for (int i = 0; i < Sh::NC; ++i) ld2c<8>(p.vcols[i].ptr, r, u.c[0][i], u.c[1][i]);
+  }
+}
+
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void eval_unit(const Plan& p, const RawUnit<Sh>& u, int k, Row<Sh, NV, F64>& x) {
+  if constexpr (Sh::kStatic) {
+    x.q = Sh::np(p) > 0 ? pred_ok<Sh>(p, 0, u.pr[k]) : true;
+    x.fast = true;
+    uint64_t kk[kMaxKeys] = {0, 0};
+#pragma unroll
+    for (int i = 0; i < kMaxKeys; ++i) {
+      if (i >= Sh::nk(p)) break;
+      kk[i] = u.k[k][i];
+    }
+    x.key = pack_key<Sh>(p, kk);
+#pragma unroll
+    for (int v = 0; v < NV; ++v) value_of<Sh, NV, F64>(p, v, u.c[k][Sh::ia(v)], u.c[k][Sh::ib(v)], u.c[k][Sh::ic(v)], x);
+  }
+}
+
 // One row with scalar loads (ragged tail, unaligned columns).
 template <class Sh, int NV, bool F64>
 __device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F64>& x) {

@@ -217,6 +217,7 @@ constexpr int kGroupCache = 256;
 
 __global__ void __launch_bounds__(256) k_group_insert(const __grid_constant__ Plan p, int32_t* gid_out,
                                                       int64_t max_rows) {
+  constexpr int R = 4;                     // rows per thread per iteration (independent gathers in flight)
   __shared__ unsigned long long ck[kGroupCache];
   __shared__ unsigned int cs[kGroupCache];
   for (int i = threadIdx.x; i < kGroupCache; i += blockDim.x) {
@@ -226,35 +227,41 @@ __global__ void __launch_bounds__(256) k_group_insert(const __grid_constant__ Pl
   __syncthreads();
   const int lane = threadIdx.x & 31;
   const int64_t m = p.m_dev ? *p.m_dev : max_rows;
-  for (int64_t j0 = blockIdx.x * (int64_t)blockDim.x; j0 < m; j0 += (int64_t)gridDim.x * blockDim.x) {
-    const int64_t j = j0 + threadIdx.x;
-    const bool act = j < m;
-    uint64_t key = 0;
-    uint32_t slot = 0xFFFFFFFFu;
-    int h = 0;
-    if (act) {
-      const int64_t r = p.oids ? (int64_t)__ldg(p.oids + j) : j;
-      key = row_key_scalar(p, r);
-      h = (int)(fmix64(key) & (kGroupCache - 1));
-      if (*(volatile unsigned long long*)&ck[h] == ~key && key != ~0ULL) slot = *(volatile unsigned int*)&cs[h];
+  const int64_t step = (int64_t)gridDim.x * blockDim.x * R;
+  for (int64_t j0 = (int64_t)blockIdx.x * blockDim.x * R; j0 < m; j0 += step) {
+    uint64_t key[R];
+    int64_t j[R];
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      j[k] = j0 + k * (int64_t)blockDim.x + threadIdx.x;
+      key[k] = 0;
+      if (j[k] < m) key[k] = row_key_scalar(p, p.oids ? (int64_t)__ldg(p.oids + j[k]) : j[k]);
     }
-    const bool miss = act && slot == 0xFFFFFFFFu;
-    const unsigned mmask = __ballot_sync(0xffffffffu, miss);
-    if (miss) {
-      const unsigned peers = __match_any_sync(mmask, key);
-      const int leader = __ffs(peers) - 1;
-      uint32_t s = 0xFFFFFFFFu;
-      if (lane == leader) {
-        uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
-        if (e) {
-          s = (uint32_t)((e - p.table) / p.stride);
-          if (key != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key) == 0ULL)
-            *(volatile unsigned int*)&cs[h] = s;
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      const bool act = j[k] < m;
+      uint32_t slot = 0xFFFFFFFFu;
+      const int h = (int)(fmix64(key[k]) & (kGroupCache - 1));
+      if (act && key[k] != ~0ULL && *(volatile unsigned long long*)&ck[h] == ~key[k])
+        slot = *(volatile unsigned int*)&cs[h];
+      const bool miss = act && slot == 0xFFFFFFFFu;
+      const unsigned mmask = __ballot_sync(0xffffffffu, miss);
+      if (miss) {
+        const unsigned peers = __match_any_sync(mmask, key[k]);
+        const int leader = __ffs(peers) - 1;
+        uint32_t s = 0xFFFFFFFFu;
+        if (lane == leader) {
+          uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
+          if (e) {
+            s = (uint32_t)((e - p.table) / p.stride);
+            if (key[k] != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key[k]) == 0ULL)
+              *(volatile unsigned int*)&cs[h] = s;
+          }
         }
+        slot = __shfl_sync(peers, s, leader);
       }
-      slot = __shfl_sync(peers, s, leader);
+      if (act) gid_out[j[k]] = (int32_t)slot;   // slot index; remapped to the dense id by k_group_lookup
     }
-    if (act) gid_out[j] = (int32_t)slot;   // slot index; remapped to the dense id by k_group_lookup
   }
 }
 
@@ -353,7 +360,7 @@ cudaError_t launch_finalize_dense(const uint8_t* table, int32_t stride, const in
 
 cudaError_t launch_group_insert(const Plan& p, int32_t* gid_out, int64_t max_rows, int grid, cudaStream_t s) {
   if (max_rows == 0) return cudaSuccess;
-  int64_t g = (max_rows + 255) / 256;
+  int64_t g = (max_rows + 1023) / 1024;
   if (g > grid) g = grid;
   count_launch();
   k_group_insert<<<(int)g, 256, 0, s>>>(p, gid_out, max_rows);
