@@ -375,6 +375,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   p.status = a->dev_status;
   p.bitmap_out = a->bitmap_out;
   p.smem_cap = plan_smem_cap(a, p);
+  p.miss_agg = a->expected_groups > reg_tier_slots() ? 1 : 0;
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;
   f.keys_out = a->keys_out;

@@ -30,6 +30,7 @@ template <int NV, bool F64>
 __device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<DynShape, NV, F64>& x) {
   x.q = true;
   x.fast = true;
+  x.bad = 0;
   x.key = (uint64_t)(uint32_t)g;
 #pragma unroll
   for (int v = 0; v < NV; ++v) {
@@ -44,6 +45,7 @@ __device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Ro
     const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
     value_of<DynShape, NV, F64>(p, v, a, b, c, x);
   }
+  x.fast = x.fast && x.bad == 0;
 }
 
 // Group g goes to the private records when g < npriv, else to the CTA array when
@@ -89,6 +91,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
     } else {
       x.q = false;
       x.fast = true;
+      x.bad = 0;
       x.key = 0;
     }
     bool miss = false;
@@ -98,7 +101,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
       else if (g < nc_) cta_add<DynShape, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
       else miss = true;
     }
-    warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);
+    warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);   // (always on: G may exceed the tiers)
   }
   __syncthreads();
   for (int64_t g = 0; g < np_; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);

@@ -161,7 +161,7 @@ struct Plan {
   int32_t smem_cap;     // register tier: per-CTA shared-memory hash table entries (0 = none; power of two)
   int32_t cta_stride;   // bytes per CTA-table entry
   int32_t direct;       // 1: HBM table indexed by the key itself (grouped aggregation over dense gids)
-  int32_t pad3_;
+  int32_t miss_agg;     // 1: rows that miss the private slots / CTA table are warp-aggregated (many groups)
   int32_t* status;      // device status word (may be null)
   uint32_t* bitmap_out; // optional selection bitmap
   const int32_t* gids;  // unfused aggregate: direct group ids (table indexed by gid)

@@ -38,7 +38,7 @@
 namespace ocl {
 
 // ------------------------------------------------------------------ the kernel
-template <class Sh, int NV, bool F64>
+template <class Sh, int NV, bool F64, bool MISS>
 __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ Plan p) {
   using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
@@ -46,7 +46,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
   extern __shared__ __align__(16) uint8_t sm[];
   __shared__ uint64_t dir[L];
   __shared__ __align__(16) uint64_t blk[L * 32];   // CTA-level entry per slot (stride <= 256 B)
-  __shared__ MissStage<NV, F64> stages[T / 32];
+  __shared__ MissStage<MISS ? NV : 1, F64> stages[MISS ? T / 32 : 1];
   const int tid = threadIdx.x, lane = tid & 31;
   uint8_t* cta_tab = sm + (size_t)L * p.priv_rec * T;
   {
@@ -60,7 +60,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
   Key rk[L];
 #pragma unroll
   for (int s = 0; s < L; ++s) rk[s] = (Key)~0ULL;   // never matches an admissible key
-  MissStage<NV, F64>& stage = stages[tid >> 5];
+  MissStage<MISS ? NV : 1, F64>& stage = stages[MISS ? tid >> 5 : 0];
 
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
@@ -70,7 +70,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
   const int64_t first = (int64_t)blockIdx.x * (T / 32);
   const int64_t rounds = ntiles > first ? (ntiles - first + nwarps - 1) / nwarps : 0;
   for (int64_t round = 0; round < rounds; ++round) {
-    if (p.smem_cap && round > 0 && round % kCtaFlushRounds == 0) {
+    if (Sh::kCta && p.smem_cap && round > 0 && round % kCtaFlushRounds == 0) {
       __syncthreads();
       for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
       __syncthreads();
@@ -90,8 +90,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
           eval_unit<Sh, NV, F64>(p, raw[u], 0, x0);
           eval_unit<Sh, NV, F64>(p, raw[u], 1, x1);
           if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
-          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
         }
       } else {
         Row<Sh, NV, F64> x[kUnits][2];
@@ -101,8 +101,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
         for (int u = 0; u < kUnits; ++u) {
           const int64_t r = base + 64 * u + 2 * lane;
           if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x[u][0].q, x[u][1].q);
-          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][0], r);
-          place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x[u][1], r + 1);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x[u][0], r);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x[u][1], r + 1);
         }
       }
     } else {
@@ -112,8 +112,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
         eval_one<Sh, NV, F64>(p, r, x0);
         eval_one<Sh, NV, F64>(p, r + 1, x1);
         if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
-        place_row<Sh, NV, F64>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+        place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+        place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
       }
     }
   }
@@ -133,7 +133,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
       if (e) entry_merge(p, blkb + tid * 256, e);
     }
   }
-  if (p.smem_cap)
+  if (Sh::kCta && p.smem_cap)
     for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
 }
 
@@ -254,7 +254,7 @@ static bool shape_match(const Plan& g) {
     if (g.preds[i].col.width != Sh::pw(g, i) || (bool)g.preds[i].is_f64 != Sh::pf64(g, i)) return false;
   for (int i = 0; i < g.nkeys; ++i)
     if (g.keys[i].col.width != Sh::kw(g, i)) return false;
-  if (g.ncols != Sh::NC) return false;
+  if (g.ncols != Sh::NC || g.priv_rec != Sh::rec(g)) return false;
   for (int i = 0; i < g.ncols; ++i)
     if (g.vcols[i].width != 8 || (g.vcols[i].dtype == OCL_F64) != Sh::vf64(g, 0)) return false;
   for (int v = 0; v < g.nvals; ++v) {
@@ -262,6 +262,9 @@ static bool shape_match(const Plan& g) {
     if (d.expr != Sh::kind(g, v) || (bool)d.is_f64 != Sh::vf64(g, v)) return false;
     if ((d.off_sum >= 0) != Sh::fsum(g, v) || (d.off_min >= 0) != Sh::fmn(g, v) ||
         (d.off_max >= 0) != Sh::fmx(g, v))
+      return false;
+    if (d.po_sum != Sh::po_sum(g, v) || d.po_hi != Sh::po_hi(g, v) || d.po_min != Sh::po_min(g, v) ||
+        d.po_max != Sh::po_max(g, v))
       return false;
     if (d.ia != Sh::ia(v)) return false;
     if (d.expr >= OCL_EXPR_MUL_1MINUS && d.ib != Sh::ib(v)) return false;
@@ -275,21 +278,27 @@ static size_t reg_smem(const Plan& p) {
   return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.cta_stride;
 }
 
-template <class Sh, int NV, bool F64>
-static cudaError_t launch_k(const Plan& p, int sms, cudaStream_t s) {
+template <class Sh, int NV, bool F64, bool MISS>
+static cudaError_t launch_km(const Plan& p, int sms, cudaStream_t s) {
   const size_t smem = reg_smem(p);
-  cudaError_t e = cudaFuncSetAttribute(k_sga<Sh, NV, F64>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+  auto fn = k_sga<Sh, NV, F64, MISS>;
+  cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
   int nb = 0;
-  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, k_sga<Sh, NV, F64>, kFusedThreads, smem) != cudaSuccess ||
-      nb < 1)
-    nb = 1;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, smem) != cudaSuccess || nb < 1) nb = 1;
   int64_t grid = (int64_t)sms * nb;
   const int64_t need = ((p.n + kTileRows - 1) / kTileRows + (kFusedThreads / 32) - 1) / (kFusedThreads / 32);
   if (need < grid) grid = need > 0 ? need : 1;
   count_launch();
-  k_sga<Sh, NV, F64><<<(int)grid, kFusedThreads, smem, s>>>(p);
+  fn<<<(int)grid, kFusedThreads, smem, s>>>(p);
   return cudaGetLastError();
+}
+
+// The warp-aggregated miss path is compiled in only for plans that expect more groups
+// than private slots (Plan::miss_agg): few-group plans keep the lean row loop.
+template <class Sh, int NV, bool F64>
+static cudaError_t launch_k(const Plan& p, int sms, cudaStream_t s) {
+  return p.miss_agg ? launch_km<Sh, NV, F64, true>(p, sms, s) : launch_km<Sh, NV, F64, false>(p, sms, s);
 }
 
 template <bool F64>

@@ -26,6 +26,7 @@ __host__ __device__ constexpr uint32_t vop(uint32_t kind, uint32_t flags, uint32
 
 struct DynShape {
   static constexpr bool kStatic = false;
+  static constexpr bool kCta = true;       // the CTA table may be used (decided at run time by smem_cap)
   static constexpr int NC = 1;
   using Key = uint64_t;
   __device__ static int np(const Plan& p) { return p.npreds; }
@@ -40,6 +41,11 @@ struct DynShape {
   __device__ static bool fmx(const Plan& p, int v) { return p.vals[v].off_max >= 0; }
   __device__ static bool vf64(const Plan& p, int v) { return p.vals[v].is_f64; }
   __device__ static bool special(uint64_t k) { return k == ~0ULL; }
+  __device__ static int po_sum(const Plan& p, int v) { return p.vals[v].po_sum; }
+  __device__ static int po_hi(const Plan& p, int v) { return p.vals[v].po_hi; }
+  __device__ static int po_min(const Plan& p, int v) { return p.vals[v].po_min; }
+  __device__ static int po_max(const Plan& p, int v) { return p.vals[v].po_max; }
+  __device__ static int rec(const Plan& p) { return p.priv_rec; }
 };
 
 // PW: predicate width (0 = none); K0W/K1W: key widths (0 = absent); NC distinct
@@ -55,6 +61,12 @@ struct StaticShape {
     const uint32_t a[NVS] = {OPS...};
     return a[v];
   }
+  __host__ __device__ static constexpr bool all_int_cols() {
+    for (int v = 0; v < NVS; ++v)
+      if ((op(v) & 3) != 0) return false;
+    return !F64;
+  }
+  static constexpr bool kCta = all_int_cols();   // the CTA table holds int32 COL values only
   __host__ __device__ static constexpr int np(const Plan&) { return PW ? 1 : 0; }
   __host__ __device__ static constexpr int pw(const Plan&, int) { return PW; }
   __host__ __device__ static constexpr bool pf64(const Plan&, int) { return PF64; }
@@ -73,12 +85,53 @@ struct StaticShape {
     if constexpr (KBITS > 0 && KBITS < 32) return false;        // narrow keys can never be ~0
     else return k == (Key)~0ULL;
   }
+  // Private-record layout at compile time; the planner (abi.cu plan_values) builds the
+  // same layout at run time and shape_match checks they agree.  field: 0 sum, 1 hi, 2 min, 3 max.
+  __host__ __device__ static constexpr int po_field(int v, int field) {
+    int rec = 4, out = -1;
+    for (int i = 0; i <= v; ++i) {
+      const uint32_t f = op(i) >> 11;
+      int ps = -1, ph = -1, pn = -1, px = -1;
+      if (f & VF_SUM) {
+        rec = (rec + 7) & ~7;
+        ps = rec;
+        rec += 8;
+        if (!F64 && (op(i) & 3) != 0) { ph = rec; rec += 4; }
+      }
+      if (f & VF_MIN) { rec = (rec + 7) & ~7; pn = rec; rec += 8; }
+      if (f & VF_MAX) { rec = (rec + 7) & ~7; px = rec; rec += 8; }
+      if (i == v) out = field == 0 ? ps : field == 1 ? ph : field == 2 ? pn : px;
+    }
+    return out;
+  }
+  __host__ __device__ static constexpr int rec_bytes() {
+    int rec = 4;
+    for (int i = 0; i < NVS; ++i) {
+      const uint32_t f = op(i) >> 11;
+      if (f & VF_SUM) { rec = ((rec + 7) & ~7) + 8; if (!F64 && (op(i) & 3) != 0) rec += 4; }
+      if (f & VF_MIN) rec = ((rec + 7) & ~7) + 8;
+      if (f & VF_MAX) rec = ((rec + 7) & ~7) + 8;
+    }
+    return (rec + 7) & ~7;
+  }
+  __host__ __device__ static constexpr int po_sum(const Plan&, int v) { return po_field(v, 0); }
+  __host__ __device__ static constexpr int po_hi(const Plan&, int v) { return po_field(v, 1); }
+  __host__ __device__ static constexpr int po_min(const Plan&, int v) { return po_field(v, 2); }
+  __host__ __device__ static constexpr int po_max(const Plan&, int v) { return po_field(v, 3); }
+  __host__ __device__ static constexpr int rec(const Plan&) { return rec_bytes(); }
 };
 
 // ------------------------------------------------------------------ row evaluation
+// Non-zero iff x does not fit int32: the high word differs from the sign of the low
+// word (SHF + LOP3; checks are OR-ed and tested once per row).
+__device__ __forceinline__ uint32_t i32_bad(int64_t x) {
+  return (uint32_t)((uint64_t)x >> 32) ^ (uint32_t)((int32_t)(uint32_t)x >> 31);
+}
+
 template <class Sh, int NV, bool F64>
 struct Row {
   bool q, fast;
+  uint32_t bad;                            // int32 range violations of the fast path (0 = none)
   typename Sh::Key key;
   int64_t vi[F64 ? 1 : NV];
   double vd[F64 ? NV : 1];
@@ -156,15 +209,15 @@ __device__ __forceinline__ void value_of(const Plan& p, int v, uint64_t ra, uint
   } else {
     const int64_t a = (int64_t)ra;
     if (kind == OCL_EXPR_COL) {
-      x.fast = x.fast && fits_i32(a);
+      x.bad |= i32_bad(a);
       x.vi[v] = a;
     } else {
       const int64_t t = (int64_t)((uint64_t)d.S - rb);
-      x.fast = x.fast && fits_i32(a) && fits_i32(t);
+      x.bad |= i32_bad(a) | i32_bad(t);
       int64_t e = mul_wide_s32((int32_t)a, (int32_t)t);
       if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) {
         const int64_t u = (int64_t)((uint64_t)d.S + rc);
-        x.fast = x.fast && fits_i32(e) && fits_i32(u);
+        x.bad |= i32_bad(e) | i32_bad(u);
         e = mul_wide_s32((int32_t)e, (int32_t)u);
       }
       x.vi[v] = e;
@@ -188,6 +241,7 @@ template <class Sh, int NV, bool F64>
 __device__ __forceinline__ void eval_pair(const Plan& p, int64_t r, Row<Sh, NV, F64>& x0, Row<Sh, NV, F64>& x1) {
   x0.q = x1.q = true;
   x0.fast = x1.fast = true;
+  x0.bad = x1.bad = 0;
 #pragma unroll
   for (int i = 0; i < kMaxPreds; ++i) {
     if (i >= Sh::np(p)) break;
@@ -230,6 +284,8 @@ __device__ __forceinline__ void eval_pair(const Plan& p, int64_t r, Row<Sh, NV, 
       value_of<Sh, NV, F64>(p, v, a1, b1, c1, x1);
     }
   }
+  x0.fast = x0.fast && x0.bad == 0;
+  x1.fast = x1.fast && x1.bad == 0;
 }
 
 // Static shapes: raw column words of one 64-row unit (both rows of the lane), loaded
@@ -261,6 +317,7 @@ __device__ __forceinline__ void eval_unit(const Plan& p, const RawUnit<Sh>& u, i
   if constexpr (Sh::kStatic) {
     x.q = Sh::np(p) > 0 ? pred_ok<Sh>(p, 0, u.pr[k]) : true;
     x.fast = true;
+    x.bad = 0;
     uint64_t kk[kMaxKeys] = {0, 0};
 #pragma unroll
     for (int i = 0; i < kMaxKeys; ++i) {
@@ -270,6 +327,7 @@ __device__ __forceinline__ void eval_unit(const Plan& p, const RawUnit<Sh>& u, i
     x.key = pack_key<Sh>(p, kk);
 #pragma unroll
     for (int v = 0; v < NV; ++v) value_of<Sh, NV, F64>(p, v, u.c[k][Sh::ia(v)], u.c[k][Sh::ib(v)], u.c[k][Sh::ic(v)], x);
+    x.fast = x.bad == 0;
   }
 }
 
@@ -277,6 +335,7 @@ __device__ __forceinline__ void eval_unit(const Plan& p, const RawUnit<Sh>& u, i
 template <class Sh, int NV, bool F64>
 __device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F64>& x) {
   x.fast = true;
+  x.bad = 0;
   x.key = 0;
   x.q = r < p.n;
   if (!x.q) return;
@@ -305,6 +364,7 @@ __device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F
     const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
     value_of<Sh, NV, F64>(p, v, a, b, c, x);
   }
+  x.fast = x.fast && x.bad == 0;
 }
 
 // ------------------------------------------------------------------ 1. private slots
@@ -315,21 +375,20 @@ __device__ __forceinline__ void eval_one(const Plan& p, int64_t r, Row<Sh, NV, F
 template <class Sh, int NV, bool F64>
 __device__ __forceinline__ void priv_add(const Plan& p, uint8_t* sm, int slot, int tid, const Row<Sh, NV, F64>& x) {
   constexpr int T = kFusedThreads;
-  uint8_t* base = sm + (size_t)slot * p.priv_rec * T;
+  uint8_t* base = sm + (size_t)slot * Sh::rec(p) * T;
   ((uint32_t*)base)[tid] += 1u;
 #pragma unroll
   for (int v = 0; v < NV; ++v) {
     if (v >= Sh::nv(p)) break;
-    const DevValue& d = p.vals[v];
     if constexpr (F64) {
       const double val = x.vd[v];
-      if (Sh::fsum(p, v)) ((double*)(base + d.po_sum * T))[tid] += val;
+      if (Sh::fsum(p, v)) ((double*)(base + Sh::po_sum(p, v) * T))[tid] += val;
       if (Sh::fmn(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
+        uint64_t* m = (uint64_t*)(base + Sh::po_min(p, v) * T) + tid;
         *m = max(*m, enc_min_f(val));
       }
       if (Sh::fmx(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
+        uint64_t* m = (uint64_t*)(base + Sh::po_max(p, v) * T) + tid;
         *m = max(*m, enc_max_f(val));
       }
     } else {
@@ -337,10 +396,10 @@ __device__ __forceinline__ void priv_add(const Plan& p, uint8_t* sm, int slot, i
       const int64_t val = x.vi[v];
       if (Sh::fsum(p, v)) {
         if (Sh::kind(p, v) == OCL_EXPR_COL) {
-          ((int64_t*)(base + d.po_sum * T))[tid] += (int64_t)(int32_t)val;
+          ((int64_t*)(base + Sh::po_sum(p, v) * T))[tid] += (int64_t)(int32_t)val;
         } else {
-          uint64_t* lo = (uint64_t*)(base + d.po_sum * T) + tid;
-          uint32_t* hi = (uint32_t*)(base + d.po_hi * T) + tid;
+          uint64_t* lo = (uint64_t*)(base + Sh::po_sum(p, v) * T) + tid;
+          uint32_t* hi = (uint32_t*)(base + Sh::po_hi(p, v) * T) + tid;
           uint64_t l = *lo;
           uint32_t h = *hi;
           uint32_t l0 = (uint32_t)l, l1 = (uint32_t)(l >> 32);
@@ -352,11 +411,11 @@ __device__ __forceinline__ void priv_add(const Plan& p, uint8_t* sm, int slot, i
         }
       }
       if (Sh::fmn(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_min * T) + tid;
+        uint64_t* m = (uint64_t*)(base + Sh::po_min(p, v) * T) + tid;
         *m = max(*m, enc_min_i(val));
       }
       if (Sh::fmx(p, v)) {
-        uint64_t* m = (uint64_t*)(base + d.po_max * T) + tid;
+        uint64_t* m = (uint64_t*)(base + Sh::po_max(p, v) * T) + tid;
         *m = max(*m, enc_max_i(val));
       }
     }
@@ -559,9 +618,9 @@ __device__ __forceinline__ void warp_miss_update(const Plan& p, MissStage<NV, F6
 }
 
 // ------------------------------------------------------------------ per-row dispatch
-template <class Sh, int NV, bool F64>
+template <class Sh, int NV, bool F64, bool MISS>
 __device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename Sh::Key (&rk)[kRegSlots],
-                                          uint8_t* sm, uint8_t* cta_tab, int tid, MissStage<NV, F64>& stage,
+                                          uint8_t* sm, uint8_t* cta_tab, int tid, MissStage<MISS ? NV : 1, F64>& stage,
                                           const Row<Sh, NV, F64>& x, int64_t r) {
   using Key = typename Sh::Key;
   constexpr int L = kRegSlots;
@@ -583,10 +642,12 @@ __device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename
       go = true;
     } else {
       uint8_t* e = nullptr;
-      if (p.smem_cap && x.fast && !special) e = cta_find_or_insert(cta_tab, (uint32_t)p.smem_cap, p.cta_stride, x.key);
+      if constexpr (Sh::kCta) {
+        if (p.smem_cap && x.fast && !special) e = cta_find_or_insert(cta_tab, (uint32_t)p.smem_cap, p.cta_stride, x.key);
+      }
       if (e) {
         cta_add<Sh, NV, F64>(p, e, x);
-      } else if (x.fast && !special) {
+      } else if (MISS && x.fast && !special) {
         miss = true;                      // warp-aggregated HBM update below
       } else {
         e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x.key, p.status);
@@ -595,7 +656,7 @@ __device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename
     }
   }
   if (go) priv_add<Sh, NV, F64>(p, sm, slot, tid, x);
-  warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);
+  if constexpr (MISS) warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);
 }
 
 }  // namespace ocl
