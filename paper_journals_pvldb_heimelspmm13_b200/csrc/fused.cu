@@ -64,6 +64,42 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
 
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
+  if constexpr (Sh::kStatic) {
+    // Static shapes: 64-row units with a one-unit-ahead software pipeline — the next
+    // unit's loads are in flight while the current unit is evaluated and placed.
+    const int64_t nunits = (p.n + 63) / 64;
+    const int64_t first = (int64_t)blockIdx.x * (T / 32);
+    const int64_t rounds = nunits > first ? (nunits - first + nwarps - 1) / nwarps : 0;
+    auto full = [&](int64_t u) { return p.vec_ok && u < nunits && u * 64 + 64 <= p.n; };
+    RawUnit<Sh> cur, nxt;
+    int64_t t = warp;
+    if (full(t)) load_unit<Sh>(p, t * 64 + 2 * lane, cur);
+    for (int64_t round = 0; round < rounds; ++round) {
+      if (Sh::kCta && p.smem_cap && round > 0 && round % (kCtaFlushRounds * kUnits) == 0) {
+        __syncthreads();
+        for (int i = tid; i < p.smem_cap; i += T) cta_flush_entry(p, cta_tab + (size_t)i * p.cta_stride);
+        __syncthreads();
+      }
+      const int64_t tn = t + nwarps;
+      if (full(tn)) load_unit<Sh>(p, tn * 64 + 2 * lane, nxt);
+      if (t < nunits) {
+        const int64_t r = t * 64 + 2 * lane;
+        Row<Sh, NV, F64> x0, x1;
+        if (full(t)) {
+          eval_unit<Sh, NV, F64>(p, cur, 0, x0);
+          eval_unit<Sh, NV, F64>(p, cur, 1, x1);
+        } else {
+          eval_one<Sh, NV, F64>(p, r, x0);
+          eval_one<Sh, NV, F64>(p, r + 1, x1);
+        }
+        if (p.bitmap_out) emit_bitmap_unit(p, t * 64, lane, x0.q, x1.q);
+        place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+        place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+      }
+      cur = nxt;
+      t = tn;
+    }
+  } else {
   const int64_t ntiles = (p.n + kTileRows - 1) / kTileRows;
   // CTA-uniform round count (the CTA's first warp has the most tiles): the whole CTA
   // meets at the periodic CTA-table flushes
@@ -79,21 +115,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
     if (t >= ntiles) continue;
     const int64_t base = t * kTileRows;
     if (p.vec_ok && base + kTileRows <= p.n) {
-      if constexpr (Sh::kStatic) {
-        RawUnit<Sh> raw[kUnits];
-#pragma unroll
-        for (int u = 0; u < kUnits; ++u) load_unit<Sh>(p, base + 64 * u + 2 * lane, raw[u]);
-#pragma unroll
-        for (int u = 0; u < kUnits; ++u) {
-          const int64_t r = base + 64 * u + 2 * lane;
-          Row<Sh, NV, F64> x0, x1;
-          eval_unit<Sh, NV, F64>(p, raw[u], 0, x0);
-          eval_unit<Sh, NV, F64>(p, raw[u], 1, x1);
-          if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
-          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
-          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
-        }
-      } else {
+      {
         Row<Sh, NV, F64> x[kUnits][2];
 #pragma unroll
         for (int u = 0; u < kUnits; ++u) eval_pair<Sh, NV, F64>(p, base + 64 * u + 2 * lane, x[u][0], x[u][1]);
@@ -117,6 +139,8 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
       }
     }
   }
+
+  }  // dynamic shapes
 
   // ---- flush: warp-reduce the private records -> CTA entry per slot -> HBM table
   __syncthreads();
