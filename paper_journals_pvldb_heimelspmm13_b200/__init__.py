@@ -22,7 +22,7 @@ import os
 import torch
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "_lib", "libocelot_b200.so")
+LIB_PATH = os.environ.get("OCL_LIB_PATH") or os.path.join(_HERE, "_lib", "libocelot_b200.so")
 
 OCL_OK, OCL_ERR_INVALID_ARG, OCL_ERR_UNSUPPORTED, OCL_ERR_CAPACITY, OCL_ERR_OUT_OF_MEMORY, OCL_ERR_CUDA = range(6)
 _DTYPE = {torch.uint8: 1, torch.int32: 2, torch.int64: 3, torch.float64: 4}

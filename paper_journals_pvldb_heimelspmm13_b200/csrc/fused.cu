@@ -33,6 +33,8 @@
 //    (no dtype dispatch, every value column loaded once, narrow keys in 32 bits) — the
 //    B200 stand-in for Ocelot's run-time kernel compilation.
 //    Plans whose shape matches an instantiated StaticShape run the specialised code.
+#include <stdlib.h>
+
 #include "sga_device.cuh"
 
 namespace ocl {
@@ -64,7 +66,7 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
 
   const int64_t warp = (blockIdx.x * (int64_t)T + tid) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * T) >> 5;
-  if constexpr (Sh::kStatic) {
+  if constexpr (Sh::kStatic && OCL_VAR_PIPE) {
     // Static shapes: 64-row units with a one-unit-ahead software pipeline — the next
     // unit's loads are in flight while the current unit is evaluated and placed.
     const int64_t nunits = (p.n + 63) / 64;
@@ -115,7 +117,21 @@ __global__ void __launch_bounds__(kFusedThreads) k_sga(const __grid_constant__ P
     if (t >= ntiles) continue;
     const int64_t base = t * kTileRows;
     if (p.vec_ok && base + kTileRows <= p.n) {
-      {
+      if constexpr (Sh::kStatic) {
+        RawUnit<Sh> raw[kUnits];
+#pragma unroll
+        for (int u = 0; u < kUnits; ++u) load_unit<Sh>(p, base + 64 * u + 2 * lane, raw[u]);
+#pragma unroll
+        for (int u = 0; u < kUnits; ++u) {
+          const int64_t r = base + 64 * u + 2 * lane;
+          Row<Sh, NV, F64> x0, x1;
+          eval_unit<Sh, NV, F64>(p, raw[u], 0, x0);
+          eval_unit<Sh, NV, F64>(p, raw[u], 1, x1);
+          if (p.bitmap_out) emit_bitmap_unit(p, base + 64 * u, lane, x0.q, x1.q);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x0, r);
+          place_row<Sh, NV, F64, MISS>(p, dir, rk, sm, cta_tab, tid, stage, x1, r + 1);
+        }
+      } else {
         Row<Sh, NV, F64> x[kUnits][2];
 #pragma unroll
         for (int u = 0; u < kUnits; ++u) eval_pair<Sh, NV, F64>(p, base + 64 * u + 2 * lane, x[u][0], x[u][1]);
@@ -356,6 +372,10 @@ cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cuda
   *kind = 0;
   if (p.n == 0) return cudaSuccess;
   if (mode == 2) return values_f64 ? launch_glb<true>(p, sms, s) : launch_glb<false>(p, sms, s);
+  if (mode == 0 && p.vec_ok && !p.miss_agg && p.smem_cap == 0 && getenv("OCL_NO_SPEC") == nullptr) {
+    cudaError_t err = cudaSuccess;
+    if (launch_fused_spec(p, sms, s, &err, kind)) return err;
+  }
   if (mode == 0 && p.vec_ok) {
     if (shape_match<ShQ1I>(p)) {
       *kind = 1;

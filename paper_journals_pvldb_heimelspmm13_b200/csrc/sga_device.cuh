@@ -4,6 +4,13 @@
 // accumulation tiers.  See fused.cu for the design notes and paper citations.
 #pragma once
 
+#ifndef OCL_VAR_FITS
+#define OCL_VAR_FITS 0
+#endif
+#ifndef OCL_VAR_PIPE
+#define OCL_VAR_PIPE 1
+#endif
+
 #include <type_traits>
 
 #include "launch.cuh"
@@ -34,6 +41,8 @@ struct DynShape {
   __device__ static bool pf64(const Plan& p, int i) { return p.preds[i].is_f64; }
   __device__ static int nk(const Plan& p) { return p.nkeys; }
   __device__ static int kw(const Plan& p, int i) { return p.keys[i].col.width; }
+  __device__ static uint64_t kmask(const Plan& p, int i) { return p.keys[i].mask; }
+  __device__ static int kshift(const Plan& p, int i) { return p.keys[i].shift; }
   __device__ static int nv(const Plan& p) { return p.nvals; }
   __device__ static int kind(const Plan& p, int v) { return p.vals[v].expr; }
   __device__ static bool fsum(const Plan& p, int v) { return p.vals[v].off_sum >= 0; }
@@ -72,6 +81,10 @@ struct StaticShape {
   __host__ __device__ static constexpr bool pf64(const Plan&, int) { return PF64; }
   __host__ __device__ static constexpr int nk(const Plan&) { return (K0W > 0) + (K1W > 0); }
   __host__ __device__ static constexpr int kw(const Plan&, int i) { return i == 0 ? K0W : K1W; }
+  __host__ __device__ static constexpr uint64_t kmask(const Plan&, int i) {
+    return (i == 0 ? K0W : K1W) >= 8 ? ~0ULL : ((1ULL << (8 * (i == 0 ? K0W : K1W))) - 1);
+  }
+  __host__ __device__ static constexpr int kshift(const Plan&, int i) { return i == 0 ? 8 * K1W : 0; }
   __host__ __device__ static constexpr int nv(const Plan&) { return NVS; }
   __host__ __device__ static constexpr int kind(const Plan&, int v) { return (int)(op(v) & 3); }
   __host__ __device__ static constexpr int ia(int v) { return (int)((op(v) >> 2) & 7); }
@@ -209,15 +222,27 @@ __device__ __forceinline__ void value_of(const Plan& p, int v, uint64_t ra, uint
   } else {
     const int64_t a = (int64_t)ra;
     if (kind == OCL_EXPR_COL) {
+#if OCL_VAR_FITS
+      x.fast = x.fast && fits_i32(a);
+#else
       x.bad |= i32_bad(a);
+#endif
       x.vi[v] = a;
     } else {
       const int64_t t = (int64_t)((uint64_t)d.S - rb);
+#if OCL_VAR_FITS
+      x.fast = x.fast && fits_i32(a) && fits_i32(t);
+#else
       x.bad |= i32_bad(a) | i32_bad(t);
+#endif
       int64_t e = mul_wide_s32((int32_t)a, (int32_t)t);
       if (kind == OCL_EXPR_MUL_1MINUS_1PLUS) {
         const int64_t u = (int64_t)((uint64_t)d.S + rc);
+#if OCL_VAR_FITS
+        x.fast = x.fast && fits_i32(e) && fits_i32(u);
+#else
         x.bad |= i32_bad(e) | i32_bad(u);
+#endif
         e = mul_wide_s32((int32_t)e, (int32_t)u);
       }
       x.vi[v] = e;
@@ -231,7 +256,7 @@ __device__ __forceinline__ typename Sh::Key pack_key(const Plan& p, const uint64
 #pragma unroll
   for (int i = 0; i < kMaxKeys; ++i) {
     if (i >= Sh::nk(p)) break;
-    k |= (typename Sh::Key)((raw[i] & p.keys[i].mask) << p.keys[i].shift);
+    k |= (typename Sh::Key)((raw[i] & Sh::kmask(p, i)) << Sh::kshift(p, i));
   }
   return k;
 }
@@ -327,7 +352,7 @@ __device__ __forceinline__ void eval_unit(const Plan& p, const RawUnit<Sh>& u, i
     x.key = pack_key<Sh>(p, kk);
 #pragma unroll
     for (int v = 0; v < NV; ++v) value_of<Sh, NV, F64>(p, v, u.c[k][Sh::ia(v)], u.c[k][Sh::ib(v)], u.c[k][Sh::ic(v)], x);
-    x.fast = x.bad == 0;
+    x.fast = x.fast && x.bad == 0;
   }
 }
 

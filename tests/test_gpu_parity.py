@@ -369,3 +369,15 @@ def test_device_generator_matches_host():
     sd = datagen.sweep_device(n, 7, 1 << 12, s=1.5, f64=True)
     for f in sh:
         assert np.array_equal(sd[f].cpu().numpy(), sh[f]), f
+
+
+def test_fused_q1_unified_static_shape(monkeypatch):
+    """The unified kernel's static Q1 shape (OCL_NO_SPEC=1 bypasses the hand-specialised Q1 kernel)."""
+    monkeypatch.setenv("OCL_NO_SPEC", "1")
+    for n in (1000, 300001):
+        li = _lineitem(n, datagen.BASE_SEED + 1)
+        p, k, v, a = _q1(li)
+        _check_sga(p, k, v, a, tier=1, order_by_key=True, bitmap=True)
+        lf = _lineitem(n, datagen.BASE_SEED + 2, f64=True)
+        p, k, v, a = _q1(lf, f64=True)
+        _check_sga(p, k, v, a, tier=1)
