@@ -288,6 +288,7 @@ def main():
     clk.window(h0, h1)
     clk.stop()
     ocl.set_kernel_events(ctx, None, None)
+    kernel_name = ocl.last_kernel(ctx)
     launches = ocl.launch_count() - launches0
     if world > 1:
         dist.barrier()
@@ -369,8 +370,7 @@ def main():
                        "l2": f"inputs {bpr * length / 1e9:.1f} GB per GPU >> 126 MB L2, no flush needed"
                              if bpr * length > 2e9 else "inputs smaller than L2: L2-resident"},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
-                         "traffic": profiled_traffic(args.workload, length), "kernel": "ocl::k_sga_reg (fused)" if
-                         (args.tier == 1 or (args.tier == 0 and eg <= 4)) else "ocl::k_sga_glb (fused)",
+                         "traffic": profiled_traffic(args.workload, length), "kernel": "ocl::" + kernel_name,
                          "kernel_ms": kms, "algorithmic_bytes_per_launch": algo_bytes, "peak_source": peak_src},
             "hbm_frac_step": algo_bytes / (ms / 1e3) / 1e9 / peak,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clk.summary(),

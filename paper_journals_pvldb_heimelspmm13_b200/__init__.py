@@ -108,6 +108,8 @@ def lib():
         L.ocl_last_error.restype = ctypes.c_char_p
         L.ocl_version.restype = ctypes.c_int32
         L.ocl_launch_count.restype = ctypes.c_uint64
+        L.ocl_ctx_last_kernel.argtypes = [P]
+        L.ocl_ctx_last_kernel.restype = ctypes.c_char_p
         L.ocl_ctx_set_kernel_events.argtypes = [P, P, P]
         L.ocl_ctx_set_kernel_events.restype = ctypes.c_int
         _lib = L
@@ -115,7 +117,7 @@ def lib():
 
 
 ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_last_error", "ocl_version",
-               "ocl_launch_count", "ocl_ctx_set_kernel_events",
+               "ocl_launch_count", "ocl_ctx_last_kernel", "ocl_ctx_set_kernel_events",
                "ocl_select_bitmap", "ocl_bitmap_combine", "ocl_prefix_compact_workspace_size", "ocl_prefix_compact",
                "ocl_gather", "ocl_group_build_workspace_size", "ocl_group_build",
                "ocl_group_aggregate_workspace_size", "ocl_group_aggregate",
@@ -152,6 +154,11 @@ _ctxs = {}
 def launch_count():
     """Kernels launched by the library so far (process-wide)."""
     return int(lib().ocl_launch_count())
+
+
+def last_kernel(ctx):
+    """Name of the fused kernel instantiation the last fused call on ctx used."""
+    return lib().ocl_ctx_last_kernel(ctx.handle).decode()
 
 
 def set_kernel_events(ctx, begin=None, end=None):

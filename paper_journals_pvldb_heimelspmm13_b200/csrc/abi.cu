@@ -419,6 +419,8 @@ int32_t ocl_version(void) { return 1; }
 
 uint64_t ocl_launch_count(void) { return g_launches.load(); }
 
+const char* ocl_ctx_last_kernel(ocl_ctx* ctx) { return ctx ? fused_kernel_name(ctx->last_kernel) : ""; }
+
 ocl_status ocl_ctx_set_kernel_events(ocl_ctx* ctx, void* begin_event, void* end_event) {
   if (!ctx) return fail(OCL_ERR_INVALID_ARG, "NULL ctx");
   ctx->prof_begin = (cudaEvent_t)begin_event;

@@ -26,31 +26,39 @@ namespace ocl {
 
 constexpr size_t kAggSmemBudget = 160 * 1024;
 
-template <int NV, bool F64>
-__device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<DynShape, NV, F64>& x) {
+template <class Sh, int NV, bool F64>
+__device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<Sh, NV, F64>& x) {
   x.q = true;
   x.fast = true;
   x.bad = 0;
-  x.key = (uint64_t)(uint32_t)g;
+  x.key = (typename Sh::Key)(uint32_t)g;
+  if constexpr (Sh::kStatic) {
+    uint64_t c[Sh::NC];                   // each distinct value column gathered once
 #pragma unroll
-  for (int v = 0; v < NV; ++v) {
-    if (v >= p.nvals) break;
-    const DevValue& d = p.vals[v];
-    if (!F64 && d.is_f64) {
-      x.fast = false;
-      continue;
+    for (int i = 0; i < Sh::NC; ++i) c[i] = (uint64_t)__ldg((const long long*)p.vcols[i].ptr + r);
+#pragma unroll
+    for (int v = 0; v < NV; ++v) value_of<Sh, NV, F64>(p, v, c[Sh::ia(v)], c[Sh::ib(v)], c[Sh::ic(v)], x);
+  } else {
+#pragma unroll
+    for (int v = 0; v < NV; ++v) {
+      if (v >= p.nvals) break;
+      const DevValue& d = p.vals[v];
+      if (!F64 && d.is_f64) {
+        x.fast = false;
+        continue;
+      }
+      const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
+      const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
+      const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
+      value_of<Sh, NV, F64>(p, v, a, b, c, x);
     }
-    const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
-    const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
-    const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
-    value_of<DynShape, NV, F64>(p, v, a, b, c, x);
   }
   x.fast = x.fast && x.bad == 0;
 }
 
 // Group g goes to the private records when g < npriv, else to the CTA array when
 // g < ncta (integer COL values), else to the warp-aggregated HBM update.
-template <int NV, bool F64>
+template <class Sh, int NV, bool F64>
 __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_constant__ Plan p, int64_t max_rows,
                                                                    const int64_t* ngroups_dev, int64_t max_groups,
                                                                    int32_t npriv, int32_t ncta) {
@@ -82,12 +90,12 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
       __syncthreads();
     }
     const int64_t j = round * per_round + (int64_t)blockIdx.x * T + tid;
-    Row<DynShape, NV, F64> x;
+    Row<Sh, NV, F64> x;
     const int32_t g = j < m ? __ldg(p.gids + j) : -1;
     const bool valid = g >= 0 && g < G;
     const int64_t r = valid ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : 0;
     if (valid) {
-      agg_eval<NV, F64>(p, r, g, x);
+      agg_eval<Sh, NV, F64>(p, r, g, x);
     } else {
       x.q = false;
       x.fast = true;
@@ -97,18 +105,18 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
     bool miss = false;
     if (valid) {
       if (!x.fast) update_entry_slow(p, p.table + (int64_t)g * p.stride, r);
-      else if (g < np_) priv_add<DynShape, NV, F64>(p, sm, g, tid, x);
-      else if (g < nc_) cta_add<DynShape, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
+      else if (g < np_) priv_add<Sh, NV, F64>(p, sm, g, tid, x);
+      else if (g < nc_) cta_add<Sh, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
       else miss = true;
     }
-    warp_miss_update<DynShape, NV, F64>(p, stage, miss, x, tid & 31);   // (always on: G may exceed the tiers)
+    warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);   // (always on: G may exceed the tiers)
   }
   __syncthreads();
   for (int64_t g = 0; g < np_; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);
   for (int64_t g = np_ + tid; g < nc_; g += T) cta_flush_entry(p, cta + g * p.cta_stride, g);
 }
 
-template <int NV, bool F64>
+template <class Sh, int NV, bool F64>
 static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
                                  int sms, cudaStream_t s) {
   // private records for the first groups (up to 96 KB), then a CTA array for integer COL plans
@@ -120,7 +128,7 @@ static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t*
     ncta = std::min<int64_t>(max_groups, npriv + (int64_t)((kAggSmemBudget - (size_t)npriv * p.priv_rec * kFusedThreads) /
                                                             (size_t)p.cta_stride));
   const size_t smem = (size_t)npriv * p.priv_rec * kFusedThreads + (size_t)ncta * p.cta_stride;
-  auto fn = k_group_aggregate<NV, F64>;
+  auto fn = k_group_aggregate<Sh, NV, F64>;
   cudaError_t e = cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
   if (e != cudaSuccess) return e;
   int nb = 0;
@@ -133,13 +141,24 @@ static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t*
   return cudaGetLastError();
 }
 
+// Static value shapes of the grouped aggregation: the TPC-H Q1 value set (int64 and
+// fp64 decimals) and COUNT/SUM/MIN/MAX of one int64 column.
+using AgQ1I = StaticShape<0, false, 0, 0, 4, false, vop(0, VF_SUM, 0), vop(0, VF_SUM, 1), vop(1, VF_SUM, 1, 2),
+                          vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
+using AgQ1F = StaticShape<0, false, 0, 0, 4, true, vop(0, VF_SUM, 0), vop(0, VF_SUM, 1), vop(1, VF_SUM, 1, 2),
+                          vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
+using AgV1 = StaticShape<0, false, 0, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+
 template <bool F64>
 static cudaError_t launch_agg_f(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
                                 int sms, cudaStream_t s) {
-  if (p.nvals <= 1) return launch_agg_nv<1, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
-  if (p.nvals <= 2) return launch_agg_nv<2, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
-  if (p.nvals <= 4) return launch_agg_nv<4, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
-  return launch_agg_nv<6, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (!F64 && values_match<AgQ1I>(p)) return launch_agg_nv<AgQ1I, 5, false>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (F64 && values_match<AgQ1F>(p)) return launch_agg_nv<AgQ1F, 5, true>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (!F64 && values_match<AgV1>(p)) return launch_agg_nv<AgV1, 1, false>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (p.nvals <= 1) return launch_agg_nv<DynShape, 1, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (p.nvals <= 2) return launch_agg_nv<DynShape, 2, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  if (p.nvals <= 4) return launch_agg_nv<DynShape, 4, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
+  return launch_agg_nv<DynShape, 6, F64>(p, max_rows, ngroups_dev, max_groups, sms, s);
 }
 
 cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,

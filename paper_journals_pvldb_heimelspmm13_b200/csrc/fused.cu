@@ -289,28 +289,12 @@ using ShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | 
 
 template <class Sh>
 static bool shape_match(const Plan& g) {
-  if (g.npreds != Sh::np(g) || g.nkeys != Sh::nk(g) || g.nvals != Sh::nv(g)) return false;
+  if (g.npreds != Sh::np(g) || g.nkeys != Sh::nk(g)) return false;
   for (int i = 0; i < g.npreds; ++i)
     if (g.preds[i].col.width != Sh::pw(g, i) || (bool)g.preds[i].is_f64 != Sh::pf64(g, i)) return false;
   for (int i = 0; i < g.nkeys; ++i)
     if (g.keys[i].col.width != Sh::kw(g, i)) return false;
-  if (g.ncols != Sh::NC || g.priv_rec != Sh::rec(g)) return false;
-  for (int i = 0; i < g.ncols; ++i)
-    if (g.vcols[i].width != 8 || (g.vcols[i].dtype == OCL_F64) != Sh::vf64(g, 0)) return false;
-  for (int v = 0; v < g.nvals; ++v) {
-    const DevValue& d = g.vals[v];
-    if (d.expr != Sh::kind(g, v) || (bool)d.is_f64 != Sh::vf64(g, v)) return false;
-    if ((d.off_sum >= 0) != Sh::fsum(g, v) || (d.off_min >= 0) != Sh::fmn(g, v) ||
-        (d.off_max >= 0) != Sh::fmx(g, v))
-      return false;
-    if (d.po_sum != Sh::po_sum(g, v) || d.po_hi != Sh::po_hi(g, v) || d.po_min != Sh::po_min(g, v) ||
-        d.po_max != Sh::po_max(g, v))
-      return false;
-    if (d.ia != Sh::ia(v)) return false;
-    if (d.expr >= OCL_EXPR_MUL_1MINUS && d.ib != Sh::ib(v)) return false;
-    if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS && d.ic != Sh::ic(v)) return false;
-  }
-  return true;
+  return values_match<Sh>(g);
 }
 
 // ------------------------------------------------------------------ dispatch
@@ -371,10 +355,16 @@ int reg_tier_slots() { return kRegSlots; }
 cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind) {
   *kind = 0;
   if (p.n == 0) return cudaSuccess;
-  if (mode == 2) return values_f64 ? launch_glb<true>(p, sms, s) : launch_glb<false>(p, sms, s);
+  if (mode == 2) {
+    *kind = 20;
+    return values_f64 ? launch_glb<true>(p, sms, s) : launch_glb<false>(p, sms, s);
+  }
   if (mode == 0 && p.vec_ok && !p.miss_agg && p.smem_cap == 0 && getenv("OCL_NO_SPEC") == nullptr) {
     cudaError_t err = cudaSuccess;
-    if (launch_fused_spec(p, sms, s, &err, kind)) return err;
+    if (launch_fused_spec(p, sms, s, &err, kind)) {
+      *kind += 10;                       // 11 / 12: Q1-signature kernel (int / fp64)
+      return err;
+    }
   }
   if (mode == 0 && p.vec_ok) {
     if (shape_match<ShQ1I>(p)) {
@@ -395,6 +385,19 @@ cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cuda
     }
   }
   return values_f64 ? launch_dyn<true>(p, sms, s) : launch_dyn<false>(p, sms, s);
+}
+
+const char* fused_kernel_name(int kind) {
+  switch (kind) {
+    case 1: return "k_sga<StaticShape Q1 int64>";
+    case 2: return "k_sga<StaticShape Q1 fp64>";
+    case 3: return "k_sga<StaticShape key i64, COUNT/SUM/MIN/MAX>";
+    case 4: return "k_sga<StaticShape pred i32, key i64, COUNT/SUM/MIN/MAX>";
+    case 11: return "k_sga_priv<Sig Q1 int64>";
+    case 12: return "k_sga_priv<Sig Q1 fp64>";
+    case 20: return "k_sga_glb<DynShape>";
+    default: return "k_sga<DynShape>";
+  }
 }
 
 }  // namespace ocl

@@ -57,6 +57,7 @@ cudaError_t launch_group_aggregate(const Plan& p, int64_t max_rows, const int64_
 // matches the plan, else dynamic; 1: dynamic shape only; 2: HBM-only kernel.
 cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind);
 int reg_tier_slots();
+const char* fused_kernel_name(int kind);
 // Proven few-group Q1 kernel (fused_spec.cu) used while the unified kernel is tuned.
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 }  // namespace ocl

@@ -684,4 +684,28 @@ __device__ __forceinline__ void place_row(const Plan& p, uint64_t* dir, typename
   if constexpr (MISS) warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);
 }
 
+// ------------------------------------------------------------------ static-shape matching (host)
+// The value part of a plan (distinct 8-byte value columns, expressions, accumulator
+// flags, private-record layout) equals the compile-time shape Sh.
+template <class Sh>
+inline bool values_match(const Plan& g) {
+  if (g.nvals != Sh::nv(g) || g.ncols != Sh::NC || g.priv_rec != Sh::rec(g)) return false;
+  for (int i = 0; i < g.ncols; ++i)
+    if (g.vcols[i].width != 8 || (g.vcols[i].dtype == OCL_F64) != Sh::vf64(g, 0)) return false;
+  for (int v = 0; v < g.nvals; ++v) {
+    const DevValue& d = g.vals[v];
+    if (d.expr != Sh::kind(g, v) || (bool)d.is_f64 != Sh::vf64(g, v)) return false;
+    if ((d.off_sum >= 0) != Sh::fsum(g, v) || (d.off_min >= 0) != Sh::fmn(g, v) ||
+        (d.off_max >= 0) != Sh::fmx(g, v))
+      return false;
+    if (d.po_sum != Sh::po_sum(g, v) || d.po_hi != Sh::po_hi(g, v) || d.po_min != Sh::po_min(g, v) ||
+        d.po_max != Sh::po_max(g, v))
+      return false;
+    if (d.ia != Sh::ia(v)) return false;
+    if (d.expr >= OCL_EXPR_MUL_1MINUS && d.ib != Sh::ib(v)) return false;
+    if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS && d.ic != Sh::ic(v)) return false;
+  }
+  return true;
+}
+
 }  // namespace ocl
