@@ -581,16 +581,9 @@ ocl_status ocl_group_build(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, 
   p.n = max_rows;
   OCL_CUDA(cudaMemsetAsync(ws, 0, tbytes, st), "table init");
   if (dev_status) OCL_CUDA(cudaMemsetAsync(dev_status, 0, 4, st), "status init");
-  OCL_CUDA(launch_group_insert(p, gid_out, max_rows, ctx->grid, st), "group insert");
-  EmitArgs ea;
-  memset(&ea, 0, sizeof(ea));
-  ea.kind = EMIT_GROUP_IDS;
-  ea.keys_out = keys_out;
-  ea.out_capacity = keys_out ? out_capacity : INT64_MAX;
-  ea.status = dev_status;
-  OCL_CUDA(launch_emit(p.table, cap, 16, ea, ngroups_out, keys_out ? out_capacity : INT64_MAX, dev_status, false,
-                       (uint8_t*)ws + tbytes, ctx->grid, st), "group emit");
-  OCL_CUDA(launch_group_lookup(p.table, 16, m_dev, max_rows, gid_out, ctx->grid, st), "group lookup");
+  OCL_CUDA(cudaMemsetAsync(ngroups_out, 0, 8, st), "group count init");
+  OCL_CUDA(launch_group_build(p, gid_out, max_rows, ngroups_out, keys_out, keys_out ? out_capacity : INT64_MAX,
+                              ctx->grid, st), "group build");
   return OCL_OK;
 }
 

@@ -26,16 +26,16 @@ namespace ocl {
 
 constexpr size_t kAggSmemBudget = 160 * 1024;
 
+// Static shapes: the NC distinct value columns of row r were gathered into c[] by the
+// caller (all loads of a thread's R rows are issued before any update).
 template <class Sh, int NV, bool F64>
-__device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Row<Sh, NV, F64>& x) {
+__device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, const uint64_t* c,
+                                         Row<Sh, NV, F64>& x) {
   x.q = true;
   x.fast = true;
   x.bad = 0;
   x.key = (typename Sh::Key)(uint32_t)g;
   if constexpr (Sh::kStatic) {
-    uint64_t c[Sh::NC];                   // each distinct value column gathered once
-#pragma unroll
-    for (int i = 0; i < Sh::NC; ++i) c[i] = (uint64_t)__ldg((const long long*)p.vcols[i].ptr + r);
 #pragma unroll
     for (int v = 0; v < NV; ++v) value_of<Sh, NV, F64>(p, v, c[Sh::ia(v)], c[Sh::ib(v)], c[Sh::ic(v)], x);
   } else {
@@ -49,8 +49,8 @@ __device__ __forceinline__ void agg_eval(const Plan& p, int64_t r, int32_t g, Ro
       }
       const uint64_t a = ld1w(d.a.width, d.a.ptr, r);
       const uint64_t b = d.expr >= OCL_EXPR_MUL_1MINUS ? ld1w(d.b.width, d.b.ptr, r) : 0;
-      const uint64_t c = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
-      value_of<Sh, NV, F64>(p, v, a, b, c, x);
+      const uint64_t cc = d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS ? ld1w(d.c.width, d.c.ptr, r) : 0;
+      value_of<Sh, NV, F64>(p, v, a, b, cc, x);
     }
   }
   x.fast = x.fast && x.bad == 0;
@@ -81,35 +81,61 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
     __syncthreads();
   }
   MissStage<NV, F64>& stage = stages[tid >> 5];
-  const int64_t per_round = (int64_t)gridDim.x * T;
+  // R rows per thread per round: every gid/oid/value load of the R rows is in flight
+  // before the first update (the value loads depend on the oid loads: memory-level
+  // parallelism, not bandwidth, bounds a one-row-at-a-time gather).
+  constexpr int R = Sh::kStatic ? 4 : 1;
+  constexpr int NCc = Sh::kStatic ? Sh::NC : 1;
+  constexpr int64_t kFlushRounds = 256 / R;                   // 2^16 rows per CTA between CTA-tier flushes
+  const int64_t per_round = (int64_t)gridDim.x * T * R;
   const int64_t rounds = (m + per_round - 1) / per_round;    // uniform across the grid
   for (int64_t round = 0; round < rounds; ++round) {
-    if (nc_ > np_ && round > 0 && round % 256 == 0) {          // 256 rounds x 256 threads = 2^16 rows per CTA
+    if (nc_ > np_ && round > 0 && round % kFlushRounds == 0) {
       __syncthreads();
       for (int64_t g = np_ + tid; g < nc_; g += T) cta_flush_entry(p, cta + g * p.cta_stride, g);
       __syncthreads();
     }
-    const int64_t j = round * per_round + (int64_t)blockIdx.x * T + tid;
-    Row<Sh, NV, F64> x;
-    const int32_t g = j < m ? __ldg(p.gids + j) : -1;
-    const bool valid = g >= 0 && g < G;
-    const int64_t r = valid ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : 0;
-    if (valid) {
-      agg_eval<Sh, NV, F64>(p, r, g, x);
-    } else {
-      x.q = false;
-      x.fast = true;
-      x.bad = 0;
-      x.key = 0;
+    const int64_t base = round * per_round + (int64_t)blockIdx.x * T * R + tid;
+    int32_t gk[R];
+    int64_t rk[R];
+    uint64_t c[R][NCc];
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      const int64_t j = base + (int64_t)k * T;
+      gk[k] = j < m ? __ldg(p.gids + j) : -1;
+      if (gk[k] >= G) gk[k] = -1;
+      rk[k] = gk[k] >= 0 ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : 0;
     }
-    bool miss = false;
-    if (valid) {
-      if (!x.fast) update_entry_slow(p, p.table + (int64_t)g * p.stride, r);
-      else if (g < np_) priv_add<Sh, NV, F64>(p, sm, g, tid, x);
-      else if (g < nc_) cta_add<Sh, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
-      else miss = true;
+    if constexpr (Sh::kStatic) {
+#pragma unroll
+      for (int k = 0; k < R; ++k)
+#pragma unroll
+        for (int i = 0; i < NCc; ++i)
+          c[k][i] = gk[k] >= 0 ? (uint64_t)__ldg((const long long*)p.vcols[i].ptr + rk[k]) : 0;
     }
-    warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);   // (always on: G may exceed the tiers)
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      const int32_t g = gk[k];
+      const int64_t r = rk[k];
+      const bool valid = g >= 0;
+      Row<Sh, NV, F64> x;
+      if (valid) {
+        agg_eval<Sh, NV, F64>(p, r, g, c[k], x);
+      } else {
+        x.q = false;
+        x.fast = true;
+        x.bad = 0;
+        x.key = 0;
+      }
+      bool miss = false;
+      if (valid) {
+        if (!x.fast) update_entry_slow(p, p.table + (int64_t)g * p.stride, r);
+        else if (g < np_) priv_add<Sh, NV, F64>(p, sm, g, tid, x);
+        else if (g < nc_) cta_add<Sh, NV, F64>(p, cta + (int64_t)g * p.cta_stride, x);
+        else miss = true;
+      }
+      warp_miss_update<Sh, NV, F64>(p, stage, miss, x, tid & 31);   // (always on: G may exceed the tiers)
+    }
   }
   __syncthreads();
   for (int64_t g = 0; g < np_; ++g) priv_flush_warp(p, sm + (size_t)g * p.priv_rec * T, tid, p.table + g * p.stride);
@@ -119,8 +145,9 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
 template <class Sh, int NV, bool F64>
 static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t* ngroups_dev, int64_t max_groups,
                                  int sms, cudaStream_t s) {
-  // private records for the first groups (up to 96 KB), then a CTA array for integer COL plans
-  int64_t npriv = std::min<int64_t>(max_groups, (int64_t)(96 * 1024 / ((size_t)p.priv_rec * kFusedThreads)));
+  // private records for the first groups (up to 64 KB: three CTAs per SM), then a CTA
+  // array for integer COL plans
+  int64_t npriv = std::min<int64_t>(max_groups, (int64_t)(64 * 1024 / ((size_t)p.priv_rec * kFusedThreads)));
   bool int_cols = true;
   for (int v = 0; v < p.nvals; ++v) int_cols = int_cols && !p.vals[v].is_f64 && p.vals[v].expr == OCL_EXPR_COL;
   int64_t ncta = npriv;
@@ -134,7 +161,7 @@ static cudaError_t launch_agg_nv(const Plan& p, int64_t max_rows, const int64_t*
   int nb = 0;
   if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, kFusedThreads, smem) != cudaSuccess || nb < 1) nb = 1;
   int64_t grid = (int64_t)sms * nb;
-  const int64_t need = (max_rows + kFusedThreads - 1) / kFusedThreads;
+  const int64_t need = (max_rows + kFusedThreads * 4 - 1) / (kFusedThreads * 4);
   if (need < grid) grid = need > 0 ? need : 1;
   count_launch();
   fn<<<(int)grid, kFusedThreads, smem, s>>>(p, max_rows, ngroups_dev, max_groups, (int32_t)npriv, (int32_t)ncta);

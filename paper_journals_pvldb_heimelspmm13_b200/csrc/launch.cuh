@@ -29,7 +29,7 @@ struct EmitArgs {
   uint8_t* partial_out;
   int32_t* status;
 };
-enum EmitKind : int32_t { EMIT_FINAL = 0, EMIT_GROUP_IDS = 1, EMIT_PARTIAL = 2 };
+enum EmitKind : int32_t { EMIT_FINAL = 0, EMIT_PARTIAL = 2 };
 
 cudaError_t launch_select_bitmap(const SelParams& p, int grid, cudaStream_t s);
 cudaError_t launch_bitmap_combine(int op, const uint32_t* a, const uint32_t* b, uint32_t* out, int64_t n, int grid,
@@ -43,9 +43,8 @@ cudaError_t launch_emit(uint8_t* table, uint64_t cap, int32_t stride, const Emit
 bool sorted_emit_supported(uint64_t cap);
 cudaError_t launch_finalize_dense(const uint8_t* table, int32_t stride, const int64_t* ngroups, int64_t max_groups,
                                   const FinPlan& f, int grid, cudaStream_t s);
-cudaError_t launch_group_insert(const Plan& p, int32_t* gid_out, int64_t max_rows, int grid, cudaStream_t s);
-cudaError_t launch_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
-                                int32_t* gid_out, int grid, cudaStream_t s);
+cudaError_t launch_group_build(const Plan& p, int32_t* gid_out, int64_t max_rows, int64_t* ngroups,
+                               int64_t* keys_out, int64_t out_capacity, int grid, cudaStream_t s);
 cudaError_t launch_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
                           void* out, int grid, cudaStream_t s);
 cudaError_t launch_merge_partials(const uint8_t* partials, int32_t nparts, int64_t part_capacity,

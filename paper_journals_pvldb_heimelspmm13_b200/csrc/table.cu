@@ -59,9 +59,6 @@ __device__ __forceinline__ void emit_final(const FinPlan& f, const uint8_t* e, u
 __device__ __forceinline__ void emit_slot(const EmitArgs& a, uint8_t* e, uint64_t key, int64_t g, int32_t stride) {
   if (a.kind == EMIT_FINAL) {
     emit_final(a.fin, e, key, g);
-  } else if (a.kind == EMIT_GROUP_IDS) {
-    *(int64_t*)(e + 8) = g;                         // slot -> dense gid (read by k_group_lookup)
-    if (g < a.out_capacity && a.keys_out) a.keys_out[g] = (int64_t)key;
   } else if (g < a.out_capacity) {
     uint64_t* dst = (uint64_t*)(a.partial_out + g * (int64_t)stride);
     const uint64_t* src = (const uint64_t*)e;
@@ -209,20 +206,72 @@ __global__ void k_finalize_dense(const uint8_t* table, int32_t stride, const int
 }
 
 // ------------------------------------------------------------------ group build (K6/K7)
-// Group build (K6): per row, the packed key's table slot.  A CTA-level direct-mapped
-// cache in shared memory (key -> slot, 256 lines, filled first-come) answers repeated
-// keys without touching HBM — for few groups every row after warm-up; misses probe
-// the HBM table once per distinct key per warp (__match_any_sync) with atomicCAS.
+// Group build in one pass (K6+K7): the CTA that claims a key's table slot
+// (atomicCAS on the empty key field) also assigns its dense group id from a global
+// counter (one atomicAdd per warp for all keys the warp claims) and publishes it in
+// the entry's payload word as gid+1; a row that finds the key already claimed reads
+// the id from there (spinning the few cycles until the claimer has written it).  A
+// CTA-level direct-mapped cache in shared memory (key -> gid, 256 lines, filled
+// first-come) answers repeated keys without touching HBM — for few groups every row
+// after warm-up; misses probe the HBM table once per distinct key per warp
+// (__match_any_sync).  Ids are dense in [0, G), order unspecified (s4).
 constexpr int kGroupCache = 256;
 
-__global__ void __launch_bounds__(256) k_group_insert(const __grid_constant__ Plan p, int32_t* gid_out,
-                                                      int64_t max_rows) {
+template <int W>
+__device__ __forceinline__ uint64_t ld_key(const void* p, int64_t r) {   // raw bits, zero-extended
+  if constexpr (W == 1) return (uint64_t)__ldg((const uint8_t*)p + r);
+  else if constexpr (W == 4) return (uint64_t)(uint32_t)__ldg((const int32_t*)p + r);
+  else return (uint64_t)__ldg((const unsigned long long*)p + r);
+}
+
+// Packed key (s5) of row r; W0/W1 = key column widths known at compile time, or 0
+// for the runtime-described plan.
+template <int W0, int W1>
+__device__ __forceinline__ uint64_t group_key(const Plan& p, int64_t r) {
+  if constexpr (W0 == 0) return row_key_scalar(p, r);
+  else if constexpr (W1 == 0) return ld_key<W0>(p.keys[0].col.ptr, r);
+  else return ld_key<W0>(p.keys[0].col.ptr, r) << (8 * W1) | ld_key<W1>(p.keys[1].col.ptr, r);
+}
+
+// Slot of key in the table, claiming an empty one; *won = this call claimed it.
+__device__ __forceinline__ uint64_t* table_claim(uint8_t* table, uint64_t mask, uint64_t key, int32_t* status,
+                                                 bool* won) {
+  *won = false;
+  if (key == ~0ULL) {   // side entry: the key field is an occupancy flag
+    uint64_t* e = (uint64_t*)(table + (mask + 1) * 16);
+    if (ld_relaxed_u64(e) == 0) *won = atomicCAS((unsigned long long*)e, 0ULL, 1ULL) == 0ULL;
+    return e;
+  }
+  const uint64_t sk = ~key;
+  uint64_t h = fmix64(key) & mask;
+  for (uint64_t probe = 0; probe <= mask; ++probe) {
+    uint64_t* kp = (uint64_t*)(table + h * 16);
+    uint64_t cur = ld_relaxed_u64(kp);
+    if (cur == sk) return kp;
+    if (cur == 0) {
+      cur = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
+      if (cur == 0) {
+        *won = true;
+        return kp;
+      }
+      if (cur == sk) return kp;
+    }
+    h = (h + 1) & mask;
+  }
+  set_status(status, OCL_ERR_CAPACITY);
+  return nullptr;
+}
+
+template <int W0, int W1>
+__global__ void __launch_bounds__(256) k_group_build(const __grid_constant__ Plan p, int32_t* gid_out,
+                                                     int64_t max_rows, int64_t* ngroups, int64_t* keys_out,
+                                                     int64_t out_capacity) {
   constexpr int R = 4;                     // rows per thread per iteration (independent gathers in flight)
   __shared__ unsigned long long ck[kGroupCache];
-  __shared__ unsigned int cs[kGroupCache];
+  __shared__ int32_t cs[kGroupCache];
   for (int i = threadIdx.x; i < kGroupCache; i += blockDim.x) {
     ck[i] = 0;
-    cs[i] = 0xFFFFFFFFu;
+    cs[i] = -1;
   }
   __syncthreads();
   const int lane = threadIdx.x & 31;
@@ -230,47 +279,61 @@ __global__ void __launch_bounds__(256) k_group_insert(const __grid_constant__ Pl
   const int64_t step = (int64_t)gridDim.x * blockDim.x * R;
   for (int64_t j0 = (int64_t)blockIdx.x * blockDim.x * R; j0 < m; j0 += step) {
     uint64_t key[R];
-    int64_t j[R];
+    int64_t r[R];
 #pragma unroll
     for (int k = 0; k < R; ++k) {
-      j[k] = j0 + k * (int64_t)blockDim.x + threadIdx.x;
-      key[k] = 0;
-      if (j[k] < m) key[k] = row_key_scalar(p, p.oids ? (int64_t)__ldg(p.oids + j[k]) : j[k]);
+      const int64_t j = j0 + k * (int64_t)blockDim.x + threadIdx.x;
+      r[k] = j < m ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : -1;
     }
 #pragma unroll
+    for (int k = 0; k < R; ++k) key[k] = r[k] >= 0 ? group_key<W0, W1>(p, r[k]) : 0;
+#pragma unroll
     for (int k = 0; k < R; ++k) {
-      const bool act = j[k] < m;
-      uint32_t slot = 0xFFFFFFFFu;
-      const int h = (int)(fmix64(key[k]) & (kGroupCache - 1));
+      const int64_t j = j0 + k * (int64_t)blockDim.x + threadIdx.x;
+      const bool act = r[k] >= 0;
+      int32_t gid = -1;
+      const int h = (int)((key[k] * 0x9E3779B97F4A7C15ULL) >> 56);   // cache line (multiplicative hash)
       if (act && key[k] != ~0ULL && *(volatile unsigned long long*)&ck[h] == ~key[k])
-        slot = *(volatile unsigned int*)&cs[h];
-      const bool miss = act && slot == 0xFFFFFFFFu;
+        gid = *(volatile int32_t*)&cs[h];
+      const bool miss = act && gid < 0;
       const unsigned mmask = __ballot_sync(0xffffffffu, miss);
       if (miss) {
         const unsigned peers = __match_any_sync(mmask, key[k]);
         const int leader = __ffs(peers) - 1;
-        uint32_t s = 0xFFFFFFFFu;
-        if (lane == leader) {
-          uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
-          if (e) {
-            s = (uint32_t)((e - p.table) / p.stride);
-            if (key[k] != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key[k]) == 0ULL)
-              *(volatile unsigned int*)&cs[h] = s;
-          }
+        bool won = false;
+        uint64_t* e = nullptr;
+        if (lane == leader) e = table_claim(p.table, p.mask, key[k], p.status, &won);
+        const unsigned wm = __ballot_sync(mmask, won);
+        unsigned long long base = 0;
+        if (wm) {
+          const int first = __ffs(wm) - 1;
+          if (lane == first) base = atomicAdd((unsigned long long*)ngroups, (unsigned long long)__popc(wm));
+          base = __shfl_sync(mmask, base, first);
         }
-        slot = __shfl_sync(peers, s, leader);
+        if (lane == leader && e) {
+          int64_t g;
+          if (won) {
+            g = (int64_t)base + __popc(wm & ((1u << lane) - 1));
+            *(volatile uint64_t*)(e + 1) = (uint64_t)g + 1;
+            if (g < out_capacity) {
+              if (keys_out) keys_out[g] = (int64_t)key[k];
+            } else {
+              set_status(p.status, OCL_ERR_CAPACITY);
+            }
+          } else {
+            uint64_t v;
+            while ((v = *(volatile uint64_t*)(e + 1)) == 0) {
+            }
+            g = (int64_t)v - 1;
+          }
+          gid = (int32_t)g;
+          if (key[k] != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key[k]) == 0ULL)
+            *(volatile int32_t*)&cs[h] = gid;
+        }
+        gid = __shfl_sync(peers, gid, leader);
       }
-      if (act) gid_out[j[k]] = (int32_t)slot;   // slot index; remapped to the dense id by k_group_lookup
+      if (act) gid_out[j] = gid;
     }
-  }
-}
-
-__global__ void k_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
-                               int32_t* gid_out) {
-  const int64_t m = m_dev ? *m_dev : max_rows;
-  for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
-    const uint32_t s = (uint32_t)gid_out[j];
-    gid_out[j] = s != 0xFFFFFFFFu ? (int32_t)*(const int64_t*)(table + (int64_t)s * stride + 8) : -1;
   }
 }
 
@@ -358,22 +421,20 @@ cudaError_t launch_finalize_dense(const uint8_t* table, int32_t stride, const in
   return cudaGetLastError();
 }
 
-cudaError_t launch_group_insert(const Plan& p, int32_t* gid_out, int64_t max_rows, int grid, cudaStream_t s) {
+cudaError_t launch_group_build(const Plan& p, int32_t* gid_out, int64_t max_rows, int64_t* ngroups,
+                               int64_t* keys_out, int64_t out_capacity, int grid, cudaStream_t s) {
   if (max_rows == 0) return cudaSuccess;
   int64_t g = (max_rows + 1023) / 1024;
   if (g > grid) g = grid;
+  auto fn = k_group_build<0, 0>;
+  const int w0 = p.keys[0].col.width, w1 = p.nkeys > 1 ? p.keys[1].col.width : 0;
+  if (p.nkeys == 2 && w0 == 1 && w1 == 1) fn = k_group_build<1, 1>;
+  else if (p.nkeys == 2 && w0 == 4 && w1 == 4) fn = k_group_build<4, 4>;
+  else if (p.nkeys == 1 && w0 == 1) fn = k_group_build<1, 0>;
+  else if (p.nkeys == 1 && w0 == 4) fn = k_group_build<4, 0>;
+  else if (p.nkeys == 1 && w0 == 8) fn = k_group_build<8, 0>;
   count_launch();
-  k_group_insert<<<(int)g, 256, 0, s>>>(p, gid_out, max_rows);
-  return cudaGetLastError();
-}
-
-cudaError_t launch_group_lookup(const uint8_t* table, int32_t stride, const int64_t* m_dev, int64_t max_rows,
-                                int32_t* gid_out, int grid, cudaStream_t s) {
-  if (max_rows == 0) return cudaSuccess;
-  int64_t g = (max_rows + 255) / 256;
-  if (g > grid) g = grid;
-  count_launch();
-  k_group_lookup<<<(int)g, 256, 0, s>>>(table, stride, m_dev, max_rows, gid_out);
+  fn<<<(int)g, 256, 0, s>>>(p, gid_out, max_rows, ngroups, keys_out, out_capacity);
   return cudaGetLastError();
 }
 

@@ -100,7 +100,8 @@ def test_gather():
 
 
 # ---------------------------------------------------------------- a4-a6
-@pytest.mark.parametrize("kind,G", [("u8u8", 6), ("i64", 1000), ("i64", 200000), ("i32", 50), ("u8", 256)])
+@pytest.mark.parametrize("kind,G", [("u8u8", 6), ("i64", 1000), ("i64", 200000), ("i32", 50), ("u8", 256),
+                                    ("i32i32", 500), ("u8i32", 300), ("i64neg1", 10)])
 def test_group_build(kind, G):
     rng = np.random.default_rng(G)
     n = 300000
@@ -110,12 +111,18 @@ def test_group_build(kind, G):
         keys = [(rng.integers(0, G, n) * 7919 - 5).astype(np.int64)]
     elif kind == "i32":
         keys = [rng.integers(-G // 2, G // 2, n).astype(np.int32)]
+    elif kind == "i32i32":
+        keys = [rng.integers(-G // 2, G // 2, n).astype(np.int32), rng.integers(-3, 3, n).astype(np.int32)]
+    elif kind == "u8i32":   # mixed widths: the runtime-described key path
+        keys = [rng.integers(0, 3, n).astype(np.uint8), rng.integers(-G // 6, G // 6, n).astype(np.int32)]
+    elif kind == "i64neg1":  # key ~0 (all bits set) lives in the table's side entry
+        keys = [rng.integers(-G // 2, G // 2, n).astype(np.int64)]
     else:
         keys = [rng.integers(0, 256, n).astype(np.uint8)]
     oids = np.flatnonzero(rng.random(n) < 0.7).astype(np.uint32)
     ref_g, ref_k = oracle.group_hash(keys, oids)
     gids, kout, ng, st = ocl.group_build([dev(k) for k in keys], oids=dev(oids.view(np.int32)),
-                                         expected_groups=max(G, 16))
+                                         expected_groups=max(len(ref_k), 16))
     torch.cuda.synchronize()
     assert int(st.item()) == 0
     Gg = int(ng.item())
