@@ -10,8 +10,8 @@
 // every predecessor tile is owned by a running CTA (forward progress).  Per
 // tile: popcounts -> warp/CTA scan -> publish the tile aggregate -> warp 0 looks
 // back over predecessors' {flag|value} words (32 at a time) -> publish the
-// inclusive prefix.  Oids are written warp-round by warp-round through a 4 KB
-// per-warp shared staging buffer so every global store is a coalesced run.
+// inclusive prefix.  Oids are written word by word: the set bits of one word
+// go out as one contiguous (coalesced) run of the warp's lanes.
 #include "launch.cuh"
 
 namespace ocl {
@@ -33,7 +33,6 @@ __device__ __forceinline__ void st_release(uint64_t* p, uint64_t v) {
 __global__ void __launch_bounds__(kCompactWarps * 32)
     k_prefix_compact(const uint32_t* __restrict__ bitmap, int64_t n, uint32_t* __restrict__ oids,
                      int64_t* m_out, unsigned long long* tile_counter, uint64_t* status, int64_t ntiles) {
-  __shared__ uint32_t stage[kCompactWarps][1024];
   __shared__ uint32_t warp_tot[kCompactWarps];
   __shared__ uint64_t sh_tile, sh_excl;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -96,30 +95,20 @@ __global__ void __launch_bounds__(kCompactWarps * 32)
       }
     }
     __syncthreads();
-    // scatter: round by round through the warp's staging buffer
+    // scatter, word by word: for word i the warp's ballot of "bit lane set" is the
+    // word itself, so lane l's rank among the set bits is popc(word & lanemask_lt)
+    // and the warp's set rows leave as one contiguous (coalesced) store run.
     uint64_t out_base = sh_excl + warp_base;
-    uint32_t* buf = stage[warp];
+    const uint32_t lt = (1u << lane) - 1;
 #pragma unroll
     for (int r = 0; r < kCompactRounds; ++r) {
-      uint32_t c = __popc(wd[r]);
-      uint32_t incl = c;
-      for (int o = 1; o < 32; o <<= 1) {
-        uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
-        if (lane >= o) incl += y;
+      const uint32_t row0 = (uint32_t)((w0 + 32 * r) << 5) + lane;
+#pragma unroll 8
+      for (int i = 0; i < 32; ++i) {
+        const uint32_t w = __shfl_sync(0xffffffffu, wd[r], i);
+        if ((w >> lane) & 1u) __stcs(oids + out_base + __popc(w & lt), row0 + 32u * i);
+        out_base += __popc(w);
       }
-      uint32_t round_tot = __shfl_sync(0xffffffffu, incl, 31);
-      uint32_t off = incl - c;
-      uint32_t w = wd[r];
-      const uint32_t row0 = (uint32_t)((w0 + 32 * r + lane) << 5);
-      while (w) {
-        int b = __ffs(w) - 1;
-        buf[off++] = row0 + b;
-        w &= w - 1;
-      }
-      __syncwarp();
-      for (uint32_t i = lane; i < round_tot; i += 32) __stcs(oids + out_base + i, buf[i]);
-      __syncwarp();
-      out_base += round_tot;
     }
     __syncthreads();
   }

@@ -20,6 +20,7 @@ struct SelParams {
   int64_t lo, hi;      // normalised inclusive bounds
   double flo, fhi;
   uint32_t* out;
+  int32_t lo32, hi32;  // bounds clamped to the column's range (empty range: lo32 > hi32); set by the launcher
 };
 struct EmitArgs {
   int32_t kind;

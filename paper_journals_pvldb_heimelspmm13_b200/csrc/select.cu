@@ -21,16 +21,19 @@ template <int W>
 __device__ __forceinline__ uint32_t chunk_bits(const SelParams& p, uint4 v) {
   uint32_t b = 0;
   if constexpr (W == 1) {
-    uint32_t w4[4] = {v.x, v.y, v.z, v.w};
+    // four bytes per SIMD compare: 0xFF per byte in range, then gather the four byte
+    // flags into four bits with one multiply (bit 0 of byte i lands on bit 24+i)
+    const uint32_t lo4 = (uint32_t)p.lo32 * 0x01010101u, hi4 = (uint32_t)p.hi32 * 0x01010101u;
+    const uint32_t w4[4] = {v.x, v.y, v.z, v.w};
 #pragma unroll
-    for (int i = 0; i < 16; ++i) {
-      int64_t x = (int64_t)((w4[i >> 2] >> (8 * (i & 3))) & 0xFF);
-      b |= (uint32_t)(x >= p.lo && x <= p.hi) << i;
+    for (int i = 0; i < 4; ++i) {
+      uint32_t f = __vcmpgeu4(w4[i], lo4) & __vcmpleu4(w4[i], hi4) & 0x01010101u;
+      b |= ((f * 0x01020408u) >> 24) << (4 * i);
     }
   } else if constexpr (W == 4) {
     int32_t x4[4] = {(int32_t)v.x, (int32_t)v.y, (int32_t)v.z, (int32_t)v.w};
 #pragma unroll
-    for (int i = 0; i < 4; ++i) b |= (uint32_t)((int64_t)x4[i] >= p.lo && (int64_t)x4[i] <= p.hi) << i;
+    for (int i = 0; i < 4; ++i) b |= (uint32_t)(x4[i] >= p.lo32 && x4[i] <= p.hi32) << i;
   } else {
     uint64_t u0 = ((uint64_t)v.y << 32) | v.x, u1 = ((uint64_t)v.w << 32) | v.z;
     if (p.is_f64) {
@@ -99,11 +102,50 @@ __global__ void __launch_bounds__(256) k_select_bitmap(const __grid_constant__ S
   }
 }
 
-__global__ void k_bitmap_combine(int op, const uint32_t* __restrict__ a, const uint32_t* __restrict__ b,
-                                 uint32_t* __restrict__ out, int64_t n) {
+__device__ __forceinline__ uint32_t combine_op(int op, uint32_t x, uint32_t y) {
+  return op == 0 ? (x & y) : (op == 1 ? (x | y) : (x & ~y));
+}
+
+// 16-byte vectors (4 words) per thread and iteration, 4 vectors in flight; the
+// last word is masked to n (bits past n are zero, s1).
+__global__ void __launch_bounds__(256) k_bitmap_combine(int op, const uint32_t* __restrict__ a,
+                                                        const uint32_t* __restrict__ b, uint32_t* __restrict__ out,
+                                                        int64_t n, int32_t vec) {
   const int64_t words = (n + 31) >> 5;
   const uint32_t tail_mask = (n & 31) ? ((1u << (n & 31)) - 1) : 0xFFFFFFFFu;
-  for (int64_t w = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; w < words; w += (int64_t)gridDim.x * blockDim.x) {
+  int64_t done = 0;
+  if (vec) {
+    constexpr int U = 4;
+    const int64_t nv = words >> 2;
+    const uint4* a4 = (const uint4*)a;
+    const uint4* b4 = (const uint4*)b;
+    uint4* o4 = (uint4*)out;
+    const int64_t stride = (int64_t)gridDim.x * blockDim.x;
+    for (int64_t v0 = blockIdx.x * (int64_t)blockDim.x * U + threadIdx.x; v0 < nv; v0 += stride * U) {
+      uint4 x[U], y[U];
+#pragma unroll
+      for (int u = 0; u < U; ++u) {
+        const int64_t v = v0 + (int64_t)u * blockDim.x;
+        if (v < nv) {
+          x[u] = __ldcs(a4 + v);
+          y[u] = __ldcs(b4 + v);
+        }
+      }
+#pragma unroll
+      for (int u = 0; u < U; ++u) {
+        const int64_t v = v0 + (int64_t)u * blockDim.x;
+        if (v < nv) {
+          uint4 r = make_uint4(combine_op(op, x[u].x, y[u].x), combine_op(op, x[u].y, y[u].y),
+                               combine_op(op, x[u].z, y[u].z), combine_op(op, x[u].w, y[u].w));
+          if (4 * v + 3 == words - 1) r.w &= tail_mask;
+          __stcs(o4 + v, r);
+        }
+      }
+    }
+    done = nv * 4;
+  }
+  for (int64_t w = done + blockIdx.x * (int64_t)blockDim.x + threadIdx.x; w < words;
+       w += (int64_t)gridDim.x * blockDim.x) {
     uint32_t x = __ldg(a + w), y = __ldg(b + w);
     uint32_t v = op == 0 ? (x & y) : (op == 1 ? (x | y) : (x & ~y));
     if (w == words - 1) v &= tail_mask;
@@ -112,8 +154,19 @@ __global__ void k_bitmap_combine(int op, const uint32_t* __restrict__ a, const u
 }
 
 // ---------------------------------------------------------------- host launchers
-cudaError_t launch_select_bitmap(const SelParams& p, int grid, cudaStream_t s) {
-  if (p.n == 0) return cudaSuccess;
+cudaError_t launch_select_bitmap(const SelParams& p0, int grid, cudaStream_t s) {
+  if (p0.n == 0) return cudaSuccess;
+  SelParams p = p0;
+  if (p.dtype == OCL_U8 || p.dtype == OCL_I32) {   // clamp the int64 bounds to the column's value range
+    const int64_t tmin = p.dtype == OCL_U8 ? 0 : INT32_MIN, tmax = p.dtype == OCL_U8 ? 255 : INT32_MAX;
+    if (p.lo > tmax || p.hi < tmin || p.lo > p.hi) {
+      p.lo32 = 1;
+      p.hi32 = 0;
+    } else {
+      p.lo32 = (int32_t)(p.lo < tmin ? tmin : p.lo);
+      p.hi32 = (int32_t)(p.hi > tmax ? tmax : p.hi);
+    }
+  }
   int64_t tiles = (p.n + 1023) >> 10;
   int64_t g = (tiles + 7) / 8;             // 8 warps per block
   if (g > grid) g = grid;
@@ -129,10 +182,11 @@ cudaError_t launch_bitmap_combine(int op, const uint32_t* a, const uint32_t* b, 
                                   cudaStream_t s) {
   if (n == 0) return cudaSuccess;
   int64_t words = (n + 31) >> 5;
-  int64_t g = (words + 255) / 256;
+  const int vec = ((uintptr_t)a % 16 == 0) && ((uintptr_t)b % 16 == 0) && ((uintptr_t)out % 16 == 0);
+  int64_t g = (words + 1023) / 1024;
   if (g > grid) g = grid;
   count_launch();
-  k_bitmap_combine<<<(int)g, 256, 0, s>>>(op, a, b, out, n);
+  k_bitmap_combine<<<(int)g, 256, 0, s>>>(op, a, b, out, n, vec);
   return cudaGetLastError();
 }
 

@@ -338,15 +338,31 @@ __global__ void __launch_bounds__(256) k_group_build(const __grid_constant__ Pla
 }
 
 // ------------------------------------------------------------------ projection (K4)
-__global__ void k_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
-                         void* out) {
+// U oids per thread and iteration: the oid loads, then the dependent column loads,
+// are all in flight before the first store.
+template <class T>
+__global__ void __launch_bounds__(256) k_gather(const T* __restrict__ col, const uint32_t* __restrict__ oids,
+                                                const int64_t* m_dev, int64_t max_m, T* __restrict__ out) {
+  constexpr int U = 4;
   int64_t m = m_dev ? *m_dev : max_m;
   if (m > max_m) m = max_m;
-  for (int64_t j = blockIdx.x * (int64_t)blockDim.x + threadIdx.x; j < m; j += (int64_t)gridDim.x * blockDim.x) {
-    uint32_t r = __ldg(oids + j);
-    if (width == 1) ((uint8_t*)out)[j] = __ldg((const uint8_t*)col + r);
-    else if (width == 4) ((int32_t*)out)[j] = __ldg((const int32_t*)col + r);
-    else ((long long*)out)[j] = __ldg((const long long*)col + r);
+  const int64_t stride = (int64_t)gridDim.x * blockDim.x * U;
+  for (int64_t j0 = blockIdx.x * (int64_t)blockDim.x * U + threadIdx.x; j0 < m; j0 += stride) {
+    uint32_t r[U];
+    T v[U];
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      const int64_t j = j0 + (int64_t)u * blockDim.x;
+      r[u] = j < m ? __ldcs(oids + j) : 0u;
+    }
+#pragma unroll
+    for (int u = 0; u < U; ++u)
+      if (j0 + (int64_t)u * blockDim.x < m) v[u] = __ldg(col + r[u]);
+#pragma unroll
+    for (int u = 0; u < U; ++u) {
+      const int64_t j = j0 + (int64_t)u * blockDim.x;
+      if (j < m) __stcs(out + j, v[u]);
+    }
   }
 }
 
@@ -441,10 +457,12 @@ cudaError_t launch_group_build(const Plan& p, int32_t* gid_out, int64_t max_rows
 cudaError_t launch_gather(const void* col, int32_t width, const uint32_t* oids, const int64_t* m_dev, int64_t max_m,
                           void* out, int grid, cudaStream_t s) {
   if (max_m == 0) return cudaSuccess;
-  int64_t g = (max_m + 255) / 256;
+  int64_t g = (max_m + 1023) / 1024;
   if (g > grid) g = grid;
   count_launch();
-  k_gather<<<(int)g, 256, 0, s>>>(col, width, oids, m_dev, max_m, out);
+  if (width == 1) k_gather<uint8_t><<<(int)g, 256, 0, s>>>((const uint8_t*)col, oids, m_dev, max_m, (uint8_t*)out);
+  else if (width == 4) k_gather<int32_t><<<(int)g, 256, 0, s>>>((const int32_t*)col, oids, m_dev, max_m, (int32_t*)out);
+  else k_gather<long long><<<(int)g, 256, 0, s>>>((const long long*)col, oids, m_dev, max_m, (long long*)out);
   return cudaGetLastError();
 }
 
