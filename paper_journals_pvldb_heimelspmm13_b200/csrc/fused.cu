@@ -362,7 +362,7 @@ cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cuda
   if (mode == 0 && p.vec_ok && !p.miss_agg && p.smem_cap == 0 && getenv("OCL_NO_SPEC") == nullptr) {
     cudaError_t err = cudaSuccess;
     if (launch_fused_spec(p, sms, s, &err, kind)) {
-      *kind += 10;                       // 11 / 12: Q1-signature kernel (int / fp64)
+      *kind += 10;                       // 11 / 12: Q1-signature kernel (int / fp64); 13 / 14: bulk pipeline
       return err;
     }
   }
@@ -395,6 +395,8 @@ const char* fused_kernel_name(int kind) {
     case 4: return "k_sga<StaticShape pred i32, key i64, COUNT/SUM/MIN/MAX>";
     case 11: return "k_sga_priv<Sig Q1 int64>";
     case 12: return "k_sga_priv<Sig Q1 fp64>";
+    case 13: return "k_sga_bulk<Sig Q1 int64> (TMA bulk pipeline)";
+    case 14: return "k_sga_bulk<Sig Q1 fp64> (TMA bulk pipeline)";
     case 20: return "k_sga_glb<DynShape>";
     default: return "k_sga<DynShape>";
   }
