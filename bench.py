@@ -9,7 +9,7 @@ configuration the north-star target (>= 60% of HBM bandwidth on one B200) is
 quoted on.  N > 1 (torchrun): rows are sharded across ranks (fixed total work,
 "strong" scaling) and the partial group tables are merged with an NCCL allgather.
 
-    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload c4|c2|c1|c3] [--impl ours|reference]
+    python bench.py [--gpus N] [--steps K] [--warmup W] [--workload c4|c2|c1|c3|c3c|c5] [--impl ours|reference]
 """
 from __future__ import annotations
 
@@ -47,8 +47,12 @@ WORKLOADS = {
     "c1": dict(desc="C1: lineitem SF0.01, 60,000 rows; Q1-style 4 groups, int64 decimals",
                rows=60_000, seed=datagen.BASE_SEED + 1, kind="q1", f64=False, groups=4),
     "c3": dict(desc="C3: lineitem SF10, 60,000,000 rows; GROUP BY l_orderkey (15M groups, HBM hash table), "
-                    "COUNT/SUM/MIN/MAX(l_quantity), clustered row order",
-               rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000),
+                    "COUNT/SUM/MIN/MAX(l_quantity), shuffled row order (seeded Feistel permutation)",
+               rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000,
+               shuffled=True),
+    "c3c": dict(desc="C3 clustered: lineitem SF10, 60,000,000 rows; GROUP BY l_orderkey (15M groups), "
+                     "COUNT/SUM/MIN/MAX(l_quantity), dbgen (clustered) row order",
+                rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000),
     "c5": dict(desc="C5 sweep point: 2^28 rows, p i32 ~ U[0,1e6), key = hash(Zipf(s) rank over G), v i64; "
                     "WHERE p < T GROUP BY key: COUNT, SUM, MIN, MAX(v)",
                rows=1 << 28, seed=datagen.BASE_SEED + 5, kind="sweep", f64=False, groups=1 << 10),
@@ -85,7 +89,8 @@ def wl_fields(wl):
 def gen_device(wl, length, start, n, dev):
     if wl["kind"] == "sweep":
         return datagen.sweep_device(length, wl["seed"], wl["groups"], s=wl["zipf"], row0=start, device=dev)
-    return datagen.lineitem_device(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, device=dev)
+    return datagen.lineitem_device(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n,
+                                   shuffled=wl.get("shuffled", False), device=dev)
 
 
 def gen_host(wl, length, start, n, out=None):
@@ -96,7 +101,8 @@ def gen_host(wl, length, start, n, out=None):
                 out[f][:] = h[f]
             return out
         return h
-    return datagen.lineitem_host(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n, out=out)
+    return datagen.lineitem_host(length, wl["seed"], fields=wl_fields(wl), row0=start, n_total=n,
+                                 shuffled=wl.get("shuffled", False), out=out)
 
 
 class ClockSampler:

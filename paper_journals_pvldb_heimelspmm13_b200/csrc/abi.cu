@@ -116,6 +116,7 @@ struct Planned {
   bool values_f64;   // every value expression is fp64
   uint64_t cap;      // table capacity (power of two)
   size_t table_bytes;
+  int32_t pbits;     // >= 0: hash-partitioned high-cardinality tier with 2^pbits partitions (partition.cu)
 };
 
 ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* aggs, int32_t naggs, Planned* P) {
@@ -316,6 +317,9 @@ ocl_status plan_preds(const ocl_column* pred_cols, const ocl_range* preds, int32
 
 // Shared-memory budget of one register-tier CTA (private records + mid-G table).
 constexpr size_t kRegTierSmem = 200 * 1024;
+// Auto selection of the hash-partitioned tier.
+constexpr int64_t kPartMinGroups = 4096;
+constexpr int64_t kPartMinRows = 1 << 20;
 
 // Tier selection: 0 auto; 1 register tier (private slots + HBM);
 // 2 HBM-only kernel; 3 register tier with the dynamic (unspecialised) shape;
@@ -376,6 +380,11 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   p.bitmap_out = a->bitmap_out;
   p.smem_cap = plan_smem_cap(a, p);
   p.miss_agg = a->expected_groups > reg_tier_slots() ? 1 : 0;
+  // High-cardinality tier: more groups than the shared-memory tiers hold, integer
+  // column values, enough rows to amortise its five launches (tier 5 forces it).
+  P->pbits = -1;
+  const bool many = a->tier == 0 && p.smem_cap == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
+  if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;
   f.keys_out = a->keys_out;
@@ -389,7 +398,10 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
 
 
 // table + finalize workspace of a fused call
-size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) { return P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256); }
+size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) {
+  return P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256) +
+         (P.pbits >= 0 ? part_ws_bytes(P.plan, P.pbits, ctx->sms) : 0);
+}
 
 // Run the fused pass into a zeroed table carved from ws; returns the emit workspace.
 ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, size_t ws_bytes, cudaStream_t s,
@@ -403,7 +415,12 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   if (P.plan.n > 0) {
     if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, s), "profile event");
     int kind = 0;
-    OCL_CUDA(launch_fused(P.plan, fused_mode(a), P.values_f64, ctx->sms, s, &kind), "fused kernel launch");
+    if (P.pbits >= 0) {
+      void* pws = (uint8_t*)ws + P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256);
+      OCL_CUDA(launch_partitioned(P.plan, P.pbits, pws, ctx->sms, s, &kind), "partitioned aggregation launch");
+    } else {
+      OCL_CUDA(launch_fused(P.plan, fused_mode(a), P.values_f64, ctx->sms, s, &kind), "fused kernel launch");
+    }
     ctx->last_kernel = kind;
     if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, s), "profile event");
   }
@@ -790,6 +807,7 @@ ocl_status ocl_select_group_aggregate_host_workspace_size(ocl_ctx* ctx, const oc
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
+  P.pbits = -1;             // chunks stream through the one-pass fused kernel
   HostCols h;
   collect_host_cols(P, h, chunk_rows);
   *bytes = sga_ws_bytes(ctx, P) + 2 * h.slot_bytes + host_out_bytes(args, P);
@@ -806,6 +824,7 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
   if (!ws || ws_bytes < need) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
   Planned P;
   if ((s = plan_sga(args, &P))) return s;
+  P.pbits = -1;
   HostCols h;
   collect_host_cols(P, h, chunk_rows);
   // carve: [table | emit ws] [staging slot 0] [staging slot 1] [device outputs]

@@ -216,7 +216,9 @@ __device__ __forceinline__ uint8_t* table_find_or_insert(uint8_t* table, uint64_
     return e;
   }
   uint64_t sk = ~key;
-  uint64_t h = fmix64(key) & mask;
+  // start slot = the top log2(cap) bits of the hash: the keys of hash partition q
+  // (top bits = q, partition.cu) occupy one contiguous slot range
+  uint64_t h = __umul64hi(fmix64(key), mask + 1);
   for (uint64_t probe = 0; probe <= mask; ++probe) {
     uint64_t* kp = (uint64_t*)(table + h * (uint64_t)stride);
     uint64_t cur = ld_relaxed_u64(kp);

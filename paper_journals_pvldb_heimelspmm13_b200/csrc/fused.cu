@@ -398,6 +398,9 @@ const char* fused_kernel_name(int kind) {
     case 13: return "k_sga_bulk<Sig Q1 int64> (TMA bulk pipeline)";
     case 14: return "k_sga_bulk<Sig Q1 fp64> (TMA bulk pipeline)";
     case 20: return "k_sga_glb<DynShape>";
+    case 30: return "k_part_count/scatter/agg<DynShape> (hash-partitioned)";
+    case 31: return "k_part_count/scatter/agg<StaticShape key i64> (hash-partitioned)";
+    case 32: return "k_part_count/scatter/agg<StaticShape pred i32, key i64> (hash-partitioned)";
     default: return "k_sga<DynShape>";
   }
 }

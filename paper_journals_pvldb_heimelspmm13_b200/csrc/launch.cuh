@@ -60,4 +60,9 @@ int reg_tier_slots();
 const char* fused_kernel_name(int kind);
 // Proven few-group Q1 kernel (fused_spec.cu) used while the unified kernel is tuned.
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
+// High-cardinality tier (partition.cu): hash-partitioned two-pass aggregation.
+bool part_eligible(const Plan& p);
+int part_bits_for(int64_t expected_groups);
+size_t part_ws_bytes(const Plan& p, int pbits, int sms);
+cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind);
 }  // namespace ocl

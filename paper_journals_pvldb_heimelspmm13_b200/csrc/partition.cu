@@ -1,0 +1,763 @@
+// partition.cu — high-cardinality tier of the fused select -> group -> aggregate:
+// hash-partitioned two-pass aggregation.
+//
+// The paper's GPU group-by inserts every row into one device-wide hash table with
+// atomics and names hashing "one of the major shortcomings" (PAPER.md L949-954
+// §5.2.1); for many groups the table lives in device memory and every row pays a
+// random read-modify-write there (§4.1.6, §4.1.7).  It also
+// suggests partitioning the work over a global hash table.  On B200 a
+// random atomic into a table larger than L2 costs ~10x a streamed row
+// (tools/micro/atom_bench.cu: 10.9 G rows/s for 4 atomics per row into 1 GB), while
+// 32-bit shared-memory atomics on random addresses sustain ~8 per clock per SM
+// (tools/micro/smem_atom_bench.cu).  So for many groups the rows are first routed by
+// hash to P = 2^pbits partitions small enough for a shared-memory table:
+//
+//   pass 1a  k_part_count    fused select + key + values, per row-block histogram of
+//                            partition ids (shared-memory counters)
+//   scan     k_scan_*        exclusive scan of the partition counts
+//   pass 1b  k_part_scatter  the same rows again: each qualifying row becomes a
+//                            record {key, int32 values} at its partition's global
+//                            cursor (one atomic per row, or per warp for a hot one)
+//   pass 2   k_part_agg      work items of <= kPartItem records of one partition; a
+//                            CTA aggregates an item in a shared-memory hash table
+//                            (32-bit atomics, the CTA-table layout of the fused
+//                            kernel) and merges every entry once into the HBM table
+//                            (plain read-modify-write when the partition is one item)
+//
+// The HBM table's start slot is the top bits of the key hash (common.cuh), so a
+// partition's keys occupy one contiguous slot range: pass-2 merges stay L2-local.
+// Rows the fast path cannot take (values outside int32, the key ~0) and records
+// whose partition overflows the shared table update the HBM table directly (exact).
+#include "launch.cuh"
+#include "sga_device.cuh"
+
+namespace ocl {
+
+constexpr int kPartThreads = 512;
+constexpr int kPartCap = 2048;        // shared-table entries per CTA in pass 2 (power of two)
+constexpr int kPartItem = 16384;      // records per pass-2 work item (< 2^16: split-sum bound of the table)
+constexpr int kPartILP = 4;           // rows / records per thread in flight (part_rows: 2 units x 2 rows)
+constexpr int kTileMapBits = 12;      // scatter: per-tile partition map (2 x the tile's rows)
+constexpr int kPartLevelBits = 7;     // partitions reached per scatter level (tile claims aggregate ~16x)
+constexpr int kTileMap = 1 << kTileMapBits;
+constexpr int kScanThreads = 1024;
+constexpr int kScanPer = 8;           // elements per thread per scan chunk
+constexpr int kScanChunk = kScanThreads * kScanPer;
+
+struct PartArgs {
+  int32_t pbits;
+  int32_t nblk;
+  int64_t rows_per_blk;
+  uint32_t* counts;     // [P] histogram of partition ids
+  uint32_t* offs;       // [P] exclusive scan of counts: partition starts
+  uint32_t* cur;        // [P] global write cursors of pass 1b (start = offs)
+  uint32_t* sums;       // scan chunk sums
+  int64_t* m_dev;       // number of records
+  uint8_t* recs;        // records: {key u64, int32 value x NV}, rec_bytes each, grouped by partition
+  uint8_t* tmp;         // level-1 records (two-level scatter), grouped by the top b1 hash bits
+  uint32_t* cur1;       // [2^b1] level-1 cursors
+  uint32_t* icnt;       // [P] pass-2 work items per partition
+  uint32_t* ioff;       // [P] exclusive scan of icnt
+  uint32_t* isums;      // scan chunk sums of icnt
+  int64_t* nitems_dev;  // number of pass-2 work items
+  int32_t rec_bytes;
+};
+
+__device__ __forceinline__ uint32_t part_of(uint64_t key, int pbits) {
+  return pbits ? (uint32_t)(fmix64(key) >> (64 - pbits)) : 0u;
+}
+
+// Lanes whose partition equals lane 0's are served by one shared-memory atomic of
+// lane 0 (hot keys of skewed data); the others each take one.  Returns the base
+// position for the aggregated group (valid in lanes of `same`) via *base.
+__device__ __forceinline__ uint32_t lanemask_lt() {
+  uint32_t m;
+  asm("mov.u32 %0, %%lanemask_lt;" : "=r"(m));
+  return m;
+}
+
+template <class Sh, int NV>
+__device__ __forceinline__ void part_eval(const Plan& p, int64_t r, int64_t r1, Row<Sh, NV, false>& x, bool& ok) {
+  eval_one<Sh, NV, false>(p, r, x);
+  x.q = x.q && r < r1;
+  ok = x.q && x.fast && !Sh::special(x.key);
+}
+
+// The kPartILP = 4 rows of a lane in a tile: warp w owns the 128 rows [wbase, wbase +
+// 128) as two 64-row units, lane l their rows 2l, 2l+1 (the fused kernel's layout).
+// Static shapes with aligned columns load both units with vector loads, no branches,
+// all loads in flight before any row is evaluated; the rest evaluate row by row.
+__device__ __forceinline__ int64_t part_row(int64_t wbase, int lane, int i) {
+  return wbase + (i >> 1) * 64 + 2 * lane + (i & 1);
+}
+
+template <class Sh, int NV>
+__device__ __forceinline__ void part_rows(const Plan& p, int64_t wbase, int64_t r1, int lane,
+                                          Row<Sh, NV, false> (&x)[4], bool (&ok)[4]) {
+  if constexpr (Sh::kStatic) {
+    if (p.vec_ok && wbase + 128 <= r1) {
+      RawUnit<Sh> u[2];
+      load_unit<Sh>(p, wbase + 2 * lane, u[0]);
+      load_unit<Sh>(p, wbase + 64 + 2 * lane, u[1]);
+#pragma unroll
+      for (int i = 0; i < 4; ++i) {
+        eval_unit<Sh, NV, false>(p, u[i >> 1], i & 1, x[i]);
+        ok[i] = x[i].q && x[i].fast && !Sh::special(x[i].key);
+      }
+      return;
+    }
+  }
+#pragma unroll
+  for (int i = 0; i < 4; ++i) part_eval<Sh, NV>(p, part_row(wbase, lane, i), r1, x[i], ok[i]);
+}
+
+// ------------------------------------------------------------------ pass 1a: histogram
+template <class Sh, int NV>
+__global__ void __launch_bounds__(kPartThreads) k_part_count(const __grid_constant__ Plan p, PartArgs a) {
+  extern __shared__ uint32_t hist[];
+  const int P = 1 << a.pbits;
+  const int lane = threadIdx.x & 31;
+  for (int i = threadIdx.x; i < P; i += blockDim.x) hist[i] = 0;
+  __syncthreads();
+  const int64_t r0 = blockIdx.x * a.rows_per_blk;
+  const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
+  const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
+  for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
+    Row<Sh, NV, false> x[kPartILP];
+    bool ok[kPartILP];
+    part_rows<Sh, NV>(p, base + woff, r1, lane, x, ok);
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      const uint32_t part = ok[k] ? part_of((uint64_t)x[k].key, a.pbits) : 0xFFFFFFFFu;
+      const uint32_t p0 = __shfl_sync(0xffffffffu, part, 0);
+      const unsigned same = __ballot_sync(0xffffffffu, ok[k] && part == p0);
+      if (ok[k] && part != p0) atomicAdd(&hist[part], 1u);
+      if (lane == 0 && same) atomicAdd(&hist[p0], (uint32_t)__popc(same));
+    }
+  }
+  __syncthreads();
+  for (int i = threadIdx.x; i < P; i += blockDim.x)
+    if (hist[i]) atomicAdd(&a.counts[i], hist[i]);
+}
+
+// ------------------------------------------------------------------ pass 1b: scatter
+// Scatter claims, aggregated per tile of kPartILP x T rows or records: a shared-memory
+// map partition -> count gives every item its rank, then one global atomic per
+// distinct partition of the tile claims the range from that partition's cursor
+// (shared by all CTAs).  Shared cursors keep only a couple of lines per partition
+// open in L2, so the 16-byte record stores combine into full lines (per-CTA ranges
+// kept P x #CTAs partial lines open, overflowed L2 and turned every store into a
+// partial-sector read-modify-write: measured 2x writes, 2.4x reads).  Aggregation
+// needs several items per partition per tile, so more than 128 partitions are
+// reached in two levels (k_part_scatter2).
+struct TileMap {
+  uint32_t key[kTileMap];
+  uint32_t cnt[kTileMap];                  // count, then the global base of the slot's range
+  uint32_t off[kTileMap];                  // the slot's first index in the staging area
+  uint16_t sslot[kPartILP * kPartThreads]; // slot of each staged item
+  uint4 stage[kPartILP * kPartThreads];    // the tile's records, grouped by partition
+  uint32_t total;                          // items in the tile
+};
+
+__device__ __forceinline__ void tile_map_clear(TileMap& m) {
+  for (int i = threadIdx.x; i < kTileMap; i += blockDim.x) {
+    m.key[i] = 0xFFFFFFFFu;
+    m.cnt[i] = 0;
+  }
+}
+
+// slot of `part` in the map (inserted if new) and this item's rank within it
+__device__ __forceinline__ void tile_map_add(TileMap& m, uint32_t part, uint32_t& slot, uint32_t& rank) {
+  volatile uint32_t* vk = m.key;
+  uint32_t h = (part * 0x9E3779B1u) >> (32 - kTileMapBits);
+  while (true) {                           // < kTileMap / 2 distinct partitions per tile: terminates
+    const uint32_t cur = vk[h];
+    if (cur == part) break;
+    if (cur == 0xFFFFFFFFu) {
+      const uint32_t prev = atomicCAS(&m.key[h], 0xFFFFFFFFu, part);
+      if (prev == 0xFFFFFFFFu || prev == part) break;
+    }
+    h = (h + 1) & (kTileMap - 1);
+  }
+  slot = h;
+  rank = atomicAdd(&m.cnt[h], 1u);
+}
+
+// After a barrier: counts -> global bases, and each slot's offset in the staging area
+// (exclusive scan of the counts: kPartThreads threads x kTileMap / kPartThreads slots).
+__device__ __forceinline__ void tile_map_claim(TileMap& m, uint32_t* cur, uint32_t* wsum) {
+  constexpr int PER = kTileMap / kPartThreads;
+  const int t = threadIdx.x, lane = t & 31, w = t >> 5;
+  uint32_t c[PER], tot = 0;
+#pragma unroll
+  for (int i = 0; i < PER; ++i) {
+    c[i] = m.cnt[t * PER + i];
+    tot += c[i];
+  }
+  uint32_t incl = tot;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+    if (lane >= o) incl += y;
+  }
+  if (lane == 31) wsum[w] = incl;
+  __syncthreads();
+  if (w == 0) {
+    const uint32_t x = lane < kPartThreads / 32 ? wsum[lane] : 0u;
+    uint32_t xi = x;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, xi, o);
+      if (lane >= o) xi += y;
+    }
+    if (lane < kPartThreads / 32) wsum[lane] = xi - x;
+  }
+  __syncthreads();
+  uint32_t run = wsum[w] + incl - tot;
+#pragma unroll
+  for (int i = 0; i < PER; ++i) {
+    const int sl = t * PER + i;
+    m.off[sl] = run;
+    run += c[i];
+    if (c[i]) m.cnt[sl] = atomicAdd(&cur[m.key[sl]], c[i]);
+  }
+  if (t == kPartThreads - 1) m.total = run;
+}
+
+// Stage item (slot, rank) in the tile's partition-grouped order.
+__device__ __forceinline__ void tile_stage(TileMap& m, uint32_t slot, uint32_t rank, uint4 rec) {
+  const uint32_t i = m.off[slot] + rank;
+  m.stage[i] = rec;
+  m.sslot[i] = (uint16_t)slot;
+}
+
+// After a barrier: write the staged records; consecutive lanes write consecutive
+// records of one partition (coalesced runs instead of one line per lane).
+__device__ __forceinline__ void tile_flush(TileMap& m, uint32_t nitems, uint8_t* out, int rec_bytes) {
+  for (uint32_t i = threadIdx.x; i < nitems; i += blockDim.x) {
+    const uint32_t sl = m.sslot[i];
+    *(uint4*)(out + (size_t)(m.cnt[sl] + (i - m.off[sl])) * rec_bytes) = m.stage[i];
+  }
+}
+
+template <int NV>
+__device__ __forceinline__ uint4 pack_rec16(uint64_t key, const int32_t (&v)[NV > 0 ? NV : 1]) {
+  return make_uint4((uint32_t)key, (uint32_t)(key >> 32), NV > 0 ? (uint32_t)v[0] : 0u,
+                    NV > 1 ? (uint32_t)v[NV > 1 ? 1 : 0] : 0u);
+}
+
+template <int NV>
+__device__ __forceinline__ void store_rec(uint8_t* rec, uint64_t key, const int32_t (&v)[NV > 0 ? NV : 1]) {
+  uint32_t z[8] = {(uint32_t)key, (uint32_t)(key >> 32), 0, 0, 0, 0, 0, 0};
+#pragma unroll
+  for (int i = 0; i < NV; ++i) z[2 + i] = (uint32_t)v[i];
+  *(uint4*)rec = make_uint4(z[0], z[1], z[2], z[3]);
+  if constexpr (NV > 2) *(uint4*)(rec + 16) = make_uint4(z[4], z[5], z[6], z[7]);
+}
+
+template <int NV>
+__device__ __forceinline__ void load_rec(const uint8_t* rec, uint64_t& key, int32_t (&v)[NV > 0 ? NV : 1]) {
+  const uint4 q0 = *(const uint4*)rec;
+  key = (uint64_t)q0.x | ((uint64_t)q0.y << 32);
+  uint32_t z[6] = {q0.z, q0.w, 0, 0, 0, 0};
+  if constexpr (NV > 2) {
+    const uint4 q1 = *(const uint4*)(rec + 16);
+    z[2] = q1.x; z[3] = q1.y; z[4] = q1.z; z[5] = q1.w;
+  }
+#pragma unroll
+  for (int i = 0; i < NV; ++i) v[i] = (int32_t)z[i];
+}
+
+// Level 1: rows -> records grouped by the top `pb` hash bits (cursors `cur`, output `out`).
+template <class Sh, int NV>
+__global__ void __launch_bounds__(kPartThreads) k_part_scatter(const __grid_constant__ Plan p, PartArgs a, int pb,
+                                                               uint32_t* cur, uint8_t* out) {
+  extern __shared__ __align__(16) uint8_t dsm[];
+  TileMap& map = *(TileMap*)dsm;
+  __shared__ uint32_t wsum[32];
+  const int64_t r0 = blockIdx.x * a.rows_per_blk;
+  const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
+  const int lane = threadIdx.x & 31;
+  // software pipeline: the next tile's rows are loaded before this tile's claims,
+  // whose global atomics and barriers would otherwise serialise with the loads
+  Row<Sh, NV, false> nx[kPartILP];
+  bool nok[kPartILP];
+  const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
+  if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
+  for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
+    tile_map_clear(map);
+    Row<Sh, NV, false> x[kPartILP];
+    bool ok[kPartILP];
+    uint32_t slot[kPartILP], rank[kPartILP];
+    const int64_t wbase = base + woff;
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      x[k] = nx[k];
+      ok[k] = nok[k];
+    }
+    if (base + kPartILP * blockDim.x < r1) part_rows<Sh, NV>(p, wbase + kPartILP * blockDim.x, r1, lane, nx, nok);
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      if (x[k].q && !ok[k]) {               // exact per-row path straight into the HBM table
+        uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
+        if (e) update_entry_slow(p, e, part_row(wbase, lane, k));
+      }
+      if (ok[k]) tile_map_add(map, part_of((uint64_t)x[k].key, pb), slot[k], rank[k]);
+    }
+    __syncthreads();
+    tile_map_claim(map, cur, wsum);
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      if (!ok[k]) continue;
+      int32_t v[NV > 0 ? NV : 1];
+#pragma unroll
+      for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
+      if constexpr (NV <= 2) tile_stage(map, slot[k], rank[k], pack_rec16<NV>((uint64_t)x[k].key, v));
+      else store_rec<NV>(out + (size_t)(map.cnt[slot[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
+    }
+    __syncthreads();
+    if constexpr (NV <= 2) {
+      tile_flush(map, map.total, out, a.rec_bytes);
+      __syncthreads();
+    }
+  }
+}
+
+// Level 2: records grouped by their top b1 hash bits -> records grouped by all pbits.
+// A tile of consecutive level-1 records spans one or two level-1 partitions, so it
+// meets at most ~2^(pbits-b1) final partitions: the tile claims aggregate again.
+template <int NV>
+__global__ void __launch_bounds__(kPartThreads) k_part_scatter2(PartArgs a) {
+  extern __shared__ __align__(16) uint8_t dsm[];
+  TileMap& map = *(TileMap*)dsm;
+  __shared__ uint32_t wsum[32];
+  const int64_t m = *a.m_dev;
+  constexpr int TILE = kPartILP * kPartThreads;
+  const int64_t per = ((m + gridDim.x - 1) / gridDim.x + TILE - 1) / TILE * TILE;
+  const int64_t j0 = blockIdx.x * per, j1 = min(m, j0 + per);
+  uint64_t nkey[kPartILP];
+  int32_t nv[kPartILP][NV > 0 ? NV : 1];
+  auto fetch = [&](int64_t b) {
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      const int64_t j = b + k * kPartThreads + threadIdx.x;
+      if (j < j1) load_rec<NV>(a.tmp + (size_t)j * a.rec_bytes, nkey[k], nv[k]);
+    }
+  };
+  if (j0 < j1) fetch(j0);
+  for (int64_t base = j0; base < j1; base += TILE) {
+    tile_map_clear(map);
+    uint64_t key[kPartILP];
+    int32_t v[kPartILP][NV > 0 ? NV : 1];
+    bool ok[kPartILP];
+    uint32_t slot[kPartILP], rank[kPartILP];
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      ok[k] = base + k * kPartThreads + threadIdx.x < j1;
+      key[k] = nkey[k];
+#pragma unroll
+      for (int i = 0; i < NV; ++i) v[k][i] = nv[k][i];
+    }
+    if (base + TILE < j1) fetch(base + TILE);
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k)
+      if (ok[k]) tile_map_add(map, part_of(key[k], a.pbits), slot[k], rank[k]);
+    __syncthreads();
+    tile_map_claim(map, a.cur, wsum);
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      if (!ok[k]) continue;
+      if constexpr (NV <= 2) tile_stage(map, slot[k], rank[k], pack_rec16<NV>(key[k], v[k]));
+      else store_rec<NV>(a.recs + (size_t)(map.cnt[slot[k]] + rank[k]) * a.rec_bytes, key[k], v[k]);
+    }
+    __syncthreads();
+    if constexpr (NV <= 2) {
+      tile_flush(map, map.total, a.recs, a.rec_bytes);
+      __syncthreads();
+    }
+  }
+}
+
+// cursors of level 1: start of level-1 partition q1 = start of final partition q1 << b2
+__global__ void k_part_cur1(const uint32_t* offs, uint32_t* cur1, int b1, int b2) {
+  const int i = blockIdx.x * blockDim.x + threadIdx.x;
+  if (i < (1 << b1)) cur1[i] = offs[(size_t)i << b2];
+}
+
+// ------------------------------------------------------------------ scan (exclusive, u32)
+__global__ void __launch_bounds__(kScanThreads) k_scan_chunks(const uint32_t* in, uint32_t* out, uint32_t* sums,
+                                                               int64_t n) {
+  __shared__ uint32_t wsum[kScanThreads / 32];
+  const int64_t c0 = (int64_t)blockIdx.x * kScanChunk + (int64_t)threadIdx.x * kScanPer;
+  uint32_t v[kScanPer], t = 0;
+#pragma unroll
+  for (int i = 0; i < kScanPer; ++i) {
+    v[i] = c0 + i < n ? in[c0 + i] : 0u;
+    t += v[i];
+  }
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  uint32_t incl = t;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+    if (lane >= o) incl += y;
+  }
+  if (lane == 31) wsum[w] = incl;
+  __syncthreads();
+  if (w == 0) {
+    uint32_t s = wsum[lane];
+    uint32_t si = s;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, si, o);
+      if (lane >= o) si += y;
+    }
+    wsum[lane] = si - s;
+    if (lane == 31) sums[blockIdx.x] = si;
+  }
+  __syncthreads();
+  uint32_t run = wsum[w] + incl - t;
+#pragma unroll
+  for (int i = 0; i < kScanPer; ++i) {
+    if (c0 + i < n) out[c0 + i] = run;
+    run += v[i];
+  }
+}
+
+// One CTA: exclusive scan of the chunk sums in place; total -> *total.
+__global__ void __launch_bounds__(kScanThreads) k_scan_sums(uint32_t* sums, int64_t nchunks, int64_t* total) {
+  __shared__ uint32_t wsum[kScanThreads / 32];
+  __shared__ uint32_t carry;
+  if (threadIdx.x == 0) carry = 0;
+  __syncthreads();
+  const int lane = threadIdx.x & 31, w = threadIdx.x >> 5;
+  for (int64_t base = 0; base < nchunks; base += kScanThreads) {
+    const int64_t i = base + threadIdx.x;
+    const uint32_t v = i < nchunks ? sums[i] : 0u;
+    uint32_t incl = v;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+      if (lane >= o) incl += y;
+    }
+    if (lane == 31) wsum[w] = incl;
+    __syncthreads();
+    if (w == 0) {
+      uint32_t s = wsum[lane], si = s;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, si, o);
+        if (lane >= o) si += y;
+      }
+      wsum[lane] = si - s;
+    }
+    __syncthreads();
+    const uint32_t c = carry;
+    if (i < nchunks) sums[i] = c + wsum[w] + incl - v;
+    __syncthreads();
+    if (threadIdx.x == kScanThreads - 1) carry = c + wsum[w] + incl;
+    __syncthreads();
+  }
+  if (threadIdx.x == 0) *total = (int64_t)carry;
+}
+
+__global__ void k_scan_add(uint32_t* out, uint32_t* cur, const uint32_t* sums, int64_t n) {
+  const int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x;
+  if (i < n) cur[i] = out[i] += sums[i / kScanChunk];
+}
+
+// ------------------------------------------------------------------ pass 2: aggregate
+// Exact HBM update of one record that the shared table could not take.
+__device__ __forceinline__ void update_entry_rec(const Plan& p, uint8_t* e, const int32_t* v, int nv) {
+  atomicAdd((unsigned long long*)(e + 8), 1ULL);
+  for (int i = 0; i < nv; ++i) {
+    const DevValue& d = p.vals[i];
+    const int64_t x = v[i];
+    if (d.off_sum >= 0) atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)x, (uint64_t)(x >> 63));
+    if (d.off_min >= 0) atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(x));
+    if (d.off_max >= 0) atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(x));
+  }
+}
+
+// A whole warp of records with the same key (heavy hitters): one combined update.
+template <int NV>
+__device__ __forceinline__ void cta_add_warp(const Plan& p, uint8_t* e, const int32_t (&v)[NV > 0 ? NV : 1], int lane) {
+  if (lane == 0) atomicAdd((unsigned int*)(e + 8), 32u);
+#pragma unroll
+  for (int i = 0; i < NV; ++i) {
+    if (i >= p.nvals) break;
+    const DevValue& d = p.vals[i];
+    const uint32_t lo = __reduce_add_sync(0xffffffffu, (uint32_t)v[i] & 0xFFFFu);
+    const int32_t hi = (int32_t)__reduce_add_sync(0xffffffffu, (uint32_t)(v[i] >> 16));
+    const int32_t mn = __reduce_min_sync(0xffffffffu, v[i]);
+    const int32_t mx = __reduce_max_sync(0xffffffffu, v[i]);
+    if (lane == 0) {
+      if (d.co_lo >= 0) {
+        atomicAdd((unsigned int*)(e + d.co_lo), lo);
+        atomicAdd((int*)(e + d.co_hi), hi);
+      }
+      if (d.co_min >= 0) atomicMax((unsigned int*)(e + d.co_min), enc32_min(mn));
+      if (d.co_max >= 0) atomicMax((unsigned int*)(e + d.co_max), enc32_max(mx));
+    }
+  }
+}
+
+__device__ __forceinline__ int64_t part_start(const PartArgs& a, int64_t q, int64_t m) {
+  return q >= (1LL << a.pbits) ? m : (int64_t)a.offs[q];
+}
+
+// Work items of pass 2: partition q is cut into ceil(n_q / kPartItem) items.
+__global__ void k_part_items(PartArgs a) {
+  const int64_t q = blockIdx.x * (int64_t)blockDim.x + threadIdx.x;
+  if (q >= (1LL << a.pbits)) return;
+  const int64_t m = *a.m_dev;
+  const int64_t n = part_start(a, q + 1, m) - part_start(a, q, m);
+  a.icnt[q] = (uint32_t)((n + kPartItem - 1) / kPartItem);
+}
+
+// Merge a shared-table entry into the HBM table when this CTA is the only one
+// aggregating its partition (a one-item partition): plain read-modify-write of the
+// entry's fields — no other thread updates them (the scatter's exact path and this
+// CTA's own overflow updates happened before the barrier).  The slot is still
+// claimed with atomicCAS: linear probing may run into a neighbour partition's range.
+__device__ __forceinline__ void cta_flush_entry_excl(const Plan& p, const uint8_t* ce) {
+  const uint64_t sk = *(const uint64_t*)ce;
+  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+  if (sk == 0 || cnt == 0) return;
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
+  if (!e) return;
+  *(uint64_t*)(e + 8) += cnt;
+  for (int v = 0; v < p.nvals; ++v) {
+    const DevValue& d = p.vals[v];
+    if (d.co_lo >= 0) {
+      const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
+      I128 x{*(const uint64_t*)(e + d.off_sum), *(const uint64_t*)(e + d.off_sum + 8)};
+      x = i128_add(x, i128_from_i64(sum));
+      *(uint64_t*)(e + d.off_sum) = x.lo;
+      *(uint64_t*)(e + d.off_sum + 8) = x.hi;
+    }
+    if (d.co_min >= 0) {
+      const int32_t mn = (int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u);
+      uint64_t* f = (uint64_t*)(e + d.off_min);
+      *f = max(*f, enc_min_i(mn));
+    }
+    if (d.co_max >= 0) {
+      const int32_t mx = (int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u);
+      uint64_t* f = (uint64_t*)(e + d.off_max);
+      *f = max(*f, enc_max_i(mx));
+    }
+  }
+}
+
+template <int NV>
+__global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant__ Plan p, PartArgs a) {
+  using Sh = DynShape;
+  extern __shared__ __align__(16) uint8_t tab[];
+  const int lane = threadIdx.x & 31;
+  const int64_t m = *a.m_dev;
+  const int64_t nitems = *a.nitems_dev;
+  const int64_t P = 1LL << a.pbits;
+  const int cs = p.cta_stride;
+  for (int64_t item = blockIdx.x; item < nitems; item += gridDim.x) {
+    // the partition of this item: the largest q with ioff[q] <= item
+    int64_t lo = 0, hi = P - 1;
+    while (lo < hi) {
+      const int64_t mid = (lo + hi + 1) >> 1;
+      if ((int64_t)a.ioff[mid] <= item) lo = mid;
+      else hi = mid - 1;
+    }
+    const int64_t q0 = part_start(a, lo, m), q1 = part_start(a, lo + 1, m);
+    const int64_t s = q0 + (item - (int64_t)a.ioff[lo]) * kPartItem;
+    const int64_t seg_end = min(q1, s + kPartItem);
+    const bool exclusive = q1 - q0 <= kPartItem;
+    for (int i = threadIdx.x; i < kPartCap * cs / 16; i += blockDim.x) ((uint4*)tab)[i] = make_uint4(0, 0, 0, 0);
+    __syncthreads();
+    for (int64_t base = s; base < seg_end; base += kPartILP * blockDim.x) {
+      uint64_t key[kPartILP];
+      int32_t v[kPartILP][NV > 0 ? NV : 1];
+      bool valid[kPartILP];
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k) {   // loads of kPartILP records first
+        const int64_t j = base + k * blockDim.x + threadIdx.x;
+        valid[k] = j < seg_end;
+        key[k] = 0;
+#pragma unroll
+        for (int i = 0; i < NV; ++i) v[k][i] = 0;
+        if (valid[k]) load_rec<NV>(a.recs + (size_t)j * a.rec_bytes, key[k], v[k]);
+      }
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k) {
+        const uint64_t k0 = __shfl_sync(0xffffffffu, key[k], 0);
+        if (__all_sync(0xffffffffu, valid[k] && key[k] == k0)) {    // heavy hitter: one update per warp
+          uint8_t* te = lane == 0 ? cta_find_or_insert(tab, kPartCap, cs, k0) : nullptr;
+          const unsigned long long tp = __shfl_sync(0xffffffffu, (unsigned long long)te, 0);
+          if (tp) {
+            cta_add_warp<NV>(p, (uint8_t*)tp, v[k], lane);
+            continue;
+          }
+        }
+        if (!valid[k]) continue;
+        uint8_t* te = cta_find_or_insert(tab, kPartCap, cs, key[k]);
+        if (te) {
+          Row<Sh, NV, false> x;
+          x.q = x.fast = true;
+          x.key = key[k];
+#pragma unroll
+          for (int i = 0; i < NV; ++i) x.vi[i] = v[k][i];
+          cta_add<Sh, NV, false>(p, te, x);
+        } else {
+          uint8_t* ge = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
+          if (ge) update_entry_rec(p, ge, v[k], p.nvals);
+        }
+      }
+    }
+    __syncthreads();
+    if (exclusive) {
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry_excl(p, tab + (size_t)i * cs);
+    } else {
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry(p, tab + (size_t)i * cs);
+    }
+    __syncthreads();
+  }
+}
+
+// ------------------------------------------------------------------ host
+using PShK64 = StaticShape<0, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+using PShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+
+static int part_rec_bytes(int nv) { return nv <= 2 ? 16 : 32; }
+static size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
+
+int part_bits_for(int64_t expected_groups) {
+  int b = 0;
+  while (b < 14 && ((int64_t)kPartCap / 2 << b) < expected_groups) ++b;
+  return b;
+}
+
+static int part_nblk(int sms, int64_t n) {
+  int64_t nb = (int64_t)sms * 4;
+  const int64_t need = (n + 4095) / 4096;
+  return (int)std::max<int64_t>(1, std::min(nb, need));
+}
+
+bool part_eligible(const Plan& p) {
+  if (p.nkeys < 1 || p.nvals > 6 || p.direct) return false;
+  for (int v = 0; v < p.nvals; ++v)
+    if (p.vals[v].is_f64 || p.vals[v].expr != OCL_EXPR_COL) return false;
+  return true;
+}
+
+size_t part_ws_bytes(const Plan& p, int pbits, int sms) {
+  (void)sms;
+  const int64_t L = 1LL << pbits;
+  const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
+  const bool two = pbits > kPartLevelBits;
+  return align_up((size_t)L * 4, 256) * 5 + align_up((size_t)nchunks * 4, 256) * 2 + 512 +
+         align_up((size_t)p.n * part_rec_bytes(p.nvals), 256) * (two ? 2 : 1) + (two ? align_up(4u << kPartLevelBits, 256) : 0);
+}
+
+template <class Sh, int NV>
+static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s) {
+  const size_t hsm = (size_t)4 << a.pbits;
+  auto kc = k_part_count<Sh, NV>;
+  auto ks = k_part_scatter<Sh, NV>;
+  auto ka = k_part_agg<NV>;
+  cudaError_t e;
+  if ((e = cudaFuncSetAttribute(kc, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)hsm))) return e;
+  const size_t tsm = (size_t)kPartCap * p.cta_stride;
+  if ((e = cudaFuncSetAttribute(ka, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)tsm))) return e;
+  const int64_t L = 1LL << a.pbits;
+  const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
+  if ((e = cudaMemsetAsync(a.counts, 0, (size_t)L * 4, s))) return e;
+  count_launch(5);
+  kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
+  k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
+  k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums, nchunks, a.m_dev);
+  k_scan_add<<<(int)((L + 255) / 256), 256, 0, s>>>(a.offs, a.cur, a.sums, L);
+  const int b1 = std::min(a.pbits, kPartLevelBits), b2 = a.pbits - b1;
+  const size_t msm = sizeof(TileMap);
+  auto ks2 = k_part_scatter2<NV>;
+  if ((e = cudaFuncSetAttribute(ks, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
+  if ((e = cudaFuncSetAttribute(ks2, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
+  if (b2 == 0) {
+    ks<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.pbits, a.cur, a.recs);
+  } else {
+    count_launch(3);
+    k_part_cur1<<<((1 << b1) + 255) / 256, 256, 0, s>>>(a.offs, a.cur1, b1, b2);
+    ks<<<a.nblk, kPartThreads, msm, s>>>(p, a, b1, a.cur1, a.tmp);
+    ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
+  }
+  count_launch(4);
+  k_part_items<<<(int)((L + 255) / 256), 256, 0, s>>>(a);
+  k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.icnt, a.ioff, a.isums, L);
+  k_scan_sums<<<1, kScanThreads, 0, s>>>(a.isums, nchunks, a.nitems_dev);
+  k_scan_add<<<(int)((L + 255) / 256), 256, 0, s>>>(a.ioff, a.icnt, a.isums, L);   // icnt := ioff (unused after)
+  int nb = 0;
+  if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, ka, kPartThreads, tsm) != cudaSuccess || nb < 1) nb = 1;
+  const int64_t items = (p.n + kPartItem - 1) / kPartItem + L;
+  const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)sms * nb, items));
+  count_launch();
+  ka<<<(int)grid, kPartThreads, tsm, s>>>(p, a);
+  return cudaGetLastError();
+}
+
+// Run the partitioned tier for plan p (p.table zeroed by the caller).  *kind reports
+// the shape (30 dynamic, 31 key i64, 32 pred i32 + key i64).
+cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind) {
+  if (p.n == 0) return cudaSuccess;
+  PartArgs a;
+  a.pbits = pbits;
+  a.nblk = part_nblk(sms, p.n);
+  a.rows_per_blk = ((p.n + a.nblk - 1) / a.nblk + 127) / 128 * 128;
+  const int64_t L = 1LL << pbits;
+  const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
+  uint8_t* w = (uint8_t*)ws;
+  a.counts = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.offs = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.cur = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.sums = (uint32_t*)w;
+  w += align_up((size_t)nchunks * 4, 256);
+  a.icnt = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.ioff = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.isums = (uint32_t*)w;
+  w += align_up((size_t)nchunks * 4, 256);
+  a.nitems_dev = (int64_t*)w;
+  w += 256;
+  a.m_dev = (int64_t*)w;
+  w += 256;
+  a.rec_bytes = part_rec_bytes(p.nvals);
+  a.recs = w;
+  w += align_up((size_t)p.n * a.rec_bytes, 256);
+  a.tmp = nullptr;
+  a.cur1 = nullptr;
+  if (pbits > kPartLevelBits) {
+    a.tmp = w;
+    w += align_up((size_t)p.n * a.rec_bytes, 256);
+    a.cur1 = (uint32_t*)w;
+  }
+  if (p.vec_ok && p.nkeys == 1 && p.npreds == 0 && values_match<PShK64>(p) && p.keys[0].col.width == 8) {
+    *kind = 31;
+    return part_run<PShK64, 1>(p, a, sms, s);
+  }
+  if (p.vec_ok && p.nkeys == 1 && p.npreds == 1 && p.preds[0].col.width == 4 && !p.preds[0].is_f64 &&
+      values_match<PShP32K64>(p) && p.keys[0].col.width == 8) {
+    *kind = 32;
+    return part_run<PShP32K64, 1>(p, a, sms, s);
+  }
+  *kind = 30;
+  if (p.nvals <= 1) return part_run<DynShape, 1>(p, a, sms, s);
+  if (p.nvals <= 2) return part_run<DynShape, 2>(p, a, sms, s);
+  if (p.nvals <= 4) return part_run<DynShape, 4>(p, a, sms, s);
+  return part_run<DynShape, 6>(p, a, sms, s);
+}
+
+}  // namespace ocl

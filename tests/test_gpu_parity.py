@@ -247,7 +247,7 @@ def test_fused_many_groups(G):
     preds = [(sw["p"], {"hi": 499999})]
     aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
             {"op": "avg", "a": 0}]
-    for tier in (0, 1, 2, 3, 4):
+    for tier in (0, 1, 2, 3, 4, 5):
         _check_sga(preds, [sw["key"]], [sw["v"]], aggs, expected_groups=G, tier=tier)
 
 
@@ -310,7 +310,29 @@ def test_fused_c3_orderkey():
     for shuffled in (False, True):
         li = _lineitem(n, datagen.BASE_SEED + 3, shuffled=shuffled)
         aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
-        _check_sga([], [li["orderkey"]], [li["quantity"]], aggs, expected_groups=n // 4, tier=2)
+        for tier in (2, 5):
+            _check_sga([], [li["orderkey"]], [li["quantity"]], aggs, expected_groups=n // 4, tier=tier)
+
+
+@pytest.mark.parametrize("n", [1, 1000, 70001, 1 << 20])
+def test_fused_partitioned_edges(n):
+    """Hash-partitioned tier (tier 5): ragged sizes, the key ~0, values outside int32 (exact
+    per-row path), several value columns (32-byte records), two keys, a partition holding
+    most rows (heavy hitter), more groups than expected (shared-table overflow)."""
+    rng = np.random.default_rng(n)
+    x = rng.integers(-1000, 1000, n).astype(np.int64)
+    key = rng.integers(0, max(1, n // 3), n).astype(np.int64)
+    key[::11] = -1                                       # ~0: the side entry
+    key[rng.random(n) < 0.4] = 7                         # heavy hitter
+    big = x.copy()
+    big[::13] = 2**40 + 5                                # outside int32: exact per-row path
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
+            {"op": "sum", "a": 1}, {"op": "min", "a": 2}, {"op": "max", "a": 2}, {"op": "avg", "a": 1}]
+    for G in (n // 3 + 2, 8):
+        _check_sga([(x, {"lo": -900})], [key], [x, big, x // 7], aggs, expected_groups=G, tier=5)
+    k32 = (x % 5).astype(np.int32)
+    _check_sga([], [(key & 0x7FFFFFFF).astype(np.int32), k32], [x], [{"op": "count"}, {"op": "sum", "a": 0}], expected_groups=max(8, n // 2), tier=5)
+    _check_sga([(x, {"lo": 5000})], [key], [x], [{"op": "count"}], expected_groups=n + 8, tier=5)   # empty
 
 
 def test_fused_capacity_retry():
