@@ -195,6 +195,8 @@ struct FinPlan {
   int32_t* status;
 };
 
+constexpr uint64_t kProbeWindow = 2048;   // HBM-table probe window (= partition.cu kPartCap)
+
 __device__ __forceinline__ void set_status(int32_t* status, int32_t code) {
   if (status) atomicCAS(status, 0, code);
 }
@@ -217,9 +219,14 @@ __device__ __forceinline__ uint8_t* table_find_or_insert(uint8_t* table, uint64_
   }
   uint64_t sk = ~key;
   // start slot = the top log2(cap) bits of the hash: the keys of hash partition q
-  // (top bits = q, partition.cu) occupy one contiguous slot range
+  // (top bits = q, partition.cu) occupy one contiguous slot range.  Probing wraps
+  // inside the aligned window of kProbeWindow slots holding the start slot, so a
+  // probe sequence never leaves its partition's range (partition.cu stores whole
+  // ranges position by position); at load <= 1/2 a window overflows with
+  // negligible probability, and the capacity status triggers the restart.
+  const uint64_t W = mask < kProbeWindow - 1 ? mask : (uint64_t)(kProbeWindow - 1);
   uint64_t h = __umul64hi(fmix64(key), mask + 1);
-  for (uint64_t probe = 0; probe <= mask; ++probe) {
+  for (uint64_t probe = 0; probe <= W; ++probe) {
     uint64_t* kp = (uint64_t*)(table + h * (uint64_t)stride);
     uint64_t cur = ld_relaxed_u64(kp);
     if (cur == sk) return (uint8_t*)kp;
@@ -227,7 +234,7 @@ __device__ __forceinline__ uint8_t* table_find_or_insert(uint8_t* table, uint64_
       uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
       if (prev == 0 || prev == sk) return (uint8_t*)kp;
     }
-    h = (h + 1) & mask;
+    h = (h & ~W) | ((h + 1) & W);
   }
   set_status(status, OCL_ERR_CAPACITY);
   return nullptr;

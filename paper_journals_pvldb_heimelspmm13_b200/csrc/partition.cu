@@ -34,8 +34,10 @@
 namespace ocl {
 
 constexpr int kPartThreads = 512;
-constexpr int kPartCap = 2048;        // shared-table entries per CTA in pass 2 (power of two)
-constexpr int kPartItem = 16384;      // records per pass-2 work item (< 2^16: split-sum bound of the table)
+constexpr int kPartCapBits = 11;
+constexpr int kPartCap = 1 << kPartCapBits;   // shared-table entries per CTA in pass 2
+static_assert(kPartCap == (int)kProbeWindow, "direct merges need partition ranges = HBM probe windows");
+constexpr int kPartItem = 32768;      // records per pass-2 work item (<= 2^15: 16-bit split sums of the table stay exact)
 constexpr int kPartILP = 4;           // rows / records per thread in flight (part_rows: 2 units x 2 rows)
 constexpr int kTileMapBits = 12;      // scatter: per-tile partition map (2 x the tile's rows)
 constexpr int kPartLevelBits = 7;     // partitions reached per scatter level (tile claims aggregate ~16x)
@@ -60,6 +62,8 @@ struct PartArgs {
   uint32_t* ioff;       // [P] exclusive scan of icnt
   uint32_t* isums;      // scan chunk sums of icnt
   int64_t* nitems_dev;  // number of pass-2 work items
+  uint32_t* slowflag;   // [P] 1: the exact path inserted keys of this partition in pass 1
+  int32_t direct_ok;    // the HBM table's partition regions have exactly kPartCap slots
   int32_t rec_bytes;
 };
 
@@ -302,6 +306,7 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter(const __grid_cons
       if (x[k].q && !ok[k]) {               // exact per-row path straight into the HBM table
         uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
         if (e) update_entry_slow(p, e, part_row(wbase, lane, k));
+        if ((uint64_t)x[k].key != ~0ULL) a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;   // region touched
       }
       if (ok[k]) tile_map_add(map, part_of((uint64_t)x[k].key, pb), slot[k], rank[k]);
     }
@@ -553,10 +558,56 @@ __device__ __forceinline__ void cta_flush_entry_excl(const Plan& p, const uint8_
   }
 }
 
+// Shared-table find-or-insert for pass 2.  In direct mode the start slot and the
+// linear probing (wrapping inside the table) mirror the key's slot range in the HBM
+// table — the table's start slot is the top log2(cap) hash bits and a partition's
+// range has exactly kPartCap slots — so the entries can be stored to the HBM table
+// position by position, without probing it.
+constexpr int kPartProbes = 64;
+
+__device__ __forceinline__ uint8_t* part_find(uint8_t* tab, int32_t cs, uint64_t key, bool direct, int pbits) {
+  const uint64_t sk = ~key;
+  const uint64_t h = fmix64(key);
+  uint32_t i = direct ? (uint32_t)((h << pbits) >> (64 - kPartCapBits)) : (uint32_t)h & (kPartCap - 1);
+  for (int probe = 0; probe < kPartProbes; ++probe) {
+    uint64_t* kp = (uint64_t*)(tab + (size_t)i * cs);
+    const uint64_t cur = *(volatile uint64_t*)kp;
+    if (cur == sk) return (uint8_t*)kp;
+    if (cur == 0) {
+      const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
+      if (prev == 0 || prev == sk) return (uint8_t*)kp;
+    }
+    i = (i + 1) & (kPartCap - 1);
+  }
+  return nullptr;
+}
+
+// Direct merge: shared entry i -> HBM slot region + i (the region holds no entries yet).
+__device__ __forceinline__ void cta_store_entry(const Plan& p, const uint8_t* ce, uint8_t* e) {
+  const uint64_t sk = *(const uint64_t*)ce;
+  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+  if (sk == 0 || cnt == 0) return;
+  *(uint64_t*)e = sk;
+  *(uint64_t*)(e + 8) = cnt;
+  for (int v = 0; v < p.nvals; ++v) {
+    const DevValue& d = p.vals[v];
+    if (d.co_lo >= 0) {
+      const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
+      *(uint64_t*)(e + d.off_sum) = (uint64_t)sum;
+      *(uint64_t*)(e + d.off_sum + 8) = (uint64_t)(sum >> 63);
+    }
+    if (d.co_min >= 0)
+      *(uint64_t*)(e + d.off_min) = enc_min_i((int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u));
+    if (d.co_max >= 0)
+      *(uint64_t*)(e + d.off_max) = enc_max_i((int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u));
+  }
+}
+
 template <int NV>
 __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant__ Plan p, PartArgs a) {
   using Sh = DynShape;
   extern __shared__ __align__(16) uint8_t tab[];
+  __shared__ int overflowed;
   const int lane = threadIdx.x & 31;
   const int64_t m = *a.m_dev;
   const int64_t nitems = *a.nitems_dev;
@@ -574,7 +625,9 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
     const int64_t s = q0 + (item - (int64_t)a.ioff[lo]) * kPartItem;
     const int64_t seg_end = min(q1, s + kPartItem);
     const bool exclusive = q1 - q0 <= kPartItem;
+    const bool direct = a.direct_ok && exclusive && a.slowflag[lo] == 0;
     for (int i = threadIdx.x; i < kPartCap * cs / 16; i += blockDim.x) ((uint4*)tab)[i] = make_uint4(0, 0, 0, 0);
+    if (threadIdx.x == 0) overflowed = 0;
     __syncthreads();
     for (int64_t base = s; base < seg_end; base += kPartILP * blockDim.x) {
       uint64_t key[kPartILP];
@@ -593,7 +646,7 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
       for (int k = 0; k < kPartILP; ++k) {
         const uint64_t k0 = __shfl_sync(0xffffffffu, key[k], 0);
         if (__all_sync(0xffffffffu, valid[k] && key[k] == k0)) {    // heavy hitter: one update per warp
-          uint8_t* te = lane == 0 ? cta_find_or_insert(tab, kPartCap, cs, k0) : nullptr;
+          uint8_t* te = lane == 0 ? part_find(tab, cs, k0, direct, a.pbits) : nullptr;
           const unsigned long long tp = __shfl_sync(0xffffffffu, (unsigned long long)te, 0);
           if (tp) {
             cta_add_warp<NV>(p, (uint8_t*)tp, v[k], lane);
@@ -601,7 +654,7 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
           }
         }
         if (!valid[k]) continue;
-        uint8_t* te = cta_find_or_insert(tab, kPartCap, cs, key[k]);
+        uint8_t* te = part_find(tab, cs, key[k], direct, a.pbits);
         if (te) {
           Row<Sh, NV, false> x;
           x.q = x.fast = true;
@@ -610,13 +663,18 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
           for (int i = 0; i < NV; ++i) x.vi[i] = v[k][i];
           cta_add<Sh, NV, false>(p, te, x);
         } else {
+          overflowed = 1;
           uint8_t* ge = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
           if (ge) update_entry_rec(p, ge, v[k], p.nvals);
         }
       }
     }
     __syncthreads();
-    if (exclusive) {
+    if (direct && !overflowed) {
+      uint8_t* region = p.table + ((size_t)lo << kPartCapBits) * p.stride;
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x)
+        cta_store_entry(p, tab + (size_t)i * cs, region + (size_t)i * p.stride);
+    } else if (exclusive) {
       for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry_excl(p, tab + (size_t)i * cs);
     } else {
       for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry(p, tab + (size_t)i * cs);
@@ -656,7 +714,7 @@ size_t part_ws_bytes(const Plan& p, int pbits, int sms) {
   const int64_t L = 1LL << pbits;
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   const bool two = pbits > kPartLevelBits;
-  return align_up((size_t)L * 4, 256) * 5 + align_up((size_t)nchunks * 4, 256) * 2 + 512 +
+  return align_up((size_t)L * 4, 256) * 6 + align_up((size_t)nchunks * 4, 256) * 2 + 512 +
          align_up((size_t)p.n * part_rec_bytes(p.nvals), 256) * (two ? 2 : 1) + (two ? align_up(4u << kPartLevelBits, 256) : 0);
 }
 
@@ -673,6 +731,7 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s) 
   const int64_t L = 1LL << a.pbits;
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   if ((e = cudaMemsetAsync(a.counts, 0, (size_t)L * 4, s))) return e;
+  if ((e = cudaMemsetAsync(a.slowflag, 0, (size_t)L * 4, s))) return e;
   count_launch(5);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
   k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
@@ -732,6 +791,9 @@ cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cuda
   w += align_up((size_t)nchunks * 4, 256);
   a.nitems_dev = (int64_t*)w;
   w += 256;
+  a.slowflag = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.direct_ok = ((p.mask + 1) >> pbits) == (uint64_t)kPartCap ? 1 : 0;
   a.m_dev = (int64_t*)w;
   w += 256;
   a.rec_bytes = part_rec_bytes(p.nvals);
