@@ -61,7 +61,7 @@ def lib():
         L.oracle_compact.argtypes = [P, ctypes.c_int64, P]
         L.oracle_compact.restype = ctypes.c_int64
         L.oracle_gather.argtypes = [P, P, ctypes.c_int64, P]
-        for f in (L.oracle_group_hash, L.oracle_group_sort):
+        for f in (L.oracle_group_hash, L.oracle_group_sort, L.oracle_group_sorted):
             f.argtypes = [P, ctypes.c_int, P, ctypes.c_int64, P, P]
             f.restype = ctypes.c_int64
         L.oracle_aggregate.argtypes = [P, P, ctypes.c_int64, ctypes.c_int64, P, ctypes.c_int, P, ctypes.c_int]
@@ -177,6 +177,8 @@ def _group(fn, keys, oids, m):
     gids = np.zeros(max(m, 1), np.int32)
     keys_out = np.zeros(max(m, 1), np.int64)
     G = fn(cols, len(keys), None if oids is None else oids.ctypes.data, m, gids.ctypes.data, keys_out.ctypes.data)
+    if G == -2:
+        raise ValueError("keys not sorted (non-decreasing packed key required)")
     if G < 0:
         raise ValueError("invalid group spec")
     return gids[:m].copy(), keys_out[:G].copy()
@@ -190,6 +192,11 @@ def group_hash(keys, oids=None, m=None):
 def group_sort(keys, oids=None, m=None):
     """Independent sort-based grouping; must equal group_hash exactly."""
     return _group(lib().oracle_group_sort, keys, oids, len(keys[0]) if m is None else m)
+
+
+def group_sorted(keys, oids=None, m=None):
+    """The paper's sorted-input grouping (successor compare + prefix sum, L554-556); raises on unsorted keys."""
+    return _group(lib().oracle_group_sorted, keys, oids, len(keys[0]) if m is None else m)
 
 
 def aggregate(gids, G, vals, aggs, oids=None):

@@ -227,6 +227,32 @@ int64_t oracle_group_sort(const orc_column* keys, int nkeys, const uint32_t* oid
   return (int64_t)runs.size();
 }
 
+// Sorted-input group-by, the paper's first algorithm (§4.1.6):
+// "If the input is sorted, we identify group boundaries by having each thread
+// compare its value with its successor. Then, a prefix sum operation is used to
+// generate dense group IDs."  Step 1: boundary[j] = 1 if key(j) != key(j+1)
+// (successor compare; the last row ends a group).  Step 2: exclusive prefix sum
+// of the boundaries gives gid[j] = number of group ends before row j.  Sorted
+// means non-decreasing packed key (unsigned 64-bit order); returns -2 if a row's
+// key is smaller than its predecessor's (nothing else is then guaranteed).
+int64_t oracle_group_sorted(const orc_column* keys, int nkeys, const uint32_t* oids, int64_t m,
+                            int32_t* gids, int64_t* keys_out) {
+  if (!keys_valid(keys, nkeys)) return -1;
+  std::vector<uint64_t> k((size_t)m);
+  for (int64_t j = 0; j < m; ++j) k[(size_t)j] = packed_key(keys, nkeys, oids ? (int64_t)oids[j] : j);
+  for (int64_t j = 1; j < m; ++j)
+    if (k[(size_t)j] < k[(size_t)j - 1]) return -2;
+  std::vector<int64_t> boundary((size_t)m);
+  for (int64_t j = 0; j < m; ++j) boundary[(size_t)j] = (j == m - 1 || k[(size_t)j] != k[(size_t)j + 1]) ? 1 : 0;
+  int64_t prefix = 0;                       // exclusive prefix sum of the boundaries
+  for (int64_t j = 0; j < m; ++j) {
+    gids[j] = (int32_t)prefix;
+    if (keys_out && boundary[(size_t)j]) keys_out[prefix] = (int64_t)k[(size_t)j];
+    prefix += boundary[(size_t)j];
+  }
+  return prefix;
+}
+
 int oracle_aggregate(const int32_t* gids, const uint32_t* oids, int64_t m, int64_t G,
                      const orc_column* vals, int nvals, const orc_agg* aggs, int naggs) {
   for (int i = 0; i < naggs; ++i)

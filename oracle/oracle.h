@@ -76,6 +76,12 @@ int64_t oracle_group_hash(const orc_column* keys, int nkeys, const uint32_t* oid
  * min j of each run.  Must equal oracle_group_hash exactly. */
 int64_t oracle_group_sort(const orc_column* keys, int nkeys, const uint32_t* oids, int64_t m,
                           int32_t* gids, int64_t* keys_out);
+/* a4, sorted input (L554-556 §4.1.6): successor compare marks group ends, an
+ * exclusive prefix sum of the marks is the dense gid (group g = g-th distinct key
+ * in row order).  Returns G, -1 on invalid key spec, -2 if the packed key
+ * (unsigned) decreases anywhere (input not sorted). */
+int64_t oracle_group_sorted(const orc_column* keys, int nkeys, const uint32_t* oids, int64_t m,
+                            int32_t* gids, int64_t* keys_out);
 /* a7-a8 (L562-568): per group g in [0,G):
  *   COUNT -> int64;  SUM over int64 (expr values in int128, wrapping mod 2^128)
  *   -> 16 bytes {uint64 lo, int64 hi};  SUM over f64 -> double (Neumaier

@@ -326,3 +326,49 @@ def test_sga_ungrouped():
     v = np.arange(10, dtype=np.int64)
     keys, outs = oracle.sga([(v, {"lo": 3})], [], [v], [{"op": "sum", "a": 0}, {"op": "count"}])
     assert keys.tolist() == [0] and int128_list(outs[0]) == [42] and outs[1].tolist() == [7]
+
+
+# ---------------------------------------------------------------- sorted-input grouping
+def _py_distinct_prefix(keys):
+    """Brute force for sorted keys: gid[j] = (number of distinct keys among rows 0..j) - 1."""
+    seen, out = set(), []
+    for k in keys:
+        seen.add(int(k))
+        out.append(len(seen) - 1)
+    return out
+
+
+@pytest.mark.parametrize("n", [0, 1, 2, 7, 64, 257, 3000])
+def test_group_sorted_brute_force_and_hash(n):
+    rng = np.random.default_rng(1000 + n)
+    keys = np.sort(rng.integers(0, max(n // 3, 1), n)).astype(np.int64)
+    gids, kout = oracle.group_sorted([keys])
+    assert gids.tolist() == _py_distinct_prefix(keys)
+    assert kout.tolist() == sorted(set(keys.tolist()))                  # ascending, one per group
+    hg, hk = oracle.group_hash([keys])                                   # first occurrence == run order
+    assert gids.tolist() == hg.tolist() and kout.tolist() == hk.tolist()
+
+
+def test_group_sorted_two_columns_and_oids():
+    rng = np.random.default_rng(7)
+    a = np.sort(rng.integers(0, 5, 500)).astype(np.uint8)               # sorted (a, b) pairs
+    b = np.concatenate([np.sort(rng.integers(0, 4, int((a == v).sum()))) for v in range(5)]).astype(np.uint8)
+    oids = np.flatnonzero(rng.random(500) < 0.3).astype(np.uint32)       # a subsequence stays sorted
+    gids, kout = oracle.group_sorted([a, b], oids)
+    packed = [(int(a[o]) << 8) | int(b[o]) for o in oids]
+    assert gids.tolist() == _py_distinct_prefix(packed)
+    assert kout.tolist() == sorted(set(packed))
+
+
+def test_group_sorted_degenerate_and_unsorted():
+    one = np.full(100, 42, np.int64)
+    gids, kout = oracle.group_sorted([one])
+    assert gids.tolist() == [0] * 100 and kout.tolist() == [42]
+    distinct = np.arange(50, dtype=np.int32)
+    gids, kout = oracle.group_sorted([distinct])
+    assert gids.tolist() == list(range(50)) and kout.tolist() == list(range(50))
+    with pytest.raises(ValueError, match="not sorted"):
+        oracle.group_sorted([np.array([1, 2, 1], np.int64)])
+    # unsigned packed order: -1 (all ones) sorts after every non-negative key
+    gids, kout = oracle.group_sorted([np.array([0, 5, -1, -1], np.int64)])
+    assert gids.tolist() == [0, 1, 2, 2]
