@@ -64,7 +64,8 @@ class SgaArgs(ctypes.Structure):
                 ("nvals", ctypes.c_int32), ("naggs", ctypes.c_int32), ("aggs", ctypes.c_void_p),
                 ("expected_groups", ctypes.c_int64), ("out_capacity", ctypes.c_int64),
                 ("keys_out", ctypes.c_void_p), ("ngroups_out", ctypes.c_void_p), ("bitmap_out", ctypes.c_void_p),
-                ("dev_status", ctypes.c_void_p), ("order_by_key", ctypes.c_int32), ("tier", ctypes.c_int32)]
+                ("dev_status", ctypes.c_void_p), ("order_by_key", ctypes.c_int32), ("tier", ctypes.c_int32),
+                ("key_sorted", ctypes.c_int32), ("reserved_", ctypes.c_int32)]
 
 
 _lib = None
@@ -89,6 +90,8 @@ def lib():
             "ocl_gather": [P, P, P, P, I64, P, P],
             "ocl_group_build_workspace_size": [P, I64, I64, PSZ],
             "ocl_group_build": [P, P, I32, P, P, I64, I64, P, P, I64, P, P, P, SZ, P],
+            "ocl_group_build_sorted_workspace_size": [P, I64, PSZ],
+            "ocl_group_build_sorted": [P, P, I32, P, P, I64, P, P, I64, P, P, P, SZ, P],
             "ocl_group_aggregate_workspace_size": [P, I64, P, I32, P, I32, PSZ],
             "ocl_group_aggregate": [P, P, P, P, I64, P, I64, P, I32, P, I32, P, SZ, P],
             "ocl_select_group_aggregate_workspace_size": [P, P, PSZ],
@@ -120,6 +123,7 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_launch_count", "ocl_ctx_last_kernel", "ocl_ctx_set_kernel_events",
                "ocl_select_bitmap", "ocl_bitmap_combine", "ocl_prefix_compact_workspace_size", "ocl_prefix_compact",
                "ocl_gather", "ocl_group_build_workspace_size", "ocl_group_build",
+               "ocl_group_build_sorted_workspace_size", "ocl_group_build_sorted",
                "ocl_group_aggregate_workspace_size", "ocl_group_aggregate",
                "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate", "ocl_partial_row_bytes",
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
@@ -303,6 +307,28 @@ def group_build(keys, oids=None, m=None, max_rows=None, expected_groups=1024, ou
     return gids, keys_out, ng, status
 
 
+def group_build_sorted(keys, oids=None, m=None, max_rows=None, out_capacity=None, stream=None):
+    """Sorted-input group-by (successor compare + prefix sum) -> (gids int32[max_rows],
+    keys_out int64[cap], ngroups int64[1], status int32[1]); gids ascend with the key."""
+    dev = keys[0].device
+    ctx = context(dev)
+    max_rows = (oids.numel() if oids is not None else keys[0].numel()) if max_rows is None else max_rows
+    out_capacity = max_rows if out_capacity is None else out_capacity
+    sz = ctypes.c_size_t()
+    _check(lib().ocl_group_build_sorted_workspace_size(ctx.handle, max_rows, ctypes.byref(sz)))
+    ws = _workspace(sz.value, dev)
+    gids = torch.empty(max(max_rows, 1), dtype=torch.int32, device=dev)
+    keys_out = torch.empty(max(out_capacity, 1), dtype=torch.int64, device=dev)
+    ng = torch.zeros(1, dtype=torch.int64, device=dev)
+    status = torch.zeros(1, dtype=torch.int32, device=dev)
+    kc = _cols(keys)
+    _check(lib().ocl_group_build_sorted(ctx.handle, kc, len(keys), None if oids is None else oids.data_ptr(),
+                                        None if m is None else m.data_ptr(), max_rows, gids.data_ptr(),
+                                        keys_out.data_ptr(), out_capacity, ng.data_ptr(), status.data_ptr(),
+                                        ws.data_ptr(), sz.value, _stream(stream)))
+    return gids, keys_out, ng, status
+
+
 # ---------------------------------------------------------------- a7-a8
 def group_aggregate(gids, ngroups, max_groups, vals, aggs, oids=None, m=None, max_rows=None, stream=None):
     """Grouped aggregation over dense gids -> list of per-aggregate outputs [max_groups]."""
@@ -328,7 +354,7 @@ class SgaCall:
     across launches (the benchmark times only ``launch``)."""
 
     def __init__(self, preds, keys, vals, aggs, expected_groups=1024, out_capacity=None, order_by_key=False,
-                 bitmap=False, tier=0, host=False, chunk_rows=1 << 24, device=None):
+                 bitmap=False, tier=0, host=False, chunk_rows=1 << 24, device=None, key_sorted=False):
         cols = [p[0] for p in preds] + list(keys) + list(vals)
         self.host = host
         self.device = torch.device(device) if device is not None else (
@@ -365,6 +391,7 @@ class SgaCall:
         a.bitmap_out = self.bitmap.data_ptr() if bitmap else None
         a.dev_status = self.status.data_ptr()
         a.order_by_key, a.tier = int(bool(order_by_key)), int(tier)
+        a.key_sorted = int(bool(key_sorted))
         self.args = a
         self.chunk_rows = int(chunk_rows)
         sz = ctypes.c_size_t()
@@ -396,14 +423,16 @@ class SgaCall:
 
 
 def select_group_aggregate(preds, keys, vals, aggs, expected_groups=4, out_capacity=None, order_by_key=False,
-                           bitmap=False, tier=0, stream=None, max_retries=8):
+                           bitmap=False, tier=0, stream=None, max_retries=8, key_sorted=False):
     """Fused select -> group -> aggregate, blocking, with the paper's restart-with-a-larger-table on overflow
     (P:L523-527).  preds = [(column, range_spec)], keys = [column], vals = [column].
+    key_sorted=True: the packed key column is sorted -> sort-based grouping, output in key
+    order; an unsorted key column raises OcelotError(OCL_ERR_INVALID_ARG).
     Returns (keys_out[G], [outputs[G]], bitmap or None)."""
     eg = expected_groups
     for _ in range(max_retries):
         call = SgaCall(preds, keys, vals, aggs, expected_groups=eg, out_capacity=out_capacity,
-                       order_by_key=order_by_key, bitmap=bitmap, tier=tier)
+                       order_by_key=order_by_key, bitmap=bitmap, tier=tier, key_sorted=key_sorted)
         call.launch(stream)
         try:
             k, o = call.result()

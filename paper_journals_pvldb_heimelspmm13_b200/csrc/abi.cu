@@ -117,6 +117,7 @@ struct Planned {
   uint64_t cap;      // table capacity (power of two)
   size_t table_bytes;
   int32_t pbits;     // >= 0: hash-partitioned high-cardinality tier with 2^pbits partitions (partition.cu)
+  bool sorted;       // sort-based grouping of sorted input (sorted.cu)
 };
 
 ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* aggs, int32_t naggs, Planned* P) {
@@ -385,13 +386,20 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   P->pbits = -1;
   const bool many = a->tier == 0 && p.smem_cap == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
   if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
+  P->sorted = a->key_sorted != 0;
+  if (P->sorted) {
+    if (a->tier != 0) return fail(OCL_ERR_INVALID_ARG, "key_sorted needs tier 0");
+    if (a->nkeys == 0) return fail(OCL_ERR_INVALID_ARG, "key_sorted needs a key column");
+    P->pbits = -1;
+    P->table_bytes = 0;
+  }
   FinPlan& f = P->fin;
   f.order_by_key = a->order_by_key ? 1 : 0;
   f.keys_out = a->keys_out;
   f.ngroups_out = a->ngroups_out;
   f.out_capacity = a->out_capacity;
   f.status = a->dev_status;
-  if (a->order_by_key && !sorted_emit_supported(P->cap))
+  if (a->order_by_key && !P->sorted && !sorted_emit_supported(P->cap))
     return fail(OCL_ERR_UNSUPPORTED, "order_by_key needs expected_groups <= 2047 (table of %llu slots)", (unsigned long long)P->cap);
   return OCL_OK;
 }
@@ -399,6 +407,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
 
 // table + finalize workspace of a fused call
 size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) {
+  if (P.sorted) return sorted_ws_bytes(P.plan);
   return P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256) +
          (P.pbits >= 0 ? part_ws_bytes(P.plan, P.pbits, ctx->sms) : 0);
 }
@@ -604,6 +613,42 @@ ocl_status ocl_group_build(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, 
   return OCL_OK;
 }
 
+ocl_status ocl_group_build_sorted_workspace_size(ocl_ctx* ctx, int64_t max_rows, size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (max_rows < 0 || max_rows > ((int64_t)1 << 31)) return fail(OCL_ERR_UNSUPPORTED, "max_rows outside [0, 2^31]");
+  *bytes = group_build_sorted_ws_bytes(max_rows);
+  return OCL_OK;
+}
+
+ocl_status ocl_group_build_sorted(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, const uint32_t* oids,
+                                  const int64_t* m_dev, int64_t max_rows, int32_t* gid_out, int64_t* keys_out,
+                                  int64_t out_capacity, int64_t* ngroups_out, int32_t* dev_status, void* ws,
+                                  size_t ws_bytes, void* stream) {
+  if (!ctx || !ngroups_out) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/ngroups_out");
+  if (nkeys < 1) return fail(OCL_ERR_INVALID_ARG, "nkeys=%d (1..2)", nkeys);
+  if (out_capacity < 0) return fail(OCL_ERR_INVALID_ARG, "out_capacity < 0");
+  size_t need = 0;
+  ocl_status s = ocl_group_build_sorted_workspace_size(ctx, max_rows, &need);
+  if (s) return s;
+  if (max_rows > 0 && !gid_out) return fail(OCL_ERR_INVALID_ARG, "NULL gid_out");
+  Plan p;
+  memset(&p, 0, sizeof(p));
+  if ((s = plan_keys(keys, nkeys, p))) return s;
+  if (!oids)
+    for (int i = 0; i < nkeys; ++i)
+      if (keys[i].n < max_rows) return fail(OCL_ERR_INVALID_ARG, "key column shorter than max_rows");
+  if (max_rows > 0 && (!ws || ws_bytes < need)) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  cudaStream_t st = (cudaStream_t)stream;
+  p.status = dev_status;
+  p.oids = oids;
+  p.m_dev = m_dev;
+  p.n = max_rows;
+  if (dev_status) OCL_CUDA(cudaMemsetAsync(dev_status, 0, 4, st), "status init");
+  OCL_CUDA(launch_group_build_sorted(p, gid_out, keys_out, out_capacity, ngroups_out, ws, ctx->sms, st),
+           "sorted group build");
+  return OCL_OK;
+}
+
 // ---------------------------------------------------------------- a7-a8
 ocl_status ocl_group_aggregate_workspace_size(ocl_ctx* ctx, int64_t max_groups, const ocl_column* vals, int32_t nvals,
                                               const ocl_agg* aggs, int32_t naggs, size_t* bytes) {
@@ -668,6 +713,18 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
   ocl_status s = plan_sga(args, &P);
   if (s) return s;
   cudaStream_t st = (cudaStream_t)stream;
+  if (P.sorted) {                 // sort-based grouping: no table, outputs written by the kernels
+    size_t need = sga_ws_bytes(ctx, P);
+    if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+    if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, sizeof(int32_t), st), "status init");
+    if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, st), "profile event");
+    int kind = 0;
+    OCL_CUDA(launch_sorted(P.plan, P.fin, P.values_f64, ws, args->dev_status, args->ngroups_out, args->out_capacity,
+                           ctx->sms, st, &kind), "sorted group-by launch");
+    ctx->last_kernel = kind;
+    if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, st), "profile event");
+    return OCL_OK;
+  }
   void* ews = nullptr;
   if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
   EmitArgs ea;
@@ -696,6 +753,7 @@ ocl_status ocl_sga_partial(ocl_ctx* ctx, const ocl_sga_args* args, void* partial
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
+  if (P.sorted) return fail(OCL_ERR_UNSUPPORTED, "key_sorted partial tables (multi-GPU) are not implemented");
   cudaStream_t st = (cudaStream_t)stream;
   void* ews = nullptr;
   if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
@@ -807,6 +865,7 @@ ocl_status ocl_select_group_aggregate_host_workspace_size(ocl_ctx* ctx, const oc
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
+  if (P.sorted) return fail(OCL_ERR_UNSUPPORTED, "key_sorted is not available on the host-buffer path");
   P.pbits = -1;             // chunks stream through the one-pass fused kernel
   HostCols h;
   collect_host_cols(P, h, chunk_rows);

@@ -282,21 +282,6 @@ using ShQ1I = StaticShape<4, false, 1, 1, 4, false, vop(0, VF_SUM, 0), vop(0, VF
                           vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
 using ShQ1F = StaticShape<4, false, 1, 1, 4, true, vop(0, VF_SUM, 0), vop(0, VF_SUM, 1), vop(1, VF_SUM, 1, 2),
                           vop(2, VF_SUM, 1, 2, 3), vop(0, VF_SUM, 2)>;
-// GROUP BY an i64 key, COUNT/SUM/MIN/MAX of one i64 column (config C3), and the same
-// behind an i32 range predicate (config C5).
-using ShK64 = StaticShape<0, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
-using ShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
-
-template <class Sh>
-static bool shape_match(const Plan& g) {
-  if (g.npreds != Sh::np(g) || g.nkeys != Sh::nk(g)) return false;
-  for (int i = 0; i < g.npreds; ++i)
-    if (g.preds[i].col.width != Sh::pw(g, i) || (bool)g.preds[i].is_f64 != Sh::pf64(g, i)) return false;
-  for (int i = 0; i < g.nkeys; ++i)
-    if (g.keys[i].col.width != Sh::kw(g, i)) return false;
-  return values_match<Sh>(g);
-}
-
 // ------------------------------------------------------------------ dispatch
 static size_t reg_smem(const Plan& p) {
   return (size_t)kRegSlots * p.priv_rec * kFusedThreads + (size_t)p.smem_cap * p.cta_stride;
@@ -401,6 +386,9 @@ const char* fused_kernel_name(int kind) {
     case 30: return "k_part_count/scatter/agg<DynShape> (hash-partitioned)";
     case 31: return "k_part_count/scatter/agg<StaticShape key i64> (hash-partitioned)";
     case 32: return "k_part_count/scatter/agg<StaticShape pred i32, key i64> (hash-partitioned)";
+    case 40: return "k_sorted_summary/scan/agg<DynShape> (sorted input)";
+    case 41: return "k_sorted_summary/scan/agg<StaticShape key i64> (sorted input)";
+    case 42: return "k_sorted_summary/scan/agg<StaticShape pred i32, key i64> (sorted input)";
     default: return "k_sga<DynShape>";
   }
 }

@@ -65,4 +65,11 @@ bool part_eligible(const Plan& p);
 int part_bits_for(int64_t expected_groups);
 size_t part_ws_bytes(const Plan& p, int pbits, int sms);
 cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind);
+// Sorted-input GROUP BY (sorted.cu).
+size_t sorted_ws_bytes(const Plan& p);
+cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, void* ws, int32_t* status,
+                          int64_t* ngroups_out, int64_t out_capacity, int sms, cudaStream_t s, int* kind);
+size_t group_build_sorted_ws_bytes(int64_t max_rows);
+cudaError_t launch_group_build_sorted(const Plan& p, int32_t* gid_out, int64_t* keys_out, int64_t out_capacity,
+                                      int64_t* ngroups, void* ws, int sms, cudaStream_t s);
 }  // namespace ocl

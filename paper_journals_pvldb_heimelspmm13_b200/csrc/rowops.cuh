@@ -173,4 +173,39 @@ __device__ __forceinline__ void emit_bitmap_unit(const Plan& p, int64_t base, in
   if (lane == 1 && wi + 1 < words) p.bitmap_out[wi + 1] = w1;
 }
 
+// Finalisation (§4.1.7: one thread per group computes the final aggregate).
+// Decode one entry into output row g (finalize).
+__device__ __forceinline__ void emit_final(const FinPlan& f, const uint8_t* e, uint64_t key, int64_t g) {
+  if (g >= f.out_capacity) return;
+  if (f.keys_out) f.keys_out[g] = (int64_t)key;
+  const uint64_t count = *(const uint64_t*)(e + 8);
+  for (int i = 0; i < f.naggs; ++i) {
+    const OutAgg& a = f.aggs[i];
+    const uint8_t* s = e + a.off;
+    switch (a.op) {
+      case OCL_AGG_COUNT: ((int64_t*)a.out)[g] = (int64_t)count; break;
+      case OCL_AGG_SUM:
+        if (a.is_f64) ((double*)a.out)[g] = *(const double*)s;
+        else {
+          ((uint64_t*)a.out)[2 * g] = *(const uint64_t*)s;
+          ((uint64_t*)a.out)[2 * g + 1] = *(const uint64_t*)(s + 8);
+        }
+        break;
+      case OCL_AGG_AVG: {
+        double sum = a.is_f64 ? *(const double*)s : i128_to_double(*(const uint64_t*)s, *(const uint64_t*)(s + 8));
+        ((double*)a.out)[g] = __ddiv_rn(sum, __ull2double_rn(count));
+        break;
+      }
+      case OCL_AGG_MIN:
+        if (a.is_f64) ((double*)a.out)[g] = dec_min_f(*(const uint64_t*)s);
+        else ((int64_t*)a.out)[g] = dec_min_i(*(const uint64_t*)s);
+        break;
+      case OCL_AGG_MAX:
+        if (a.is_f64) ((double*)a.out)[g] = dec_max_f(*(const uint64_t*)s);
+        else ((int64_t*)a.out)[g] = dec_max_i(*(const uint64_t*)s);
+        break;
+    }
+  }
+}
+
 }  // namespace ocl

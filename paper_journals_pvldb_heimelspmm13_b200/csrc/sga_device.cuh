@@ -708,4 +708,20 @@ inline bool values_match(const Plan& g) {
   return true;
 }
 
+// GROUP BY an i64 key, COUNT/SUM/MIN/MAX of one i64 column (config C3), and the same
+// behind an i32 range predicate (config C5).
+using ShK64 = StaticShape<0, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+using ShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
+
+// Whole plan (predicate / key widths + values) equals the compile-time shape Sh.
+template <class Sh>
+inline bool shape_match(const Plan& g) {
+  if (g.npreds != Sh::np(g) || g.nkeys != Sh::nk(g)) return false;
+  for (int i = 0; i < g.npreds; ++i)
+    if (g.preds[i].col.width != Sh::pw(g, i) || (bool)g.preds[i].is_f64 != Sh::pf64(g, i)) return false;
+  for (int i = 0; i < g.nkeys; ++i)
+    if (g.keys[i].col.width != Sh::kw(g, i)) return false;
+  return values_match<Sh>(g);
+}
+
 }  // namespace ocl

@@ -22,40 +22,6 @@ __device__ __forceinline__ uint64_t slot_key(const uint8_t* table, uint64_t cap,
 }
 
 // ------------------------------------------------------------------ emitters
-// Decode one entry into output row g (finalize).
-__device__ __forceinline__ void emit_final(const FinPlan& f, const uint8_t* e, uint64_t key, int64_t g) {
-  if (g >= f.out_capacity) return;
-  if (f.keys_out) f.keys_out[g] = (int64_t)key;
-  const uint64_t count = *(const uint64_t*)(e + 8);
-  for (int i = 0; i < f.naggs; ++i) {
-    const OutAgg& a = f.aggs[i];
-    const uint8_t* s = e + a.off;
-    switch (a.op) {
-      case OCL_AGG_COUNT: ((int64_t*)a.out)[g] = (int64_t)count; break;
-      case OCL_AGG_SUM:
-        if (a.is_f64) ((double*)a.out)[g] = *(const double*)s;
-        else {
-          ((uint64_t*)a.out)[2 * g] = *(const uint64_t*)s;
-          ((uint64_t*)a.out)[2 * g + 1] = *(const uint64_t*)(s + 8);
-        }
-        break;
-      case OCL_AGG_AVG: {
-        double sum = a.is_f64 ? *(const double*)s : i128_to_double(*(const uint64_t*)s, *(const uint64_t*)(s + 8));
-        ((double*)a.out)[g] = __ddiv_rn(sum, __ull2double_rn(count));
-        break;
-      }
-      case OCL_AGG_MIN:
-        if (a.is_f64) ((double*)a.out)[g] = dec_min_f(*(const uint64_t*)s);
-        else ((int64_t*)a.out)[g] = dec_min_i(*(const uint64_t*)s);
-        break;
-      case OCL_AGG_MAX:
-        if (a.is_f64) ((double*)a.out)[g] = dec_max_f(*(const uint64_t*)s);
-        else ((int64_t*)a.out)[g] = dec_max_i(*(const uint64_t*)s);
-        break;
-    }
-  }
-}
-
 __device__ __forceinline__ void emit_slot(const EmitArgs& a, uint8_t* e, uint64_t key, int64_t g, int32_t stride) {
   if (a.kind == EMIT_FINAL) {
     emit_final(a.fin, e, key, g);
