@@ -100,6 +100,8 @@ def lib():
             "ocl_sga_partial": [P, P, P, I64, P, P, SZ, P],
             "ocl_merge_partials_workspace_size": [P, P, I32, I64, PSZ],
             "ocl_merge_partials": [P, P, P, I32, I64, P, P, SZ, P],
+            "ocl_route_partials_workspace_size": [P, I32, PSZ],
+            "ocl_route_partials": [P, P, P, I64, I32, I32, P, P, P, SZ, P],
             "ocl_select_group_aggregate_host_workspace_size": [P, P, I64, PSZ],
             "ocl_select_group_aggregate_host": [P, P, I64, P, SZ, P],
         }
@@ -127,6 +129,7 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_group_aggregate_workspace_size", "ocl_group_aggregate",
                "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate", "ocl_partial_row_bytes",
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
+               "ocl_route_partials_workspace_size", "ocl_route_partials",
                "ocl_select_group_aggregate_host_workspace_size", "ocl_select_group_aggregate_host")
 
 
@@ -481,6 +484,21 @@ def merge_partials(call, partials, counts, nparts, part_capacity, stream=None):
     ws = _workspace(sz.value, call.device)
     _check(lib().ocl_merge_partials(call.ctx.handle, ctypes.byref(call.args), partials.data_ptr(), nparts,
                                     part_capacity, counts.data_ptr(), ws.data_ptr(), sz.value, _stream(stream)))
+
+
+def route_partials(part, cnt, nparts, stream=None):
+    """Hash-route partial rows (uint8[cap, row_bytes], device count int64[1]) to nparts destinations
+    -> (rows grouped by destination uint8[cap, row_bytes], per-destination counts int64[nparts])."""
+    ctx = context(part.device)
+    cap, rb = part.shape
+    sz = ctypes.c_size_t()
+    _check(lib().ocl_route_partials_workspace_size(ctx.handle, nparts, ctypes.byref(sz)))
+    ws = _workspace(sz.value, part.device)
+    out = torch.empty_like(part)
+    counts = torch.zeros(nparts, dtype=torch.int64, device=part.device)
+    _check(lib().ocl_route_partials(ctx.handle, part.data_ptr(), cnt.data_ptr(), cap, rb, nparts, out.data_ptr(),
+                                    counts.data_ptr(), ws.data_ptr(), sz.value, _stream(stream)))
+    return out, counts
 
 
 from .distributed import distributed_select_group_aggregate, shard_range  # noqa: E402,F401

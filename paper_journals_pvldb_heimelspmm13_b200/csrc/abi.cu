@@ -815,6 +815,29 @@ ocl_status ocl_merge_partials(ocl_ctx* ctx, const ocl_sga_args* args, const void
   return OCL_OK;
 }
 
+ocl_status ocl_route_partials_workspace_size(ocl_ctx* ctx, int32_t nparts, size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (nparts < 1 || nparts > route_max_parts()) return fail(OCL_ERR_INVALID_ARG, "nparts=%d (1..%d)", nparts, route_max_parts());
+  *bytes = route_ws_bytes(nparts);
+  return OCL_OK;
+}
+
+ocl_status ocl_route_partials(ocl_ctx* ctx, const void* rows, const int64_t* nrows_dev, int64_t max_rows,
+                              int32_t row_bytes, int32_t nparts, void* out, int64_t* part_counts, void* ws,
+                              size_t ws_bytes, void* stream) {
+  size_t need = 0;
+  ocl_status s = ocl_route_partials_workspace_size(ctx, nparts, &need);
+  if (s) return s;
+  if (max_rows < 0) return fail(OCL_ERR_INVALID_ARG, "max_rows < 0");
+  if (row_bytes < 16 || row_bytes % 8) return fail(OCL_ERR_INVALID_ARG, "row_bytes=%d (multiple of 8, >= 16)", row_bytes);
+  if (!part_counts || !ws) return fail(OCL_ERR_INVALID_ARG, "NULL part_counts/ws");
+  if (max_rows > 0 && (!rows || !out)) return fail(OCL_ERR_INVALID_ARG, "NULL rows/out");
+  if (ws_bytes < need) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  OCL_CUDA(launch_route(rows, nrows_dev, max_rows, row_bytes, nparts, out, part_counts, ws, ctx->sms,
+                        (cudaStream_t)stream), "route partials");
+  return OCL_OK;
+}
+
 // ---------------------------------------------------------------- end to end from host buffers
 namespace {
 struct HostCols {

@@ -65,6 +65,11 @@ bool part_eligible(const Plan& p);
 int part_bits_for(int64_t expected_groups);
 size_t part_ws_bytes(const Plan& p, int pbits, int sms);
 cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind);
+// Hash routing of partial rows for the all-to-all merge (exchange.cu, NEXT-2).
+size_t route_ws_bytes(int32_t nparts);
+int route_max_parts();
+cudaError_t launch_route(const void* rows, const int64_t* nrows_dev, int64_t max_rows, int32_t row_bytes,
+                         int32_t nparts, void* out, int64_t* part_counts, void* ws, int sms, cudaStream_t s);
 // Sorted-input GROUP BY (sorted.cu).
 size_t sorted_ws_bytes(const Plan& p);
 cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, void* ws, int32_t* status,

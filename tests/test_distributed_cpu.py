@@ -104,3 +104,68 @@ def test_gloo_allgather_merge_equals_oracle():
         s = ((int(sums[i, 1]) & 0xFFFFFFFFFFFFFFFF) << 64) | (int(sums[i, 0]) & 0xFFFFFFFFFFFFFFFF)
         ref[k] = [int(outs[0][i]), s, int(outs[2][i]), int(outs[3][i])]
     assert merged == ref
+
+
+# ---------------------------------------------------------------- all-to-all (hash-routed) exchange, NEXT-2
+def _fmix64(k):
+    k = np.asarray(k, dtype=np.uint64).copy()
+    k ^= k >> np.uint64(33)
+    k *= np.uint64(0xFF51AFD7ED558CCD)
+    k ^= k >> np.uint64(33)
+    k *= np.uint64(0xC4CEB9FE1A85EC53)
+    k ^= k >> np.uint64(33)
+    return k
+
+
+def route_of(keys, P):
+    """Destination rank of a key (the ABI's definition, include/ocelot_b200.h ocl_route_partials)."""
+    return ((_fmix64(keys) & np.uint64(0xFFFFFFFF)) * np.uint64(P)) >> np.uint64(32)
+
+
+def _a2a_worker(rank, world, port, q):
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        from paper_journals_pvldb_heimelspmm13_b200.distributed import exchange_routed, gather_results
+        rng = np.random.default_rng(100 + rank)
+        nrows = 5000 + 1000 * rank
+        rows = np.zeros((nrows, 4), np.int64)                       # 32-byte partial rows: key, count, 2 states
+        rows[:, 0] = rng.integers(0, 1 << 40, nrows)
+        rows[:, 1] = rank + 1
+        rows[:, 2] = np.arange(nrows)
+        dest = route_of(rows[:, 0], world).astype(np.int64)
+        order = np.argsort(dest, kind="stable")                    # grouped by destination (what the kernel does)
+        routed = torch.from_numpy(rows[order].view(np.uint8).reshape(nrows, 32).copy())
+        counts = torch.from_numpy(np.bincount(dest, minlength=world).astype(np.int64))
+        recv, total = exchange_routed(routed, counts)
+        got = recv.numpy().view(np.int64).reshape(total, 4)
+        assert (route_of(got[:, 0], world).astype(np.int64) == rank).all()   # only this rank's partition
+        keys = torch.from_numpy(got[:, 0].copy())
+        allk, allo = gather_results(keys, [torch.from_numpy(got[:, 1:].copy())])
+        if rank == 0:
+            q.put((sorted(map(tuple, np.concatenate([allk.numpy()[:, None], allo[0].numpy()], 1).tolist()))))
+    finally:
+        dist.destroy_process_group()
+
+
+def test_gloo_alltoall_routed_exchange():
+    """Rows routed by key hash reach exactly their owner; the gathered union equals everything sent."""
+    world = 3
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_a2a_worker, args=(r, world, port, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    got = q.get(timeout=300)
+    for p in procs:
+        p.join(timeout=120)
+        assert p.exitcode == 0
+    sent = []
+    for rank in range(world):
+        rng = np.random.default_rng(100 + rank)
+        nrows = 5000 + 1000 * rank
+        k = rng.integers(0, 1 << 40, nrows)
+        sent += [(int(k[i]), rank + 1, i, 0) for i in range(nrows)]
+    assert got == sorted(sent)

@@ -410,3 +410,49 @@ def test_fused_q1_unified_static_shape(monkeypatch):
         lf = _lineitem(n, datagen.BASE_SEED + 2, f64=True)
         p, k, v, a = _q1(lf, f64=True)
         _check_sga(p, k, v, a, tier=1)
+
+
+# ---------------------------------------------------------------- NEXT-2: hash-routed all-to-all merge (fake exchange)
+@pytest.mark.parametrize("P,G", [(2, 5000), (3, 40000), (8, 200000)])
+def test_routed_alltoall_merge(P, G):
+    """Shards -> partial tables -> ocl_route_partials -> destination d gets block d of every shard
+    (stand-in for all_to_all) -> merge per destination: every key at its owner, union == oracle."""
+    from paper_journals_pvldb_heimelspmm13_b200.distributed import shard_range
+    from tests.test_distributed_cpu import route_of
+    rng = np.random.default_rng(G)
+    n = 600000
+    keys = (rng.integers(0, G, n) * 2654435761 % (1 << 40)).astype(np.int64)
+    v = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    f = rng.integers(0, 10**6, n).astype(np.float64) / 100.0
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
+            {"op": "avg", "a": 1}, {"op": "sum", "a": 1}]
+    cap = 2 * G
+    blocks = [[] for _ in range(P)]
+    for r in range(P):
+        s0, ln = shard_range(n, r, P)
+        call = ocl.SgaCall([], [dev(keys[s0:s0 + ln])], [dev(v[s0:s0 + ln]), dev(f[s0:s0 + ln])], aggs,
+                           expected_groups=G, out_capacity=cap)
+        part, cnt = ocl.sga_partial(call, cap)
+        routed, counts = ocl.route_partials(part, cnt, P)
+        c = counts.cpu().numpy()
+        assert c.sum() == int(cnt.item())
+        off = np.concatenate([[0], np.cumsum(c)])
+        for d in range(P):
+            blocks[d].append(routed[off[d]:off[d + 1]])
+    got_k, got_o = [], []
+    for d in range(P):
+        recv = torch.cat(blocks[d]).contiguous()
+        call = ocl.SgaCall([], [dev(keys)], [dev(v), dev(f)], aggs, expected_groups=G, out_capacity=cap)
+        total = recv.shape[0]
+        ocl.merge_partials(call, recv if total else torch.zeros((1, recv.shape[1]), dtype=torch.uint8, device=DEV),
+                           torch.tensor([total], dtype=torch.int64, device=DEV), 1, max(total, 1))
+        k, o = call.result()
+        k = k.cpu().numpy()
+        assert (route_of(k.view(np.uint64), P).astype(np.int64) == d).all()   # partition d only
+        got_k.append(k)
+        got_o.append([x.cpu().numpy() for x in o])
+    gk = np.concatenate(got_k)
+    go = [np.concatenate([g[i] for g in got_o]) for i in range(len(aggs))]
+    rk, routs = oracle.sga([], [keys], [v, f], aggs)
+    dts = [v.dtype, f.dtype]
+    assert_results_equal(by_key(gk, go, aggs, dts), by_key(rk, routs, aggs, dts), aggs, dts)
