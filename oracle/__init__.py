@@ -64,6 +64,8 @@ def lib():
         for f in (L.oracle_group_hash, L.oracle_group_sort, L.oracle_group_sorted):
             f.argtypes = [P, ctypes.c_int, P, ctypes.c_int64, P, P]
             f.restype = ctypes.c_int64
+        L.oracle_hash_join.argtypes = [P, P, P, ctypes.c_int64, P, P, ctypes.c_int64]
+        L.oracle_hash_join.restype = ctypes.c_int64
         L.oracle_aggregate.argtypes = [P, P, ctypes.c_int64, ctypes.c_int64, P, ctypes.c_int, P, ctypes.c_int]
         L.oracle_aggregate.restype = ctypes.c_int
         L.oracle_sga.argtypes = [P, P, ctypes.c_int, P, ctypes.c_int, P, ctypes.c_int, P, ctypes.c_int,
@@ -197,6 +199,24 @@ def group_sort(keys, oids=None, m=None):
 def group_sorted(keys, oids=None, m=None):
     """The paper's sorted-input grouping (successor compare + prefix sum, L554-556); raises on unsorted keys."""
     return _group(lib().oracle_group_sorted, keys, oids, len(keys[0]) if m is None else m)
+
+
+def hash_join(build, probe, oids=None):
+    """All (probe row, build row) pairs with equal keys, probe order, partners ascending -> two uint32 arrays."""
+    b, kb = _col(build)
+    p, kp = _col(probe)
+    m = len(probe)
+    if oids is not None:
+        oids = np.ascontiguousarray(oids, np.uint32)
+        m = len(oids)
+    n = lib().oracle_hash_join(ctypes.byref(b), ctypes.byref(p), None if oids is None else oids.ctypes.data, m,
+                               None, None, 0)
+    if n < 0:
+        raise ValueError("invalid join spec")
+    op, ob = np.zeros(max(n, 1), np.uint32), np.zeros(max(n, 1), np.uint32)
+    lib().oracle_hash_join(ctypes.byref(b), ctypes.byref(p), None if oids is None else oids.ctypes.data, m,
+                           op.ctypes.data, ob.ctypes.data, n)
+    return op[:n], ob[:n]
 
 
 def aggregate(gids, G, vals, aggs, oids=None):

@@ -253,6 +253,32 @@ int64_t oracle_group_sorted(const orc_column* keys, int nkeys, const uint32_t* o
   return prefix;
 }
 
+// Equi-join (§4.1.5): the plain definition — every pair (probe row
+// j, build row i) with key(j) == key(i) — evaluated with a std::unordered_map from key
+// to the ascending list of build rows.  Pairs in probe order, a probe row's partners in
+// ascending build order.  Keys: raw bits masked to the column width (both sides the
+// same dtype).  Returns the number of pairs (written only while < out_capacity), or -1.
+int64_t oracle_hash_join(const orc_column* build, const orc_column* probe, const uint32_t* oids, int64_t m,
+                         uint32_t* out_probe, uint32_t* out_build, int64_t out_capacity) {
+  if (!keys_valid(build, 1) || !keys_valid(probe, 1) || build->dtype != probe->dtype) return -1;
+  std::unordered_map<uint64_t, std::vector<uint32_t>> rows_of;
+  for (int64_t i = 0; i < build->n; ++i) rows_of[packed_key(build, 1, i)].push_back((uint32_t)i);
+  int64_t k = 0;
+  for (int64_t j = 0; j < m; ++j) {
+    const int64_t r = oids ? (int64_t)oids[j] : j;
+    auto it = rows_of.find(packed_key(probe, 1, r));
+    if (it == rows_of.end()) continue;
+    for (uint32_t i : it->second) {
+      if (k < out_capacity) {
+        out_probe[k] = (uint32_t)r;
+        out_build[k] = i;
+      }
+      ++k;
+    }
+  }
+  return k;
+}
+
 int oracle_aggregate(const int32_t* gids, const uint32_t* oids, int64_t m, int64_t G,
                      const orc_column* vals, int nvals, const orc_agg* aggs, int naggs) {
   for (int i = 0; i < naggs; ++i)

@@ -82,6 +82,12 @@ int64_t oracle_group_sort(const orc_column* keys, int nkeys, const uint32_t* oid
  * (unsigned) decreases anywhere (input not sorted). */
 int64_t oracle_group_sorted(const orc_column* keys, int nkeys, const uint32_t* oids, int64_t m,
                             int32_t* gids, int64_t* keys_out);
+/* Equi hash join (L534-550 §4.1.5): all pairs (probe row, build row) with equal keys
+ * (one integer key column per side, same dtype), in probe order, partners ascending.
+ * probe rows j < m at oids[j] (NULL: row j).  Returns the pair count (pairs written while
+ * < out_capacity), -1 on an invalid spec. */
+int64_t oracle_hash_join(const orc_column* build, const orc_column* probe, const uint32_t* oids, int64_t m,
+                         uint32_t* out_probe, uint32_t* out_build, int64_t out_capacity);
 /* a7-a8 (L562-568): per group g in [0,G):
  *   COUNT -> int64;  SUM over int64 (expr values in int128, wrapping mod 2^128)
  *   -> 16 bytes {uint64 lo, int64 hi};  SUM over f64 -> double (Neumaier

@@ -100,6 +100,10 @@ def lib():
             "ocl_sga_partial": [P, P, P, I64, P, P, SZ, P],
             "ocl_merge_partials_workspace_size": [P, P, I32, I64, PSZ],
             "ocl_merge_partials": [P, P, P, I32, I64, P, P, SZ, P],
+            "ocl_join_build_workspace_size": [P, I64, PSZ],
+            "ocl_join_build": [P, P, P, SZ, P, P],
+            "ocl_join_probe_workspace_size": [P, I64, PSZ],
+            "ocl_join_probe": [P, P, P, P, P, P, I64, I32, P, P, I64, P, P, P, SZ, P],
             "ocl_route_partials_workspace_size": [P, I32, PSZ],
             "ocl_route_partials": [P, P, P, I64, I32, I32, P, P, P, SZ, P],
             "ocl_select_group_aggregate_host_workspace_size": [P, P, I64, PSZ],
@@ -130,6 +134,7 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate", "ocl_partial_row_bytes",
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
                "ocl_route_partials_workspace_size", "ocl_route_partials",
+               "ocl_join_build_workspace_size", "ocl_join_build", "ocl_join_probe_workspace_size", "ocl_join_probe",
                "ocl_select_group_aggregate_host_workspace_size", "ocl_select_group_aggregate_host")
 
 
@@ -330,6 +335,59 @@ def group_build_sorted(keys, oids=None, m=None, max_rows=None, out_capacity=None
                                         keys_out.data_ptr(), out_capacity, ng.data_ptr(), status.data_ptr(),
                                         ws.data_ptr(), sz.value, _stream(stream)))
     return gids, keys_out, ng, status
+
+
+# ---------------------------------------------------------------- equi hash join
+class JoinBuild:
+    """Hash table over a build key column (kept on the device for any number of probes)."""
+
+    def __init__(self, build_key, stream=None):
+        self.key = build_key
+        self.ctx = context(build_key.device)
+        self._kc = _col(build_key)
+        sz = ctypes.c_size_t()
+        _check(lib().ocl_join_build_workspace_size(self.ctx.handle, build_key.numel(), ctypes.byref(sz)))
+        self.ws = _workspace(sz.value, build_key.device)
+        self.status = torch.zeros(1, dtype=torch.int32, device=build_key.device)
+        _check(lib().ocl_join_build(self.ctx.handle, ctypes.byref(self._kc), self.ws.data_ptr(), sz.value,
+                                    self.status.data_ptr(), _stream(stream)))
+
+    def probe(self, probe_key, oids=None, m=None, max_rows=None, pk_build=False, out_capacity=None, stream=None):
+        """-> (out_probe int32[cap] (uint32 oids), out_build int32[cap], npairs int64[1], status int32[1])."""
+        dev = probe_key.device
+        max_rows = (oids.numel() if oids is not None else probe_key.numel()) if max_rows is None else max_rows
+        out_capacity = max(max_rows, 1) if out_capacity is None else out_capacity
+        sz = ctypes.c_size_t()
+        _check(lib().ocl_join_probe_workspace_size(self.ctx.handle, max_rows, ctypes.byref(sz)))
+        ws = _workspace(sz.value, dev)
+        op = torch.empty(max(out_capacity, 1), dtype=torch.int32, device=dev)
+        ob = torch.empty(max(out_capacity, 1), dtype=torch.int32, device=dev)
+        nout = torch.zeros(1, dtype=torch.int64, device=dev)
+        status = torch.zeros(1, dtype=torch.int32, device=dev)
+        pc = _col(probe_key)
+        _check(lib().ocl_join_probe(self.ctx.handle, ctypes.byref(self._kc), self.ws.data_ptr(), ctypes.byref(pc),
+                                    None if oids is None else oids.data_ptr(), None if m is None else m.data_ptr(),
+                                    max_rows, int(bool(pk_build)), op.data_ptr(), ob.data_ptr(), out_capacity,
+                                    nout.data_ptr(), status.data_ptr(), ws.data_ptr(), sz.value, _stream(stream)))
+        return op, ob, nout, status
+
+
+def hash_join(build_key, probe_key, oids=None, pk_build=False, out_capacity=None):
+    """Blocking equi-join: (probe oids, build oids) of all matching pairs, grouped by probe row.
+    Grows the output and re-probes once if out_capacity was too small."""
+    jb = JoinBuild(build_key)
+    for _ in range(2):
+        op, ob, nout, st = jb.probe(probe_key, oids=oids, pk_build=pk_build, out_capacity=out_capacity)
+        torch.cuda.current_stream(probe_key.device).synchronize()
+        s = int(st.item()) or int(jb.status.item())
+        n = int(nout.item())
+        if s == OCL_ERR_CAPACITY and n > (out_capacity or 0) and int(jb.status.item()) == 0:
+            out_capacity = n
+            continue
+        if s != OCL_OK:
+            raise OcelotError(s, f"join device status ({n} pairs)")
+        return op[:n], ob[:n]
+    raise OcelotError(OCL_ERR_CAPACITY, "join output")
 
 
 # ---------------------------------------------------------------- a7-a8

@@ -649,6 +649,70 @@ ocl_status ocl_group_build_sorted(ocl_ctx* ctx, const ocl_column* keys, int32_t 
   return OCL_OK;
 }
 
+// ---------------------------------------------------------------- equi hash join
+static ocl_status join_key(const ocl_column* c, const char* what, DevKey* k) {
+  ocl_status s = check_column(c, what);
+  if (s) return s;
+  if (c->dtype == OCL_F64) return fail(OCL_ERR_INVALID_ARG, "%s: f64 join key", what);
+  const int w = 8 * dtype_width(c->dtype);
+  k->col = devcol(*c);
+  k->shift = 0;
+  k->mask = w == 64 ? ~0ULL : ((1ULL << w) - 1);
+  return OCL_OK;
+}
+
+ocl_status ocl_join_build_workspace_size(ocl_ctx* ctx, int64_t n_build, size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (n_build < 0 || n_build >= kMaxRows) return fail(OCL_ERR_INVALID_ARG, "n_build out of range");
+  *bytes = join_build_ws_bytes(n_build);
+  return OCL_OK;
+}
+
+ocl_status ocl_join_build(ocl_ctx* ctx, const ocl_column* build_key, void* build_ws, size_t build_ws_bytes,
+                          int32_t* dev_status, void* stream) {
+  if (!ctx) return fail(OCL_ERR_INVALID_ARG, "NULL ctx");
+  DevKey k;
+  ocl_status s = join_key(build_key, "build_key", &k);
+  if (s) return s;
+  if (!build_ws || build_ws_bytes < join_build_ws_bytes(build_key->n))
+    return fail(OCL_ERR_CAPACITY, "build workspace %zu B < required %zu B", build_ws_bytes, join_build_ws_bytes(build_key->n));
+  cudaStream_t st = (cudaStream_t)stream;
+  if (dev_status) OCL_CUDA(cudaMemsetAsync(dev_status, 0, 4, st), "status init");
+  OCL_CUDA(launch_join_build(k, build_key->n, build_ws, dev_status, ctx->sms, st), "join build");
+  return OCL_OK;
+}
+
+ocl_status ocl_join_probe_workspace_size(ocl_ctx* ctx, int64_t max_rows, size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (max_rows < 0 || max_rows >= kMaxRows) return fail(OCL_ERR_INVALID_ARG, "max_rows out of range");
+  *bytes = join_probe_ws_bytes(max_rows);
+  return OCL_OK;
+}
+
+ocl_status ocl_join_probe(ocl_ctx* ctx, const ocl_column* build_key, const void* build_ws,
+                          const ocl_column* probe_key, const uint32_t* probe_oids, const int64_t* m_dev,
+                          int64_t max_rows, int32_t pk_build, uint32_t* out_probe, uint32_t* out_build,
+                          int64_t out_capacity, int64_t* nout_dev, int32_t* dev_status, void* ws, size_t ws_bytes,
+                          void* stream) {
+  if (!ctx || !nout_dev) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/nout_dev");
+  DevKey bk, pk;
+  ocl_status s = join_key(build_key, "build_key", &bk);
+  if (s) return s;
+  if ((s = join_key(probe_key, "probe_key", &pk))) return s;
+  if (build_key->dtype != probe_key->dtype) return fail(OCL_ERR_INVALID_ARG, "build/probe key dtypes differ");
+  if (max_rows < 0 || max_rows >= kMaxRows) return fail(OCL_ERR_INVALID_ARG, "max_rows out of range");
+  if (!probe_oids && probe_key->n < max_rows) return fail(OCL_ERR_INVALID_ARG, "probe column shorter than max_rows");
+  if (out_capacity < 0 || (out_capacity > 0 && (!out_probe || !out_build))) return fail(OCL_ERR_INVALID_ARG, "bad outputs");
+  if (!build_ws) return fail(OCL_ERR_INVALID_ARG, "NULL build_ws");
+  if (max_rows > 0 && (!ws || ws_bytes < join_probe_ws_bytes(max_rows)))
+    return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, join_probe_ws_bytes(max_rows));
+  cudaStream_t st = (cudaStream_t)stream;
+  if (dev_status) OCL_CUDA(cudaMemsetAsync(dev_status, 0, 4, st), "status init");
+  OCL_CUDA(launch_join_probe(build_ws, build_key->n, pk, probe_oids, m_dev, max_rows, pk_build != 0, out_probe,
+                             out_build, out_capacity, nout_dev, dev_status, ws, ctx->sms, st), "join probe");
+  return OCL_OK;
+}
+
 // ---------------------------------------------------------------- a7-a8
 ocl_status ocl_group_aggregate_workspace_size(ocl_ctx* ctx, int64_t max_groups, const ocl_column* vals, int32_t nvals,
                                               const ocl_agg* aggs, int32_t naggs, size_t* bytes) {

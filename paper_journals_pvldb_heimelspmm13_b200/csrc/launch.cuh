@@ -70,6 +70,14 @@ size_t route_ws_bytes(int32_t nparts);
 int route_max_parts();
 cudaError_t launch_route(const void* rows, const int64_t* nrows_dev, int64_t max_rows, int32_t row_bytes,
                          int32_t nparts, void* out, int64_t* part_counts, void* ws, int sms, cudaStream_t s);
+// Equi hash join (join.cu).
+size_t join_build_ws_bytes(int64_t n_build);
+size_t join_probe_ws_bytes(int64_t max_rows);
+cudaError_t launch_join_build(const DevKey& bk, int64_t n_build, void* ws, int32_t* status, int sms, cudaStream_t s);
+cudaError_t launch_join_probe(const void* build_ws, int64_t n_build, const DevKey& pk, const uint32_t* oids,
+                              const int64_t* m_dev, int64_t max_rows, bool pk_build, uint32_t* out_probe,
+                              uint32_t* out_build, int64_t out_capacity, int64_t* nout, int32_t* status, void* ws,
+                              int sms, cudaStream_t s);
 // Sorted-input GROUP BY (sorted.cu).
 size_t sorted_ws_bytes(const Plan& p);
 cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, void* ws, int32_t* status,

@@ -372,3 +372,33 @@ def test_group_sorted_degenerate_and_unsorted():
     # unsigned packed order: -1 (all ones) sorts after every non-negative key
     gids, kout = oracle.group_sorted([np.array([0, 5, -1, -1], np.int64)])
     assert gids.tolist() == [0, 1, 2, 2]
+
+
+# ---------------------------------------------------------------- equi hash join
+def _py_nested_join(build, probe):
+    """Brute-force nested loop (the paper's theta-join shape with '=')."""
+    return [(j, i) for j in range(len(probe)) for i in range(len(build)) if build[i] == probe[j]]
+
+
+@pytest.mark.parametrize("dtype", [np.uint8, np.int32, np.int64])
+def test_hash_join_nested_loop(dtype):
+    rng = np.random.default_rng(3)
+    build = rng.integers(0, 40, 150).astype(dtype)
+    probe = rng.integers(0, 60, 200).astype(dtype)
+    op, ob = oracle.hash_join(build, probe)
+    assert list(zip(op.tolist(), ob.tolist())) == _py_nested_join(build.tolist(), probe.tolist())
+
+
+def test_hash_join_pk_fk_and_oids():
+    rng = np.random.default_rng(4)
+    pk = rng.permutation(1000).astype(np.int64) * 7 - 3000               # unique build keys, some negative
+    fk = rng.choice(pk, 5000)
+    fk[::10] = 10**9                                                      # dangling foreign keys
+    oids = np.flatnonzero(rng.random(5000) < 0.5).astype(np.uint32)
+    op, ob = oracle.hash_join(pk, fk, oids)
+    pos = {int(k): i for i, k in enumerate(pk.tolist())}
+    ref = [(int(j), pos[int(fk[j])]) for j in oids.tolist() if int(fk[j]) in pos]
+    assert list(zip(op.tolist(), ob.tolist())) == ref                    # <= 1 partner per probe row (PK)
+    assert len(ref) == sum(1 for j in oids.tolist() if fk[j] != 10**9)
+    with pytest.raises(ValueError):
+        oracle.hash_join(pk, fk.astype(np.int32))                         # dtypes differ
