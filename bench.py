@@ -55,6 +55,10 @@ WORKLOADS = {
                      "grouping of sorted input (P:L554-556)",
                 rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000,
                 sorted=True),
+    "j3": dict(desc="J3 (NEXT-3): PK-FK equi hash join orders.o_orderkey (15,000,000 unique keys, build) x "
+                    "lineitem.l_orderkey (60,000,000 rows, probe, dbgen order); direct one-pass PK probe; "
+                    "pairs (probe oid, build oid) out",
+               rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="join", f64=False, groups=15_000_000),
     "c5": dict(desc="C5 sweep point: 2^28 rows, p i32 ~ U[0,1e6), key = hash(Zipf(s) rank over G), v i64; "
                     "WHERE p < T GROUP BY key: COUNT, SUM, MIN, MAX(v)",
                rows=1 << 28, seed=datagen.BASE_SEED + 5, kind="sweep", f64=False, groups=1 << 10),
@@ -216,6 +220,69 @@ def run_reference(args, wl, rank):
     print(json.dumps(line), flush=True)
 
 
+def bench_join(args, wl, dev):
+    """J3: build + probe per step, device-resident inputs; value = probe rows / step time."""
+    import paper_journals_pvldb_heimelspmm13_b200 as ocl
+    n = wl["rows"]
+    nb = (n + 27) // 28 * 7                          # every order a lineitem block can reference
+    probe = datagen.lineitem_device(n, wl["seed"], fields=("orderkey",), device=dev)["orderkey"]
+    build_h = datagen.orders_keys(nb)
+    build = torch.from_numpy(build_h).to(dev)
+    torch.cuda.synchronize()
+    state = {}
+
+    def step():
+        jb = ocl.JoinBuild(build)
+        state["r"] = jb.probe(probe, pk_build=True, out_capacity=n)
+        state["jb"] = jb
+
+    clk = ClockSampler(dev.index).start()
+    for _ in range(args.warmup):
+        step()
+    torch.cuda.synchronize()
+    op, ob, nout, st = state["r"]
+    assert int(st.item()) == 0 and int(state["jb"].status.item()) == 0, "join device status"
+    npairs = int(nout.item())
+    K = args.steps
+    t0, t1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    torch.cuda.synchronize()
+    l0 = ocl.launch_count()
+    h0 = time.perf_counter()
+    t0.record()
+    for _ in range(K):
+        step()
+    t1.record()
+    torch.cuda.synchronize()
+    h1 = time.perf_counter()
+    clk.window(h0, h1)
+    clk.stop()
+    ms = t0.elapsed_time(t1) / K
+    peak, peak_src = measured_peak_gbs()
+    algo = 8 * nb + 16 * nb + 8 * n + 8 * npairs      # build keys, table entries, probe keys, pairs out
+    cpu = None
+    if not args.no_cpu:
+        import oracle
+        sample = min(n, 20_000_000)
+        ph = datagen.lineitem_host(sample, wl["seed"], fields=("orderkey",), n_total=n)["orderkey"]
+        tc = time.perf_counter()
+        oracle.hash_join(build_h, ph)
+        dt = time.perf_counter() - tc
+        cpu = {"value": sample / dt, "unit": "rows/s", "cores": 1, "kind": "oracle",
+               "sample": f"build all {nb:,} orders keys + probe the first {sample:,} lineitem rows, "
+                         f"oracle.hash_join (C++17 unordered_map, single thread), {dt:.1f} s"}
+    line = {"metric": METRIC, "value": n / (ms / 1e3), "unit": "rows/s", "n_gpus": 1, "steps": K,
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "strong",
+            "vs_baseline": None, "dtype": "int64", "data": "synthetic (datagen lineitem / orders keys)",
+            "config": {"workload": wl["desc"], "rows": n, "build_rows": nb, "pairs": npairs,
+                       "l2": "inputs 0.6 GB > 2x L2, no flush needed"},
+            "roofline": {"bound": "hbm", "achieved": algo / (ms / 1e3) / 1e9, "peak": peak, "unit": "GB/s",
+                         "frac": algo / (ms / 1e3) / 1e9 / peak, "traffic": None,
+                         "kernel": "ocl::k_join_insert/alloc/fill + k_join_probe_pk (whole step)",
+                         "algorithmic_bytes_per_launch": algo, "peak_source": peak_src},
+            "cpu_baseline": cpu, "e2e": None, "gpu_launches": ocl.launch_count() - l0, "clocks": clk.summary()}
+    print(json.dumps(line), flush=True)
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
@@ -249,6 +316,10 @@ def main():
         return
     torch.cuda.set_device(local)
     dev = torch.device("cuda", local)
+    if wl["kind"] == "join":
+        if world == 1:
+            bench_join(args, wl, dev)
+        return
     if world > 1:
         import torch.distributed as dist
         dist.init_process_group("nccl", device_id=dev)

@@ -153,3 +153,14 @@ def sweep_device(n, seed, G, s=0.0, row0=0, f64=False, device=None):
     if f64:
         out["v_f"] = v_f
     return out
+
+
+def orders_keys(n_orders, seed=None, shuffled=True):
+    """o_orderkey of the orders table behind a lineitem of 4 * n_orders rows: the sparse keys
+    (o/8)*32 + o%8 + 1 of ocl_datagen.h (8 of every 32 used, dbgen-like), optionally in a seeded
+    random row order.  int64 numpy array."""
+    o = np.arange(n_orders, dtype=np.int64)
+    k = (o // 8) * 32 + o % 8 + 1
+    if shuffled:
+        k = np.random.default_rng(BASE_SEED if seed is None else seed).permutation(k)
+    return k
