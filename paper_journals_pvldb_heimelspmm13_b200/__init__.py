@@ -100,6 +100,8 @@ def lib():
             "ocl_sga_partial": [P, P, P, I64, P, P, SZ, P],
             "ocl_merge_partials_workspace_size": [P, P, I32, I64, PSZ],
             "ocl_merge_partials": [P, P, P, I32, I64, P, P, SZ, P],
+            "ocl_radix_sort_workspace_size": [P, I64, I32, I32, PSZ],
+            "ocl_radix_sort": [P, P, I32, P, P, P, P, P, SZ, P],
             "ocl_join_build_workspace_size": [P, I64, PSZ],
             "ocl_join_build": [P, P, P, SZ, P, P],
             "ocl_join_probe_workspace_size": [P, I64, PSZ],
@@ -135,6 +137,7 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
                "ocl_route_partials_workspace_size", "ocl_route_partials",
                "ocl_join_build_workspace_size", "ocl_join_build", "ocl_join_probe_workspace_size", "ocl_join_probe",
+               "ocl_radix_sort_workspace_size", "ocl_radix_sort",
                "ocl_select_group_aggregate_host_workspace_size", "ocl_select_group_aggregate_host")
 
 
@@ -335,6 +338,28 @@ def group_build_sorted(keys, oids=None, m=None, max_rows=None, out_capacity=None
                                         keys_out.data_ptr(), out_capacity, ng.data_ptr(), status.data_ptr(),
                                         ws.data_ptr(), sz.value, _stream(stream)))
     return gids, keys_out, ng, status
+
+
+# ---------------------------------------------------------------- radix sort
+def radix_sort(keys, payload=None, rowids=False, stream=None):
+    """Stable sort by the packed key (1-2 integer columns, unsigned order) -> (packed keys int64[n],
+    payload permuted or None, source row ids int32[n] (uint32) or None)."""
+    dev = keys[0].device
+    ctx = context(dev)
+    n = keys[0].numel()
+    sz = ctypes.c_size_t()
+    _check(lib().ocl_radix_sort_workspace_size(ctx.handle, n, int(payload is not None), int(bool(rowids)),
+                                               ctypes.byref(sz)))
+    ws = _workspace(sz.value, dev)
+    ko = torch.empty(max(n, 1), dtype=torch.int64, device=dev)
+    po = torch.empty(max(n, 1), dtype=payload.dtype, device=dev) if payload is not None else None
+    ro = torch.empty(max(n, 1), dtype=torch.int32, device=dev) if rowids else None
+    kc = _cols(keys)
+    pc = _col(payload) if payload is not None else None
+    _check(lib().ocl_radix_sort(ctx.handle, kc, len(keys), ctypes.byref(pc) if pc is not None else None,
+                                ko.data_ptr(), po.data_ptr() if po is not None else None,
+                                ro.data_ptr() if ro is not None else None, ws.data_ptr(), sz.value, _stream(stream)))
+    return ko[:n], (po[:n] if po is not None else None), (ro[:n] if ro is not None else None)
 
 
 # ---------------------------------------------------------------- equi hash join (P:L534-550)

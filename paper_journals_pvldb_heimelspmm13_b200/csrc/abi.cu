@@ -118,6 +118,7 @@ struct Planned {
   size_t table_bytes;
   int32_t pbits;     // >= 0: hash-partitioned high-cardinality tier with 2^pbits partitions (partition.cu)
   bool sorted;       // sort-based grouping of sorted input (sorted.cu)
+  bool sortgrp;      // tier 6: radix sort, then the sorted path (radix.cu + sorted.cu)
 };
 
 ocl_status plan_values(const ocl_column* vals, int32_t nvals, const ocl_agg* aggs, int32_t naggs, Planned* P) {
@@ -387,6 +388,15 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   const bool many = a->tier == 0 && p.smem_cap == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
   if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
   P->sorted = a->key_sorted != 0;
+  P->sortgrp = a->tier == 6;
+  if (P->sortgrp) {
+    if (a->key_sorted) return fail(OCL_ERR_INVALID_ARG, "tier 6 sorts the input itself: key_sorted must be 0");
+    if (a->npreds != 0 || a->nkeys == 0) return fail(OCL_ERR_UNSUPPORTED, "tier 6: no predicate, >= 1 key column");
+    if (p.ncols > 1 || (p.ncols == 1 && p.vcols[0].width != 8))
+      return fail(OCL_ERR_UNSUPPORTED, "tier 6: at most one distinct 8-byte value column");
+    P->pbits = -1;
+    P->table_bytes = 0;
+  }
   if (P->sorted) {
     if (a->tier != 0) return fail(OCL_ERR_INVALID_ARG, "key_sorted needs tier 0");
     if (a->nkeys == 0) return fail(OCL_ERR_INVALID_ARG, "key_sorted needs a key column");
@@ -399,14 +409,37 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   f.ngroups_out = a->ngroups_out;
   f.out_capacity = a->out_capacity;
   f.status = a->dev_status;
-  if (a->order_by_key && !P->sorted && !sorted_emit_supported(P->cap))
+  if (a->order_by_key && !P->sorted && !P->sortgrp && !sorted_emit_supported(P->cap))
     return fail(OCL_ERR_UNSUPPORTED, "order_by_key needs expected_groups <= 2047 (table of %llu slots)", (unsigned long long)P->cap);
   return OCL_OK;
 }
 
 
 // table + finalize workspace of a fused call
+// tier 6 plan over the sorted copies: one packed i64 key column, the value column re-pointed
+Plan sortgrp_plan(const Plan& p0, const uint64_t* skeys, const uint64_t* svals) {
+  Plan q = p0;
+  q.nkeys = 1;
+  q.keys[0].col = DevCol{skeys, OCL_I64, 8};
+  q.keys[0].shift = 0;
+  q.keys[0].mask = ~0ULL;
+  const void* v0 = p0.ncols ? p0.vcols[0].ptr : nullptr;
+  auto remap = [&](DevCol& c) { if (v0 && c.ptr == v0) c.ptr = svals; };
+  for (int i = 0; i < q.ncols; ++i) remap(q.vcols[i]);
+  for (int v = 0; v < q.nvals; ++v) {
+    remap(q.vals[v].a);
+    remap(q.vals[v].b);
+    remap(q.vals[v].c);
+  }
+  q.vec_ok = 1;
+  return q;
+}
+
 size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) {
+  if (P.sortgrp) {
+    const int64_t n = P.plan.n;
+    return align_up((size_t)n * 8, 256) * 2 + radix_ws_bytes(n, P.plan.ncols > 0, false) + sorted_ws_bytes(P.plan);
+  }
   if (P.sorted) return sorted_ws_bytes(P.plan);
   return P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256) +
          (P.pbits >= 0 ? part_ws_bytes(P.plan, P.pbits, ctx->sms) : 0);
@@ -777,6 +810,30 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
   ocl_status s = plan_sga(args, &P);
   if (s) return s;
   cudaStream_t st = (cudaStream_t)stream;
+  if (P.sortgrp) {                // tier 6: radix sort then the sorted path
+    size_t need = sga_ws_bytes(ctx, P);
+    if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+    if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, sizeof(int32_t), st), "status init");
+    const int64_t n = P.plan.n;
+    uint8_t* w = (uint8_t*)ws;
+    uint64_t* skeys = (uint64_t*)w;
+    uint64_t* svals = (uint64_t*)(w + align_up((size_t)n * 8, 256));
+    void* rws = w + 2 * align_up((size_t)n * 8, 256);
+    void* sws = (uint8_t*)rws + radix_ws_bytes(n, P.plan.ncols > 0, false);
+    if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, st), "profile event");
+    if (n == 0) {
+      OCL_CUDA(cudaMemsetAsync(args->ngroups_out, 0, 8, st), "group count");
+    } else {
+      OCL_CUDA(launch_radix(P.plan, P.plan.ncols ? (const uint64_t*)P.plan.vcols[0].ptr : nullptr, skeys,
+                            P.plan.ncols ? svals : nullptr, nullptr, rws, ctx->sms, st), "radix sort");
+      int kind = 0;
+      OCL_CUDA(launch_sorted(sortgrp_plan(P.plan, skeys, svals), P.fin, P.values_f64, sws, args->dev_status,
+                             args->ngroups_out, args->out_capacity, ctx->sms, st, &kind), "sorted group-by");
+      ctx->last_kernel = 50 + (kind - 40);
+    }
+    if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, st), "profile event");
+    return OCL_OK;
+  }
   if (P.sorted) {                 // sort-based grouping: no table, outputs written by the kernels
     size_t need = sga_ws_bytes(ctx, P);
     if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
@@ -817,7 +874,7 @@ ocl_status ocl_sga_partial(ocl_ctx* ctx, const ocl_sga_args* args, void* partial
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
-  if (P.sorted) return fail(OCL_ERR_UNSUPPORTED, "key_sorted partial tables (multi-GPU) are not implemented");
+  if (P.sorted || P.sortgrp) return fail(OCL_ERR_UNSUPPORTED, "sort-based partial tables (multi-GPU) are not implemented");
   cudaStream_t st = (cudaStream_t)stream;
   void* ews = nullptr;
   if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
@@ -876,6 +933,41 @@ ocl_status ocl_merge_partials(ocl_ctx* ctx, const ocl_sga_args* args, const void
   ea.fin = P.fin;
   OCL_CUDA(launch_emit((uint8_t*)ws, cap, P.plan.stride, ea, args->ngroups_out, args->out_capacity, args->dev_status,
                        args->order_by_key != 0, (uint8_t*)ws + tbytes, ctx->grid, st), "merge finalize");
+  return OCL_OK;
+}
+
+ocl_status ocl_radix_sort_workspace_size(ocl_ctx* ctx, int64_t n, int32_t with_payload, int32_t with_rowids,
+                                         size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (n < 0 || n >= kMaxRows) return fail(OCL_ERR_INVALID_ARG, "n out of range");
+  *bytes = radix_ws_bytes(n, with_payload != 0, with_rowids != 0);
+  return OCL_OK;
+}
+
+ocl_status ocl_radix_sort(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, const ocl_column* payload,
+                          uint64_t* keys_out, void* payload_out, uint32_t* rowids_out, void* ws, size_t ws_bytes,
+                          void* stream) {
+  if (!ctx) return fail(OCL_ERR_INVALID_ARG, "NULL ctx");
+  if (nkeys < 1) return fail(OCL_ERR_INVALID_ARG, "nkeys=%d (1..2)", nkeys);
+  Plan p;
+  memset(&p, 0, sizeof(p));
+  ocl_status s = plan_keys(keys, nkeys, p);
+  if (s) return s;
+  const int64_t n = keys[0].n;
+  for (int i = 1; i < nkeys; ++i)
+    if (keys[i].n != n) return fail(OCL_ERR_INVALID_ARG, "key columns differ in length");
+  if (payload) {
+    if ((s = check_column(payload, "payload"))) return s;
+    if (dtype_width(payload->dtype) != 8 || payload->n != n) return fail(OCL_ERR_INVALID_ARG, "payload: 8-byte column of n rows");
+    if (n > 0 && !payload_out) return fail(OCL_ERR_INVALID_ARG, "NULL payload_out");
+  }
+  if (n > 0 && !keys_out) return fail(OCL_ERR_INVALID_ARG, "NULL keys_out");
+  const size_t need = radix_ws_bytes(n, payload != nullptr, rowids_out != nullptr);
+  if (n > 0 && (!ws || ws_bytes < need)) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  p.n = n;
+  OCL_CUDA(launch_radix(p, payload ? (const uint64_t*)payload->data : nullptr, keys_out,
+                        payload ? (uint64_t*)payload_out : nullptr, rowids_out, ws, ctx->sms, (cudaStream_t)stream),
+           "radix sort");
   return OCL_OK;
 }
 
@@ -952,7 +1044,7 @@ ocl_status ocl_select_group_aggregate_host_workspace_size(ocl_ctx* ctx, const oc
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
-  if (P.sorted) return fail(OCL_ERR_UNSUPPORTED, "key_sorted is not available on the host-buffer path");
+  if (P.sorted || P.sortgrp) return fail(OCL_ERR_UNSUPPORTED, "sort-based grouping is not available on the host-buffer path");
   P.pbits = -1;             // chunks stream through the one-pass fused kernel
   HostCols h;
   collect_host_cols(P, h, chunk_rows);

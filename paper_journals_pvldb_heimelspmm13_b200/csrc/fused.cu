@@ -389,6 +389,9 @@ const char* fused_kernel_name(int kind) {
     case 40: return "k_sorted_summary/scan/agg<DynShape> (sorted input)";
     case 41: return "k_sorted_summary/scan/agg<StaticShape key i64> (sorted input)";
     case 42: return "k_sorted_summary/scan/agg<StaticShape pred i32, key i64> (sorted input)";
+    case 50: return "k_rs_* radix sort + k_sorted_*<DynShape> (tier 6)";
+    case 51: return "k_rs_* radix sort + k_sorted_*<StaticShape key i64> (tier 6)";
+    case 52: return "k_rs_* radix sort + k_sorted_*<StaticShape pred i32, key i64> (tier 6)";
     default: return "k_sga<DynShape>";
   }
 }
