@@ -90,6 +90,8 @@ def lib():
             "ocl_gather": [P, P, P, P, I64, P, P],
             "ocl_group_build_workspace_size": [P, I64, I64, PSZ],
             "ocl_group_build": [P, P, I32, P, P, I64, I64, P, P, I64, P, P, P, SZ, P],
+            "ocl_group_build_paper_workspace_size": [P, I64, I64, PSZ],
+            "ocl_group_build_paper": [P, P, I32, P, P, I64, I64, P, P, I64, P, P, P, SZ, P],
             "ocl_group_build_sorted_workspace_size": [P, I64, PSZ],
             "ocl_group_build_sorted": [P, P, I32, P, P, I64, P, P, I64, P, P, P, SZ, P],
             "ocl_group_aggregate_workspace_size": [P, I64, P, I32, P, I32, PSZ],
@@ -132,6 +134,7 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_select_bitmap", "ocl_bitmap_combine", "ocl_prefix_compact_workspace_size", "ocl_prefix_compact",
                "ocl_gather", "ocl_group_build_workspace_size", "ocl_group_build",
                "ocl_group_build_sorted_workspace_size", "ocl_group_build_sorted",
+               "ocl_group_build_paper_workspace_size", "ocl_group_build_paper",
                "ocl_group_aggregate_workspace_size", "ocl_group_aggregate",
                "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate", "ocl_partial_row_bytes",
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
@@ -297,21 +300,25 @@ def gather(col, oids, m=None, max_m=None, stream=None):
 
 
 # ---------------------------------------------------------------- a4-a6
-def group_build(keys, oids=None, m=None, max_rows=None, expected_groups=1024, out_capacity=None, stream=None):
-    """Hash group-by -> (gids int32[max_rows], keys_out int64[cap], ngroups int64[1], status int32[1])."""
+def group_build(keys, oids=None, m=None, max_rows=None, expected_groups=1024, out_capacity=None, stream=None,
+                scheme="b200"):
+    """Hash group-by -> (gids int32[max_rows], keys_out int64[cap], ngroups int64[1], status int32[1]).
+    scheme "paper": the paper's optimistic / verify / pessimistic hashing, for the ablation."""
     dev = keys[0].device
     ctx = context(dev)
     max_rows = (oids.numel() if oids is not None else keys[0].numel()) if max_rows is None else max_rows
     out_capacity = max_rows if out_capacity is None else out_capacity
     sz = ctypes.c_size_t()
-    _check(lib().ocl_group_build_workspace_size(ctx.handle, max_rows, expected_groups, ctypes.byref(sz)))
+    ws_fn = lib().ocl_group_build_paper_workspace_size if scheme == "paper" else lib().ocl_group_build_workspace_size
+    build_fn = lib().ocl_group_build_paper if scheme == "paper" else lib().ocl_group_build
+    _check(ws_fn(ctx.handle, max_rows, expected_groups, ctypes.byref(sz)))
     ws = _workspace(sz.value, dev)
     gids = torch.empty(max(max_rows, 1), dtype=torch.int32, device=dev)
     keys_out = torch.empty(max(out_capacity, 1), dtype=torch.int64, device=dev)
     ng = torch.zeros(1, dtype=torch.int64, device=dev)
     status = torch.zeros(1, dtype=torch.int32, device=dev)
     kc = _cols(keys)
-    _check(lib().ocl_group_build(ctx.handle, kc, len(keys), None if oids is None else oids.data_ptr(),
+    _check(build_fn(ctx.handle, kc, len(keys), None if oids is None else oids.data_ptr(),
                                  None if m is None else m.data_ptr(), max_rows, expected_groups, gids.data_ptr(),
                                  keys_out.data_ptr(), out_capacity, ng.data_ptr(), status.data_ptr(), ws.data_ptr(),
                                  sz.value, _stream(stream)))

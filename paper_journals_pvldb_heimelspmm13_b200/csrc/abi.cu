@@ -646,6 +646,40 @@ ocl_status ocl_group_build(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, 
   return OCL_OK;
 }
 
+ocl_status ocl_group_build_paper_workspace_size(ocl_ctx* ctx, int64_t max_rows, int64_t expected_groups,
+                                                size_t* bytes) {
+  if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
+  if (max_rows < 0 || max_rows >= kMaxRows) return fail(OCL_ERR_INVALID_ARG, "max_rows out of range");
+  if (expected_groups > ((int64_t)1 << 31)) return fail(OCL_ERR_UNSUPPORTED, "expected_groups > 2^31");
+  *bytes = hp_ws_bytes(max_rows, expected_groups);
+  return OCL_OK;
+}
+
+ocl_status ocl_group_build_paper(ocl_ctx* ctx, const ocl_column* keys, int32_t nkeys, const uint32_t* oids,
+                                 const int64_t* m_dev, int64_t max_rows, int64_t expected_groups, int32_t* gid_out,
+                                 int64_t* keys_out, int64_t out_capacity, int64_t* ngroups_out, int32_t* dev_status,
+                                 void* ws, size_t ws_bytes, void* stream) {
+  if (!ctx || !ngroups_out) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/ngroups_out");
+  if (nkeys < 1) return fail(OCL_ERR_INVALID_ARG, "nkeys=%d (1..2)", nkeys);
+  size_t need = 0;
+  ocl_status s = ocl_group_build_paper_workspace_size(ctx, max_rows, expected_groups, &need);
+  if (s) return s;
+  if (max_rows > 0 && !gid_out) return fail(OCL_ERR_INVALID_ARG, "NULL gid_out");
+  Plan p;
+  memset(&p, 0, sizeof(p));
+  if ((s = plan_keys(keys, nkeys, p))) return s;
+  if (!ws || ws_bytes < need) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  cudaStream_t st = (cudaStream_t)stream;
+  p.status = dev_status;
+  p.oids = oids;
+  p.m_dev = m_dev;
+  p.n = max_rows;
+  if (dev_status) OCL_CUDA(cudaMemsetAsync(dev_status, 0, 4, st), "status init");
+  OCL_CUDA(launch_group_build_paper(p, expected_groups, gid_out, keys_out, keys_out ? out_capacity : INT64_MAX,
+                                    ngroups_out, ws, ctx->sms, st), "paper group build");
+  return OCL_OK;
+}
+
 ocl_status ocl_group_build_sorted_workspace_size(ocl_ctx* ctx, int64_t max_rows, size_t* bytes) {
   if (!ctx || !bytes) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/bytes");
   if (max_rows < 0 || max_rows > ((int64_t)1 << 31)) return fail(OCL_ERR_UNSUPPORTED, "max_rows outside [0, 2^31]");

@@ -78,6 +78,10 @@ cudaError_t launch_join_probe(const void* build_ws, int64_t n_build, const DevKe
                               const int64_t* m_dev, int64_t max_rows, bool pk_build, uint32_t* out_probe,
                               uint32_t* out_build, int64_t out_capacity, int64_t* nout, int32_t* status, void* ws,
                               int sms, cudaStream_t s);
+// The paper's hashing scheme for the ablation (hashpaper.cu).
+size_t hp_ws_bytes(int64_t max_rows, int64_t expected);
+cudaError_t launch_group_build_paper(const Plan& p, int64_t expected, int32_t* gid_out, int64_t* keys_out,
+                                     int64_t out_capacity, int64_t* ngroups, void* ws, int sms, cudaStream_t s);
 // LSD radix sort of packed keys (radix.cu).
 size_t radix_ws_bytes(int64_t n, bool val, bool row);
 cudaError_t launch_radix(const Plan& p, const uint64_t* vcol, uint64_t* kout, uint64_t* vout, uint32_t* rout,

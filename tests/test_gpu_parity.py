@@ -102,7 +102,8 @@ def test_gather():
 # ---------------------------------------------------------------- a4-a6
 @pytest.mark.parametrize("kind,G", [("u8u8", 6), ("i64", 1000), ("i64", 200000), ("i32", 50), ("u8", 256),
                                     ("i32i32", 500), ("u8i32", 300), ("i64neg1", 10)])
-def test_group_build(kind, G):
+@pytest.mark.parametrize("scheme", ["b200", "paper"])
+def test_group_build(kind, G, scheme):
     rng = np.random.default_rng(G)
     n = 300000
     if kind == "u8u8":
@@ -122,7 +123,7 @@ def test_group_build(kind, G):
     oids = np.flatnonzero(rng.random(n) < 0.7).astype(np.uint32)
     ref_g, ref_k = oracle.group_hash(keys, oids)
     gids, kout, ng, st = ocl.group_build([dev(k) for k in keys], oids=dev(oids.view(np.int32)),
-                                         expected_groups=max(len(ref_k), 16))
+                                         expected_groups=max(len(ref_k), 16), scheme=scheme)
     torch.cuda.synchronize()
     assert int(st.item()) == 0
     Gg = int(ng.item())
@@ -139,10 +140,11 @@ def test_group_build(kind, G):
         assert kk[gg] == ref_k[ref_g[j]]
 
 
-def test_group_build_capacity_status():
+@pytest.mark.parametrize("scheme", ["b200", "paper"])
+def test_group_build_capacity_status(scheme):
     n = 5000
     keys = [np.arange(n, dtype=np.int64)]
-    gids, kout, ng, st = ocl.group_build([dev(keys[0])], expected_groups=8)
+    gids, kout, ng, st = ocl.group_build([dev(keys[0])], expected_groups=8, scheme=scheme)
     torch.cuda.synchronize()
     assert int(st.item()) == ocl.OCL_ERR_CAPACITY                            # restart signal
 
