@@ -392,6 +392,7 @@ def main():
         ms, kms = tt.tolist()
     value = n / (ms / 1e3)
     peak, peak_src = measured_peak_gbs()
+    out_bytes = G * (8 + sum(o.element_size() * (o[0].numel() if o.dim() > 1 else 1) for o in outs))
     algo_bytes = bpr * length
     achieved = algo_bytes / (kms / 1e3) / 1e9
 
@@ -466,7 +467,10 @@ def main():
                        "grouping": "sort-based (sorted input)" if key_sorted else "hash"},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                          "traffic": profiled_traffic(args.workload, length), "kernel": "ocl::" + kernel_name,
-                         "kernel_ms": kms, "algorithmic_bytes_per_launch": algo_bytes, "peak_source": peak_src},
+                         "kernel_ms": kms, "algorithmic_bytes_per_launch": algo_bytes, "peak_source": peak_src,
+                         # high-G paths also report the bytes including the G output rows
+                         "achieved_with_output": (algo_bytes + out_bytes) / (kms / 1e3) / 1e9,
+                         "output_bytes_per_launch": out_bytes},
             "hbm_frac_step": algo_bytes / (ms / 1e3) / 1e9 / peak,
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clk.summary(),
         }
