@@ -50,6 +50,11 @@ WORKLOADS = {
                     "COUNT/SUM/MIN/MAX(l_quantity), shuffled row order (seeded Feistel permutation)",
                rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000,
                shuffled=True),
+    "c3s": dict(desc="C3 shuffled via sort-based grouping (tier 6): lineitem SF10, 60,000,000 rows in a seeded "
+                     "random order; radix sort of (l_orderkey, l_quantity) (P:L456-467) then the sorted-input "
+                     "GROUP BY (P:L554-556); COUNT/SUM/MIN/MAX(l_quantity), 15M groups",
+                rows=60_000_000, seed=datagen.BASE_SEED + 3, kind="orderkey", f64=False, groups=15_000_000,
+                shuffled=True, tier=6),
     "c3c": dict(desc="C3 clustered: lineitem SF10, 60,000,000 rows; GROUP BY l_orderkey (15M groups), "
                      "COUNT/SUM/MIN/MAX(l_quantity), dbgen (clustered, sorted orderkey) row order; sort-based "
                      "grouping of sorted input (P:L554-556)",
@@ -334,8 +339,9 @@ def main():
     order = wl["kind"] == "q1"
     eg = wl["groups"] if world == 1 else wl["groups"]
     key_sorted = bool(wl.get("sorted"))
+    tier = args.tier or wl.get("tier", 0)
     call = ocl.SgaCall(p, k, v, aggs, expected_groups=eg, out_capacity=max(16, 2 * eg), order_by_key=order,
-                       tier=args.tier, key_sorted=key_sorted)
+                       tier=tier, key_sorted=key_sorted)
     ctx = call.ctx
     # inputs smaller than 2x the 126 MB L2 are flushed before every step (a 512 MB write)
     flush = torch.empty(512 << 20, dtype=torch.uint8, device=dev) if bpr * length < (256 << 20) else None
@@ -464,7 +470,8 @@ def main():
                        "l2": f"inputs {bpr * length / 1e9:.2f} GB per GPU > 2x the 126 MB L2, no flush needed"
                              if flush is None else "inputs < 2x L2: L2 flushed (512 MB write) before every step, "
                                                    "per-step CUDA events exclude the flush",
-                       "grouping": "sort-based (sorted input)" if key_sorted else "hash"},
+                       "grouping": "sort-based (sorted input)" if key_sorted else
+                                   ("radix sort + sorted input (tier 6)" if tier == 6 else "hash")},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,
                          "traffic": profiled_traffic(args.workload, length), "kernel": "ocl::" + kernel_name,
                          "kernel_ms": kms, "algorithmic_bytes_per_launch": algo_bytes, "peak_source": peak_src,
