@@ -302,6 +302,7 @@ def main():
     ap.add_argument("--no-cpu", action="store_true")
     ap.add_argument("--tier", type=int, default=0)
     ap.add_argument("--no-sorted", action="store_true", help="c3c: hash grouping instead of the sorted-input path")
+    ap.add_argument("--graph", action="store_true", help="replay the fused call as one CUDA graph (1 GPU)")
     ap.add_argument("--c5-groups", type=int, default=1 << 10, help="C5: key cardinality G")
     ap.add_argument("--c5-zipf", type=float, default=0.0, help="C5: Zipf exponent s (0 = uniform)")
     ap.add_argument("--c5-sel", type=float, default=1.0, help="C5: selectivity (0.01, 0.5, 1.0)")
@@ -346,8 +347,17 @@ def main():
     # inputs smaller than 2x the 126 MB L2 are flushed before every step (a 512 MB write)
     flush = torch.empty(512 << 20, dtype=torch.uint8, device=dev) if bpr * length < (256 << 20) else None
 
+    graph = None
+    if args.graph and world == 1:
+        l0 = ocl.launch_count()
+        call.launch()                                    # kernels per call (a replay launches the same ones)
+        per_call = ocl.launch_count() - l0
+        graph = call.capture()
+
     def step():
-        if world == 1:
+        if graph is not None:
+            graph.replay()
+        elif world == 1:
             call.launch()
         else:
             distributed_select_group_aggregate(call)
@@ -373,7 +383,8 @@ def main():
     h0 = time.perf_counter()
     t0.record()
     for i in range(K):
-        ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
+        if graph is None:
+            ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
         if flush is not None:
             flush.zero_()
         sev[i][0].record()
@@ -391,7 +402,10 @@ def main():
         dist.barrier()
     # per-step device time: the whole region / K, or (L2 flushed between steps) the mean of per-step events
     ms = t0.elapsed_time(t1) / K if flush is None else statistics.mean(a.elapsed_time(b) for a, b in sev)
-    kms = statistics.mean(a.elapsed_time(b) for a, b in kev)
+    # graph replay: the library's kernel events are not in the graph -> the step events bracket the kernels
+    kms = statistics.mean(a.elapsed_time(b) for a, b in (kev if graph is None else sev))
+    if graph is not None:
+        launches = per_call * K
     if world > 1:
         tt = torch.tensor([ms, kms], dtype=torch.float64, device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
@@ -470,6 +484,7 @@ def main():
                        "l2": f"inputs {bpr * length / 1e9:.2f} GB per GPU > 2x the 126 MB L2, no flush needed"
                              if flush is None else "inputs < 2x L2: L2 flushed (512 MB write) before every step, "
                                                    "per-step CUDA events exclude the flush",
+                       "launch": "one CUDA graph replay per step" if graph is not None else "stream launches",
                        "grouping": "sort-based (sorted input)" if key_sorted else
                                    ("radix sort + sorted input (tier 6)" if tier == 6 else "hash")},
             "roofline": {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s", "frac": achieved / peak,

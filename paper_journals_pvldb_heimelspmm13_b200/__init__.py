@@ -504,6 +504,22 @@ class SgaCall:
             _check(lib().ocl_select_group_aggregate(self.ctx.handle, ctypes.byref(self.args), self.ws.data_ptr(),
                                                     self.ws_bytes, _stream(stream)))
 
+    def capture(self, stream=None):
+        """Record launch() once into a CUDA graph (torch.cuda.CUDAGraph) and return it: replay() re-runs the
+        whole fused call (table init, kernels, finalisation) with one launch — for small, launch-bound inputs.
+        The graph reuses this call's arguments, workspace and outputs."""
+        if self.host:
+            raise ValueError("the host-buffer path synchronises inside; it cannot be captured")
+        s = stream or torch.cuda.Stream(self.device)
+        s.wait_stream(torch.cuda.current_stream(self.device))
+        with torch.cuda.stream(s):
+            self.launch(s)                                   # warm-up outside the capture (lazy attributes)
+        torch.cuda.current_stream(self.device).wait_stream(s)
+        g = torch.cuda.CUDAGraph()
+        with torch.cuda.graph(g, stream=s):
+            self.launch(s)
+        return g
+
     def result(self):
         """Synchronise, check the device status, return (keys[G], [outs[G]]) (host path: CPU tensors)."""
         if not self.host:

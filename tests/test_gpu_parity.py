@@ -458,3 +458,31 @@ def test_routed_alltoall_merge(P, G):
     rk, routs = oracle.sga([], [keys], [v, f], aggs)
     dts = [v.dtype, f.dtype]
     assert_results_equal(by_key(gk, go, aggs, dts), by_key(rk, routs, aggs, dts), aggs, dts)
+
+
+def test_cuda_graph_replay():
+    """SgaCall.capture(): the whole fused call (table init, kernel, finalisation) replayed as one CUDA graph
+    gives the oracle's result, repeatedly (C1 shape, and the sorted path)."""
+    li = _lineitem(60000, datagen.BASE_SEED + 1)
+    p, k, v, a = _q1(li)
+    call = ocl.SgaCall([(dev(c), s) for c, s in p], [dev(c) for c in k], [dev(c) for c in v], a,
+                       expected_groups=4, order_by_key=True)
+    g = call.capture()
+    rk, routs = oracle.sga(p, k, v, a, order_by_key=True)
+    dts = [c.dtype for c in v]
+    for _ in range(3):
+        call.outs[0].zero_()
+        g.replay()
+        keys, outs = call.result()
+        assert keys.cpu().numpy().tolist() == rk.tolist()
+        assert_results_equal(by_key(keys.cpu().numpy(), [o.cpu().numpy() for o in outs], a, dts),
+                             by_key(rk, routs, a, dts), a, dts)
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    call = ocl.SgaCall([], [dev(li["orderkey"])], [dev(li["quantity"])], aggs, expected_groups=20000,
+                       out_capacity=20000, key_sorted=True)
+    g = call.capture()
+    g.replay()
+    keys, outs = call.result()
+    rk, routs = oracle.sga([], [li["orderkey"]], [li["quantity"]], aggs, order_by_key=True)
+    assert np.array_equal(keys.cpu().numpy(), rk)
+    assert all(np.array_equal(o.cpu().numpy(), r) for o, r in zip(outs, routs))
