@@ -469,6 +469,41 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   return OCL_OK;
 }
 
+// Sort-based grouping (key_sorted = 1: the sorted path; tier 6: radix sort, then the sorted
+// path).  partial_out != NULL: partial rows for the multi-GPU merge instead of final outputs,
+// count -> *count_out (capacity cap).
+ocl_status run_sortpath(ocl_ctx* ctx, const ocl_sga_args* args, const Planned& P, void* ws, size_t ws_bytes,
+                        cudaStream_t st, uint8_t* partial_out, int64_t cap, int64_t* count_out) {
+  size_t need = sga_ws_bytes(ctx, P);
+  if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, sizeof(int32_t), st), "status init");
+  if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, st), "profile event");
+  int kind = 0;
+  if (P.sortgrp) {                // tier 6: radix sort (P:L456-467) then the sorted path (P:L554-556)
+    const int64_t n = P.plan.n;
+    uint8_t* w = (uint8_t*)ws;
+    uint64_t* skeys = (uint64_t*)w;
+    uint64_t* svals = (uint64_t*)(w + align_up((size_t)n * 8, 256));
+    void* rws = w + 2 * align_up((size_t)n * 8, 256);
+    void* sws = (uint8_t*)rws + radix_ws_bytes(n, P.plan.ncols > 0, false);
+    if (n == 0) {
+      OCL_CUDA(cudaMemsetAsync(count_out, 0, 8, st), "group count");
+    } else {
+      OCL_CUDA(launch_radix(P.plan, P.plan.ncols ? (const uint64_t*)P.plan.vcols[0].ptr : nullptr, skeys,
+                            P.plan.ncols ? svals : nullptr, nullptr, rws, ctx->sms, st), "radix sort");
+      OCL_CUDA(launch_sorted(sortgrp_plan(P.plan, skeys, svals), P.fin, P.values_f64, sws, args->dev_status,
+                             count_out, cap, ctx->sms, st, &kind, partial_out), "sorted group-by");
+      ctx->last_kernel = 50 + (kind - 40);
+    }
+  } else {                        // sorted input: no table, outputs written by the kernels
+    OCL_CUDA(launch_sorted(P.plan, P.fin, P.values_f64, ws, args->dev_status, count_out, cap, ctx->sms, st, &kind,
+                           partial_out), "sorted group-by launch");
+    ctx->last_kernel = kind;
+  }
+  if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, st), "profile event");
+  return OCL_OK;
+}
+
 }  // namespace
 
 // ======================================================================== ABI
@@ -844,42 +879,8 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
   ocl_status s = plan_sga(args, &P);
   if (s) return s;
   cudaStream_t st = (cudaStream_t)stream;
-  if (P.sortgrp) {                // tier 6: radix sort (P:L456-467) then the sorted path (P:L554-556)
-    size_t need = sga_ws_bytes(ctx, P);
-    if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
-    if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, sizeof(int32_t), st), "status init");
-    const int64_t n = P.plan.n;
-    uint8_t* w = (uint8_t*)ws;
-    uint64_t* skeys = (uint64_t*)w;
-    uint64_t* svals = (uint64_t*)(w + align_up((size_t)n * 8, 256));
-    void* rws = w + 2 * align_up((size_t)n * 8, 256);
-    void* sws = (uint8_t*)rws + radix_ws_bytes(n, P.plan.ncols > 0, false);
-    if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, st), "profile event");
-    if (n == 0) {
-      OCL_CUDA(cudaMemsetAsync(args->ngroups_out, 0, 8, st), "group count");
-    } else {
-      OCL_CUDA(launch_radix(P.plan, P.plan.ncols ? (const uint64_t*)P.plan.vcols[0].ptr : nullptr, skeys,
-                            P.plan.ncols ? svals : nullptr, nullptr, rws, ctx->sms, st), "radix sort");
-      int kind = 0;
-      OCL_CUDA(launch_sorted(sortgrp_plan(P.plan, skeys, svals), P.fin, P.values_f64, sws, args->dev_status,
-                             args->ngroups_out, args->out_capacity, ctx->sms, st, &kind), "sorted group-by");
-      ctx->last_kernel = 50 + (kind - 40);
-    }
-    if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, st), "profile event");
-    return OCL_OK;
-  }
-  if (P.sorted) {                 // sort-based grouping: no table, outputs written by the kernels
-    size_t need = sga_ws_bytes(ctx, P);
-    if (ws_bytes < need || !ws) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
-    if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, sizeof(int32_t), st), "status init");
-    if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, st), "profile event");
-    int kind = 0;
-    OCL_CUDA(launch_sorted(P.plan, P.fin, P.values_f64, ws, args->dev_status, args->ngroups_out, args->out_capacity,
-                           ctx->sms, st, &kind), "sorted group-by launch");
-    ctx->last_kernel = kind;
-    if (ctx->prof_end) OCL_CUDA(cudaEventRecord(ctx->prof_end, st), "profile event");
-    return OCL_OK;
-  }
+  if (P.sorted || P.sortgrp) return run_sortpath(ctx, args, P, ws, ws_bytes, st, nullptr, args->out_capacity,
+                                                 args->ngroups_out);
   void* ews = nullptr;
   if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
   EmitArgs ea;
@@ -908,8 +909,9 @@ ocl_status ocl_sga_partial(ocl_ctx* ctx, const ocl_sga_args* args, void* partial
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
-  if (P.sorted || P.sortgrp) return fail(OCL_ERR_UNSUPPORTED, "sort-based partial tables (multi-GPU) are not implemented");
   cudaStream_t st = (cudaStream_t)stream;
+  if (P.sorted || P.sortgrp)
+    return run_sortpath(ctx, args, P, ws, ws_bytes, st, (uint8_t*)partial_out, partial_capacity, npartial_out);
   void* ews = nullptr;
   if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
   EmitArgs ea;

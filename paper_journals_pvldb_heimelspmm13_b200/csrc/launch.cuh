@@ -89,7 +89,8 @@ cudaError_t launch_radix(const Plan& p, const uint64_t* vcol, uint64_t* kout, ui
 // Sorted-input GROUP BY (sorted.cu).
 size_t sorted_ws_bytes(const Plan& p);
 cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, void* ws, int32_t* status,
-                          int64_t* ngroups_out, int64_t out_capacity, int sms, cudaStream_t s, int* kind);
+                          int64_t* ngroups_out, int64_t out_capacity, int sms, cudaStream_t s, int* kind,
+                          uint8_t* partial_out = nullptr);
 size_t group_build_sorted_ws_bytes(int64_t max_rows);
 cudaError_t launch_group_build_sorted(const Plan& p, int32_t* gid_out, int64_t* keys_out, int64_t out_capacity,
                                       int64_t* ngroups, void* ws, int sms, cudaStream_t s);

@@ -110,6 +110,7 @@ struct SortedArgs {
   int32_t* status;
   FinPlan fin;
   FastEmit fe;
+  uint8_t* partial_out;     // non-null: write partial rows (multi-GPU export) instead of final outputs
 };
 
 __device__ __forceinline__ uint32_t lane_lt() {
@@ -433,6 +434,28 @@ __device__ __forceinline__ void seg_emit(const Plan& p, const FinPlan& f, const 
   }
 }
 
+// Partial row g (ocl_sga_partial layout = the table entry layout with the real key first).
+template <class Sh, int NV>
+__device__ __forceinline__ void seg_partial(const Plan& p, uint8_t* out, int64_t cap, const Seg<NV>& a, uint64_t key,
+                                            int64_t g) {
+  if (g >= cap) return;
+  uint64_t* row = (uint64_t*)(out + g * (int64_t)p.stride);
+  for (int w = 2; w < p.stride / 8; ++w) row[w] = 0;
+  row[0] = key;
+  row[1] = a.cnt;
+#pragma unroll
+  for (int v = 0; v < NV; ++v) {
+    if (v >= Sh::nv(p)) break;
+    const DevValue& d = p.vals[v];
+    if (Sh::fsum(p, v)) {
+      *(uint64_t*)((uint8_t*)row + d.off_sum) = a.s[v].lo;
+      if (!Sh::vf64(p, v)) *(uint64_t*)((uint8_t*)row + d.off_sum + 8) = a.s[v].hi;
+    }
+    if (Sh::fmn(p, v)) *(uint64_t*)((uint8_t*)row + d.off_min) = a.mn[v];
+    if (Sh::fmx(p, v)) *(uint64_t*)((uint8_t*)row + d.off_max) = a.mx[v];
+  }
+}
+
 // A run piece that may continue across a unit boundary: merge into the chain table
 // entry of its group id (find-or-insert by gid, then atomics).
 template <class Sh, int NV>
@@ -540,7 +563,8 @@ struct GenOps {
     Seg<NV> s;
     uint64_t key;
     get(p, st, slot, s, key);
-    seg_emit<Sh, NV>(p, a.fin, s, key, g);
+    if (a.partial_out) seg_partial<Sh, NV>(p, a.partial_out, a.out_capacity, s, key, g);
+    else seg_emit<Sh, NV>(p, a.fin, s, key, g);
   }
 };
 
@@ -649,7 +673,8 @@ struct FastOps {
       Seg<NV> s;
       uint64_t key;
       get(p, st, slot, s, key);
-      seg_emit<Sh, NV>(p, a.fin, s, key, g);
+      if (a.partial_out) seg_partial<Sh, NV>(p, a.partial_out, a.out_capacity, s, key, g);
+      else seg_emit<Sh, NV>(p, a.fin, s, key, g);
       return;
     }
     if (g >= a.fin.out_capacity) return;
@@ -856,11 +881,19 @@ __global__ void __launch_bounds__(kSortedThreads) k_sorted_agg(const __grid_cons
 }
 
 __global__ void k_sorted_chain_emit(const uint8_t* chains, int32_t stride, const uint64_t* chain_key, uint64_t cap,
-                                    const __grid_constant__ FinPlan f) {
+                                    const __grid_constant__ FinPlan f, uint8_t* partial_out, int64_t out_capacity) {
   for (uint64_t i = blockIdx.x * (uint64_t)blockDim.x + threadIdx.x; i < cap; i += (uint64_t)gridDim.x * blockDim.x) {
     const uint8_t* e = chains + i * (uint64_t)stride;
     const uint64_t sk = *(const uint64_t*)e;
-    if (sk) emit_final(f, e, chain_key[i], (int64_t)~sk);
+    if (!sk) continue;
+    const int64_t g = (int64_t)~sk;
+    if (!partial_out) {
+      emit_final(f, e, chain_key[i], g);
+    } else if (g < out_capacity) {                            // partial row: the entry with the real key first
+      uint64_t* row = (uint64_t*)(partial_out + g * (int64_t)stride);
+      row[0] = chain_key[i];
+      for (int w = 1; w < stride / 8; ++w) row[w] = ((const uint64_t*)e)[w];
+    }
   }
 }
 
@@ -1038,7 +1071,8 @@ static cudaError_t sorted_run(const Plan& p, const SortedArgs& a, int sms, cudaS
   fn<<<grid, kSortedThreads, smem, s>>>(p, a);
   const uint64_t cap = a.chain_mask + 1;
   const int cgrid = (int)std::min<uint64_t>((cap + 255) / 256, (uint64_t)sms * 4);
-  k_sorted_chain_emit<<<cgrid, 256, 0, s>>>(a.chains, p.stride, a.chain_key, cap, a.fin);
+  k_sorted_chain_emit<<<cgrid, 256, 0, s>>>(a.chains, p.stride, a.chain_key, cap, a.fin, a.partial_out,
+                                            a.out_capacity);
   return cudaGetLastError();
 }
 
@@ -1051,7 +1085,8 @@ static cudaError_t sorted_dyn(const Plan& p, const SortedArgs& a, int sms, cudaS
 }
 
 cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, void* ws, int32_t* status,
-                          int64_t* ngroups_out, int64_t out_capacity, int sms, cudaStream_t s, int* kind) {
+                          int64_t* ngroups_out, int64_t out_capacity, int sms, cudaStream_t s, int* kind,
+                          uint8_t* partial_out) {
   *kind = 40;
   if (p.n == 0) return cudaMemsetAsync(ngroups_out, 0, 8, s);
   SortedArgs a;
@@ -1075,6 +1110,8 @@ cudaError_t launch_sorted(const Plan& p, const FinPlan& fin, bool values_f64, vo
   a.status = status;
   a.fin = fin;
   a.fe = build_fast_emit(p, fin);
+  a.partial_out = partial_out;
+  if (partial_out) a.fe.ok = 0;                               // partial rows: the generic row writer
   if (p.vec_ok && shape_match<ShK64>(p)) {
     *kind = 41;
     const char* ek = getenv("OCL_SORTED_K");               // tuning knob: rows per lane per step

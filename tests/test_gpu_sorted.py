@@ -172,3 +172,31 @@ def test_fused_sorted_edge_cases():
         ocl.select_group_aggregate([], [dev(bad)], [dev(v)], C3_AGGS, key_sorted=True)
     # output capacity too small -> the binding's restart grows it
     _check_sorted([], [keys], [v], C3_AGGS, out_capacity=10)
+
+
+@pytest.mark.parametrize("mode", ["sorted", "tier6"])
+def test_sorted_partials_merge(mode):
+    """Multi-GPU pieces for the sort-based paths: row shards (runs cut at shard boundaries) -> partial
+    rows (ocl_sga_partial) -> merge == oracle over all rows (fake exchange on one GPU)."""
+    from paper_journals_pvldb_heimelspmm13_b200.distributed import shard_range
+    n, P = 300001, 3
+    li = datagen.lineitem_host(n, datagen.BASE_SEED + 3, shuffled=(mode == "tier6"))
+    aggs = C3_AGGS + [{"op": "avg", "a": 0}]
+    kw = dict(key_sorted=True) if mode == "sorted" else dict(tier=6)
+    cap = n // 2
+    parts, counts = [], []
+    for r in range(P):
+        s0, ln = shard_range(n, r, P)
+        call = ocl.SgaCall([], [dev(li["orderkey"][s0:s0 + ln])], [dev(li["quantity"][s0:s0 + ln])], aggs,
+                           expected_groups=cap, out_capacity=cap, **kw)
+        part, cnt = ocl.sga_partial(call, cap)
+        parts.append(part)
+        counts.append(cnt)
+    allp = torch.stack(parts).contiguous()
+    call = ocl.SgaCall([], [dev(li["orderkey"])], [dev(li["quantity"])], aggs, expected_groups=cap, out_capacity=cap)
+    ocl.merge_partials(call, allp, torch.cat(counts), P, cap)
+    keys, outs = call.result()
+    rk, routs = oracle.sga([], [li["orderkey"]], [li["quantity"]], aggs)
+    dts = [np.int64]
+    assert_results_equal(by_key(keys.cpu().numpy(), [o.cpu().numpy() for o in outs], aggs, dts),
+                         by_key(rk, routs, aggs, dts), aggs, dts)
