@@ -446,8 +446,12 @@ size_t sga_ws_bytes(ocl_ctx* ctx, const Planned& P) {
 }
 
 // Run the fused pass into a zeroed table carved from ws; returns the emit workspace.
+// ea / count_out / cap: the emission the caller wants; the hash-partitioned tier performs it
+// itself (*emitted = true), otherwise the caller emits from the table.
 ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, size_t ws_bytes, cudaStream_t s,
-                     void** emit_ws) {
+                     void** emit_ws, const EmitArgs* ea = nullptr, int64_t* count_out = nullptr, int64_t cap = 0,
+                     bool* emitted = nullptr) {
+  if (emitted) *emitted = false;
   size_t need = sga_ws_bytes(ctx, P);
   if (ws_bytes < need || (!ws && need)) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
   P.plan.table = (uint8_t*)ws;
@@ -459,7 +463,8 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
     int kind = 0;
     if (P.pbits >= 0) {
       void* pws = (uint8_t*)ws + P.table_bytes + align_up(emit_ws_bytes(ctx->grid), 256);
-      OCL_CUDA(launch_partitioned(P.plan, P.pbits, pws, ctx->sms, s, &kind), "partitioned aggregation launch");
+      OCL_CUDA(launch_partitioned(P.plan, P.pbits, pws, ctx->sms, s, &kind, ea, count_out, cap, emitted),
+               "partitioned aggregation launch");
     } else {
       OCL_CUDA(launch_fused(P.plan, fused_mode(a), P.values_f64, ctx->sms, s, &kind), "fused kernel launch");
     }
@@ -882,13 +887,17 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
   if (P.sorted || P.sortgrp) return run_sortpath(ctx, args, P, ws, ws_bytes, st, nullptr, args->out_capacity,
                                                  args->ngroups_out);
   void* ews = nullptr;
-  if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
   EmitArgs ea;
   memset(&ea, 0, sizeof(ea));
   ea.kind = EMIT_FINAL;
   ea.fin = P.fin;
-  OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, args->ngroups_out, args->out_capacity, args->dev_status,
-                       args->order_by_key != 0, ews, ctx->grid, st), "finalize");
+  bool emitted = false;
+  if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews, args->order_by_key ? nullptr : &ea, args->ngroups_out,
+                     args->out_capacity, &emitted)))
+    return s;
+  if (!emitted)
+    OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, args->ngroups_out, args->out_capacity,
+                         args->dev_status, args->order_by_key != 0, ews, ctx->grid, st), "finalize");
   return OCL_OK;
 }
 
@@ -913,15 +922,17 @@ ocl_status ocl_sga_partial(ocl_ctx* ctx, const ocl_sga_args* args, void* partial
   if (P.sorted || P.sortgrp)
     return run_sortpath(ctx, args, P, ws, ws_bytes, st, (uint8_t*)partial_out, partial_capacity, npartial_out);
   void* ews = nullptr;
-  if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews))) return s;
   EmitArgs ea;
   memset(&ea, 0, sizeof(ea));
   ea.kind = EMIT_PARTIAL;
   ea.out_capacity = partial_capacity;
   ea.partial_out = (uint8_t*)partial_out;
   ea.status = args->dev_status;
-  OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, npartial_out, partial_capacity, args->dev_status, false,
-                       ews, ctx->grid, st), "partial export");
+  bool emitted = false;
+  if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews, &ea, npartial_out, partial_capacity, &emitted))) return s;
+  if (!emitted)
+    OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, npartial_out, partial_capacity, args->dev_status,
+                         false, ews, ctx->grid, st), "partial export");
   return OCL_OK;
 }
 

@@ -64,7 +64,11 @@ bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err,
 bool part_eligible(const Plan& p);
 int part_bits_for(int64_t expected_groups);
 size_t part_ws_bytes(const Plan& p, int pbits, int sms);
-cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind);
+// ea != NULL: emit the output rows (final or partial) directly, count -> *count_out, *emitted = true
+// (else the caller emits from the HBM table).
+cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind,
+                               const EmitArgs* ea = nullptr, int64_t* count_out = nullptr, int64_t out_capacity = 0,
+                               bool* emitted = nullptr);
 // Hash routing of partial rows for the all-to-all merge (exchange.cu, NEXT-2).
 size_t route_ws_bytes(int32_t nparts);
 int route_max_parts();

@@ -28,6 +28,8 @@
 // partition's keys occupy one contiguous slot range: pass-2 merges stay L2-local.
 // Rows the fast path cannot take (values outside int32, the key ~0) and records
 // whose partition overflows the shared table update the HBM table directly (exact).
+#include <string.h>
+
 #include "launch.cuh"
 #include "sga_device.cuh"
 
@@ -65,7 +67,52 @@ struct PartArgs {
   uint32_t* slowflag;   // [P] 1: the exact path inserted keys of this partition in pass 1
   int32_t direct_ok;    // the HBM table's partition regions have exactly kPartCap slots
   int32_t rec_bytes;
+  // direct emission (direct_emit = 1): partitions aggregated entirely in shared memory write
+  // their output rows (final or partial) straight from there; the others mark dirty[q] and
+  // are emitted from their HBM slot range afterwards — no pass over the whole table.
+  int32_t direct_emit;
+  int32_t npo;                     // final outputs, resolved on the host (kind, CTA-entry fields, pointer)
+  struct { int32_t kind, f0, f1, pad; void* out; } po[kMaxAggs];
+  uint32_t* dirty;                 // [P]
+  unsigned long long* out_ctr;     // output rows so far
+  int64_t* count_out;              // G (or the partial row count)
 };
+
+// One output row (final or partial) from a table-format entry e (key = the real key).
+__device__ __forceinline__ void part_emit_row(const EmitArgs& ea, int32_t stride, const uint8_t* e, uint64_t key,
+                                              int64_t g) {
+  if (ea.kind == EMIT_FINAL) {
+    emit_final(ea.fin, e, key, g);
+  } else if (g < ea.out_capacity) {
+    uint64_t* dst = (uint64_t*)(ea.partial_out + g * (int64_t)stride);
+    dst[0] = key;
+    for (int w = 1; w < stride / 8; ++w) dst[w] = ((const uint64_t*)e)[w];
+  }
+}
+
+// CTA: claim output positions for the `cnt` rows this thread emits (block scan + one atomic).
+__device__ __forceinline__ int64_t part_emit_claim(uint32_t cnt, unsigned long long* ctr, uint32_t* wsum,
+                                                   unsigned long long* base_s) {
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  uint32_t incl = cnt;
+#pragma unroll
+  for (int d = 1; d < 32; d <<= 1) {
+    const uint32_t y = __shfl_up_sync(0xffffffffu, incl, d);
+    if (lane >= d) incl += y;
+  }
+  if (lane == 31) wsum[warp] = incl;
+  __syncthreads();
+  uint32_t off = 0, tot = 0;
+  for (int w = 0; w < (int)(blockDim.x >> 5); ++w) {
+    off += w < warp ? wsum[w] : 0u;
+    tot += wsum[w];
+  }
+  if (threadIdx.x == 0) *base_s = tot ? atomicAdd(ctr, (unsigned long long)tot) : 0ULL;
+  __syncthreads();
+  const int64_t g = (int64_t)(*base_s + off + incl - cnt);
+  __syncthreads();
+  return g;
+}
 
 __device__ __forceinline__ uint32_t part_of(uint64_t key, int pbits) {
   return pbits ? (uint32_t)(fmix64(key) >> (64 - pbits)) : 0u;
@@ -603,11 +650,48 @@ __device__ __forceinline__ void cta_store_entry(const Plan& p, const uint8_t* ce
   }
 }
 
+// One output row from a CTA-table entry (32-bit fields: count, 16-bit split sums, enc32
+// MIN / MAX): final values or a partial row in the table-entry layout.
+__device__ __forceinline__ void cta_emit_row(const Plan& p, const PartArgs& a, const EmitArgs& ea, const uint8_t* ce,
+                                             int64_t g) {
+  const uint64_t key = ~*(const uint64_t*)ce;
+  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+  if (ea.kind != EMIT_FINAL) {
+    if (g >= ea.out_capacity) return;
+    uint8_t* row = ea.partial_out + g * (int64_t)p.stride;
+    cta_store_entry(p, ce, row);
+    *(uint64_t*)row = key;
+    return;
+  }
+  const FinPlan& f = ea.fin;
+  if (g >= f.out_capacity) return;
+  if (f.keys_out) f.keys_out[g] = (int64_t)key;
+  for (int i = 0; i < a.npo; ++i) {
+    const int kind = a.po[i].kind, f0 = a.po[i].f0, f1 = a.po[i].f1;
+    void* out = a.po[i].out;
+    if (kind == 0) {
+      ((int64_t*)out)[g] = cnt;
+    } else if (kind <= 2) {
+      const int64_t sum = (int64_t)(*(const int32_t*)(ce + f1)) * 65536 + (int64_t)(*(const uint32_t*)(ce + f0));
+      if (kind == 1) ((ulonglong2*)out)[g] = make_ulonglong2((uint64_t)sum, (uint64_t)(sum >> 63));
+      else ((double*)out)[g] = __ddiv_rn(__ll2double_rn(sum), __ull2double_rn(cnt));
+    } else if (kind == 3) {
+      ((int64_t*)out)[g] = (int32_t)(~*(const uint32_t*)(ce + f0) ^ 0x80000000u);
+    } else {
+      ((int64_t*)out)[g] = (int32_t)(*(const uint32_t*)(ce + f0) ^ 0x80000000u);
+    }
+  }
+}
+
 template <int NV>
-__global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant__ Plan p, PartArgs a) {
+__global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
+                                                           const __grid_constant__ EmitArgs ea) {
   using Sh = DynShape;
   extern __shared__ __align__(16) uint8_t tab[];
   __shared__ int overflowed;
+  __shared__ uint32_t wsum[kPartThreads / 32];
+  __shared__ unsigned long long base_s;
+  __shared__ uint16_t slot_list[kPartCap];
   const int lane = threadIdx.x & 31;
   const int64_t m = *a.m_dev;
   const int64_t nitems = *a.nitems_dev;
@@ -670,7 +754,30 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
       }
     }
     __syncthreads();
-    if (direct && !overflowed) {
+    if (direct && !overflowed && a.direct_emit) {               // the rows straight from shared memory
+      constexpr int PER = kPartCap / kPartThreads;
+      uint32_t occ = 0;
+#pragma unroll
+      for (int k = 0; k < PER; ++k) {
+        const uint8_t* ce = tab + (size_t)(threadIdx.x + k * kPartThreads) * cs;
+        if (*(const uint64_t*)ce != 0 && *(const uint32_t*)(ce + 8) != 0) occ |= 1u << k;
+      }
+      // occupied slots listed in shared memory, then emitted by consecutive threads into
+      // consecutive output rows (coalesced stores)
+      const int64_t g0 = part_emit_claim(__popc(occ), a.out_ctr, wsum, &base_s);
+      const uint32_t off = (uint32_t)(g0 - (int64_t)base_s);
+      uint32_t at = off;
+#pragma unroll
+      for (int k = 0; k < PER; ++k)
+        if ((occ >> k) & 1u) slot_list[at++] = (uint16_t)(threadIdx.x + k * kPartThreads);
+      uint32_t tot = 0;
+      for (int w = 0; w < kPartThreads / 32; ++w) tot += wsum[w];
+      __syncthreads();
+      for (uint32_t i = threadIdx.x; i < tot; i += kPartThreads) {
+        const uint8_t* ce = tab + (size_t)slot_list[i] * cs;
+        cta_emit_row(p, a, ea, ce, (int64_t)base_s + i);
+      }
+    } else if (direct && !overflowed) {
       uint8_t* region = p.table + ((size_t)lo << kPartCapBits) * p.stride;
       for (int i = threadIdx.x; i < kPartCap; i += blockDim.x)
         cta_store_entry(p, tab + (size_t)i * cs, region + (size_t)i * p.stride);
@@ -679,8 +786,42 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
     } else {
       for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry(p, tab + (size_t)i * cs);
     }
+    if (a.direct_emit && !(direct && !overflowed) && threadIdx.x == 0) a.dirty[lo] = 1;   // rows in the HBM range
     __syncthreads();
   }
+}
+
+// Emission of the partitions whose groups live in the HBM table (split / overflowed /
+// exact-path partitions): one CTA per partition scans its kPartCap-slot range.
+__global__ void __launch_bounds__(kPartThreads) k_part_emit_dirty(const __grid_constant__ Plan p, PartArgs a,
+                                                                  const __grid_constant__ EmitArgs ea) {
+  __shared__ uint32_t wsum[kPartThreads / 32];
+  __shared__ unsigned long long base_s;
+  const int64_t q = blockIdx.x;
+  if (!a.dirty[q] && !a.slowflag[q]) return;                  // CTA-uniform
+  constexpr int PER = kPartCap / kPartThreads;
+  const uint8_t* region = p.table + ((size_t)q << kPartCapBits) * p.stride;
+  uint32_t occ = 0;
+#pragma unroll
+  for (int k = 0; k < PER; ++k)
+    if (*(const uint64_t*)(region + (size_t)(threadIdx.x + k * kPartThreads) * p.stride) != 0) occ |= 1u << k;
+  int64_t g = part_emit_claim(__popc(occ), a.out_ctr, wsum, &base_s);
+#pragma unroll
+  for (int k = 0; k < PER; ++k)
+    if ((occ >> k) & 1u) {
+      const uint8_t* e = region + (size_t)(threadIdx.x + k * kPartThreads) * p.stride;
+      part_emit_row(ea, p.stride, e, ~*(const uint64_t*)e, g++);
+    }
+}
+
+// The side entry (key ~0), then the row count and the capacity check.
+__global__ void k_part_emit_finish(const __grid_constant__ Plan p, PartArgs a, const __grid_constant__ EmitArgs ea,
+                                   int64_t out_capacity) {
+  const uint8_t* side = p.table + (p.mask + 1) * (uint64_t)p.stride;
+  if (*(const uint64_t*)side) part_emit_row(ea, p.stride, side, ~0ULL, (int64_t)atomicAdd(a.out_ctr, 1ULL));
+  const int64_t G = (int64_t)*a.out_ctr;
+  *a.count_out = G;
+  if (G > out_capacity) set_status(p.status, OCL_ERR_CAPACITY);
 }
 
 // ------------------------------------------------------------------ host
@@ -714,12 +855,13 @@ size_t part_ws_bytes(const Plan& p, int pbits, int sms) {
   const int64_t L = 1LL << pbits;
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   const bool two = pbits > kPartLevelBits;
-  return align_up((size_t)L * 4, 256) * 6 + align_up((size_t)nchunks * 4, 256) * 2 + 512 +
+  return align_up((size_t)L * 4, 256) * 7 + align_up((size_t)nchunks * 4, 256) * 2 + 768 +
          align_up((size_t)p.n * part_rec_bytes(p.nvals), 256) * (two ? 2 : 1) + (two ? align_up(4u << kPartLevelBits, 256) : 0);
 }
 
 template <class Sh, int NV>
-static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s) {
+static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, const EmitArgs& ea,
+                            int64_t out_capacity) {
   const size_t hsm = (size_t)4 << a.pbits;
   auto kc = k_part_count<Sh, NV>;
   auto ks = k_part_scatter<Sh, NV>;
@@ -732,6 +874,10 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s) 
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   if ((e = cudaMemsetAsync(a.counts, 0, (size_t)L * 4, s))) return e;
   if ((e = cudaMemsetAsync(a.slowflag, 0, (size_t)L * 4, s))) return e;
+  if (a.direct_emit) {
+    if ((e = cudaMemsetAsync(a.dirty, 0, (size_t)L * 4, s))) return e;
+    if ((e = cudaMemsetAsync(a.out_ctr, 0, 8, s))) return e;
+  }
   count_launch(5);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
   k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
@@ -760,13 +906,20 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s) 
   const int64_t items = (p.n + kPartItem - 1) / kPartItem + L;
   const int64_t grid = std::max<int64_t>(1, std::min<int64_t>((int64_t)sms * nb, items));
   count_launch();
-  ka<<<(int)grid, kPartThreads, tsm, s>>>(p, a);
+  ka<<<(int)grid, kPartThreads, tsm, s>>>(p, a, ea);
+  if (a.direct_emit) {
+    count_launch(2);
+    k_part_emit_dirty<<<(int)L, kPartThreads, 0, s>>>(p, a, ea);
+    k_part_emit_finish<<<1, 1, 0, s>>>(p, a, ea, out_capacity);
+  }
   return cudaGetLastError();
 }
 
 // Run the partitioned tier for plan p (p.table zeroed by the caller).  *kind reports
 // the shape (30 dynamic, 31 key i64, 32 pred i32 + key i64).
-cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind) {
+cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind,
+                               const EmitArgs* ea, int64_t* count_out, int64_t out_capacity, bool* emitted) {
+  if (emitted) *emitted = false;
   if (p.n == 0) return cudaSuccess;
   PartArgs a;
   a.pbits = pbits;
@@ -805,21 +958,58 @@ cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cuda
     a.tmp = w;
     w += align_up((size_t)p.n * a.rec_bytes, 256);
     a.cur1 = (uint32_t*)w;
+    w += align_up(4u << kPartLevelBits, 256);
   }
+  a.dirty = (uint32_t*)w;
+  w += align_up((size_t)L * 4, 256);
+  a.out_ctr = (unsigned long long*)w;
+  a.count_out = count_out;
+  a.direct_emit = (ea && count_out && a.direct_ok && p.stride <= 256) ? 1 : 0;
+  EmitArgs none;
+  memset(&none, 0, sizeof(none));
+  const EmitArgs& e = ea ? *ea : none;
+  a.npo = 0;
+  if (a.direct_emit && e.kind == EMIT_FINAL) {            // outputs resolved once, not per row
+    for (int i = 0; i < e.fin.naggs; ++i) {
+      const OutAgg& o = e.fin.aggs[i];
+      auto& q = a.po[a.npo];
+      q.out = o.out;
+      q.f0 = q.f1 = 0;
+      q.kind = -1;
+      if (o.op == OCL_AGG_COUNT) q.kind = 0;
+      for (int v = 0; v < p.nvals && q.kind < 0; ++v) {
+        const DevValue& d = p.vals[v];
+        if ((o.op == OCL_AGG_SUM || o.op == OCL_AGG_AVG) && o.off == d.off_sum) {
+          q.kind = o.op == OCL_AGG_SUM ? 1 : 2;
+          q.f0 = d.co_lo;
+          q.f1 = d.co_hi;
+        } else if (o.op == OCL_AGG_MIN && o.off == d.off_min) {
+          q.kind = 3;
+          q.f0 = d.co_min;
+        } else if (o.op == OCL_AGG_MAX && o.off == d.off_max) {
+          q.kind = 4;
+          q.f0 = d.co_max;
+        }
+      }
+      if (q.kind < 0) a.direct_emit = 0;                    // unexpected aggregate: the table path
+      ++a.npo;
+    }
+  }
+  if (emitted) *emitted = a.direct_emit != 0;
   if (p.vec_ok && p.nkeys == 1 && p.npreds == 0 && values_match<PShK64>(p) && p.keys[0].col.width == 8) {
     *kind = 31;
-    return part_run<PShK64, 1>(p, a, sms, s);
+    return part_run<PShK64, 1>(p, a, sms, s, e, out_capacity);
   }
   if (p.vec_ok && p.nkeys == 1 && p.npreds == 1 && p.preds[0].col.width == 4 && !p.preds[0].is_f64 &&
       values_match<PShP32K64>(p) && p.keys[0].col.width == 8) {
     *kind = 32;
-    return part_run<PShP32K64, 1>(p, a, sms, s);
+    return part_run<PShP32K64, 1>(p, a, sms, s, e, out_capacity);
   }
   *kind = 30;
-  if (p.nvals <= 1) return part_run<DynShape, 1>(p, a, sms, s);
-  if (p.nvals <= 2) return part_run<DynShape, 2>(p, a, sms, s);
-  if (p.nvals <= 4) return part_run<DynShape, 4>(p, a, sms, s);
-  return part_run<DynShape, 6>(p, a, sms, s);
+  if (p.nvals <= 1) return part_run<DynShape, 1>(p, a, sms, s, e, out_capacity);
+  if (p.nvals <= 2) return part_run<DynShape, 2>(p, a, sms, s, e, out_capacity);
+  if (p.nvals <= 4) return part_run<DynShape, 4>(p, a, sms, s, e, out_capacity);
+  return part_run<DynShape, 6>(p, a, sms, s, e, out_capacity);
 }
 
 }  // namespace ocl
