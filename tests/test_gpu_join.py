@@ -71,3 +71,29 @@ def test_join_edge_cases():
     assert int(st.item()) == ocl.OCL_ERR_CAPACITY and int(n.item()) == 6
     with pytest.raises(ocl.OcelotError):
         jb.probe(dev(np.array([2], np.int32)))                          # dtypes differ
+
+
+@pytest.mark.parametrize("pk_build", [True, False])
+def test_join_dense_domain(pk_build):
+    """Build keys in a dense domain (range < 4 x rows, unique): the direct-array build; TPC-H orders keys
+    (8 of every 32 used) against lineitem-like foreign keys, probes below / above the range, and a dense
+    domain with a repeated key (falls back to the hash table)."""
+    import datagen
+    nb = 70007
+    pk = datagen.orders_keys(nb)                                       # sparse(o): dense within 4x
+    rng = np.random.default_rng(11)
+    fk = np.sort(rng.choice(pk, 300001))                              # clustered probe (dbgen order)
+    fk[::13] = pk.min() - 1 - (np.arange(len(fk[::13])) % 5)           # below the range
+    fk[5::17] = pk.max() + 1 + (np.arange(len(fk[5::17])) % 7)         # above the range
+    _check(pk, fk, pk_build=pk_build)
+    oids = np.flatnonzero(rng.random(len(fk)) < 0.5).astype(np.uint32)
+    _check(pk, fk, oids=oids, pk_build=pk_build)
+    dup = pk.copy()
+    dup[100] = dup[200]                                               # one repeated key
+    if pk_build:
+        jb = ocl.JoinBuild(dev(dup))
+        _, _, _, st = jb.probe(dev(fk), pk_build=True, out_capacity=2 * len(fk))
+        torch.cuda.synchronize()
+        assert int(st.item()) == ocl.OCL_ERR_INVALID_ARG
+    else:
+        _check(dup, fk, pk_build=False)
