@@ -459,6 +459,8 @@ def main():
             d2h = int(hk_.numel() * 8 + sum(o.numel() * o.element_size() for o in ho_))
         e2e = {"value": n / e2e_s, "unit": "rows/s", "h2d_bytes_per_step": int(h2d),
                "d2h_bytes_per_step": int(d2h), "steps": ke,
+               # the host link is the bound end to end: H2D bytes / step time (PCIe Gen5 x16 ~55 GB/s)
+               "h2d_gbs": h2d / e2e_s / 1e9,
                "path": "ocl_select_group_aggregate_host (pinned host columns, chunked H2D overlapped with the "
                        "fused kernel, D2H of the result)" if world == 1 else
                        "torch H2D copies + distributed fused step + D2H of the result"}
