@@ -79,3 +79,27 @@ def test_tier6_generic_and_f64():
                          by_key(rk, routs, aggs, [np.float64]), aggs, [np.float64])
     with pytest.raises(ocl.OcelotError, match="UNSUPPORTED"):
         ocl.select_group_aggregate([(dev(b), {"hi": 3})], [dev(a)], [dev(f)], aggs, tier=6)
+
+
+def test_radix_and_tier6_edges():
+    """n = 0 and n = 1; all keys equal (one run over every tile); keys at the top of the 64-bit range."""
+    e = np.zeros(0, np.int64)
+    ko, po, ro = ocl.radix_sort([dev(e)], payload=dev(e), rowids=True)
+    assert ko.numel() == 0 and po.numel() == 0 and ro.numel() == 0
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}]
+    k, outs, _ = ocl.select_group_aggregate([], [dev(e)], [dev(e)], aggs, tier=6)
+    assert k.numel() == 0
+    one = np.array([7], np.int64)
+    k, outs, _ = ocl.select_group_aggregate([], [dev(one)], [dev(one)], aggs, tier=6)
+    assert k.cpu().tolist() == [7] and outs[0].cpu().tolist() == [1]
+    n = 100000
+    same = np.full(n, 123456789, np.int64)
+    v = np.arange(n, dtype=np.int64)
+    k, outs, _ = ocl.select_group_aggregate([], [dev(same)], [dev(v)], aggs, out_capacity=4, tier=6)
+    assert k.cpu().tolist() == [123456789] and outs[0].cpu().tolist() == [n]
+    assert int(outs[1][0, 0].item()) == n * (n - 1) // 2
+    top = (np.uint64(2**64 - 1) - np.arange(1000, dtype=np.uint64) % 7).view(np.int64)
+    ko, _, ro = ocl.radix_sort([dev(top)], rowids=True)
+    perm = np.argsort(top.view(np.uint64), kind="stable")
+    assert np.array_equal(ko.cpu().numpy(), top[perm])
+    assert np.array_equal(ro.cpu().numpy().view(np.uint32), perm.astype(np.uint32))
