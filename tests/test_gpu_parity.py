@@ -486,3 +486,34 @@ def test_cuda_graph_replay():
     rk, routs = oracle.sga([], [li["orderkey"]], [li["quantity"]], aggs, order_by_key=True)
     assert np.array_equal(keys.cpu().numpy(), rk)
     assert all(np.array_equal(o.cpu().numpy(), r) for o, r in zip(outs, routs))
+
+
+@pytest.mark.parametrize("G", [50000, 1 << 20])
+def test_partitioned_partials_merge(G):
+    """Partial rows from the hash-partitioned tier (tier 5: rows emitted straight from shared memory as
+    partial rows, dirty partitions from the HBM table) -> merge == oracle; values beyond int32 and the
+    key ~0 force exact-path (dirty) partitions."""
+    from paper_journals_pvldb_heimelspmm13_b200.distributed import shard_range
+    rng = np.random.default_rng(G)
+    n, P = (1 << 21) + 3, 2
+    keys = rng.integers(0, G, n).astype(np.int64) * 2654435761 % (1 << 40)
+    keys[::4099] = -1                                                   # key ~0
+    v = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    v[::10007] = 1 << 40                                                # beyond int32: exact path
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    cap = 2 * G + 16
+    parts, counts = [], []
+    for r in range(P):
+        s0, ln = shard_range(n, r, P)
+        call = ocl.SgaCall([], [dev(keys[s0:s0 + ln])], [dev(v[s0:s0 + ln])], aggs, expected_groups=G,
+                           out_capacity=cap, tier=5)
+        part, cnt = ocl.sga_partial(call, cap)
+        parts.append(part)
+        counts.append(cnt)
+    call = ocl.SgaCall([], [dev(keys)], [dev(v)], aggs, expected_groups=G, out_capacity=cap)
+    ocl.merge_partials(call, torch.stack(parts).contiguous(), torch.cat(counts), P, cap)
+    k, outs = call.result()
+    rk, routs = oracle.sga([], [keys], [v], aggs)
+    dts = [np.int64]
+    assert_results_equal(by_key(k.cpu().numpy(), [o.cpu().numpy() for o in outs], aggs, dts),
+                         by_key(rk, routs, aggs, dts), aggs, dts)
