@@ -207,14 +207,31 @@ struct TileMap {
   uint32_t off[kTileMap];                  // the slot's first index in the staging area
   uint16_t sslot[kPartILP * kPartThreads]; // slot of each staged item
   uint4 stage[kPartILP * kPartThreads];    // the tile's records, grouped by partition
+  uint16_t used[kPartILP * kPartThreads];  // slots taken in this tile (a tile meets ~128 of the 4096)
+  uint32_t nused;
   uint32_t total;                          // items in the tile
 };
 
-__device__ __forceinline__ void tile_map_clear(TileMap& m) {
+// Whole map empty (once per CTA; the caller synchronises).
+__device__ __forceinline__ void tile_map_init(TileMap& m) {
   for (int i = threadIdx.x; i < kTileMap; i += blockDim.x) {
     m.key[i] = 0xFFFFFFFFu;
     m.cnt[i] = 0;
   }
+  if (threadIdx.x == 0) m.nused = 0;
+}
+
+// Empty again after a tile: only the slots the tile used (instead of all 4096 — the
+// per-tile clear and the claim scan over the whole map dominated the scatter passes).
+__device__ __forceinline__ void tile_map_reset(TileMap& m) {
+  const uint32_t nu = m.nused;
+  __syncthreads();
+  for (uint32_t i = threadIdx.x; i < nu; i += blockDim.x) {
+    const uint32_t sl = m.used[i];
+    m.key[sl] = 0xFFFFFFFFu;
+    m.cnt[sl] = 0;
+  }
+  if (threadIdx.x == 0) m.nused = 0;
 }
 
 // slot of `part` in the map (inserted if new) and this item's rank within it
@@ -226,7 +243,11 @@ __device__ __forceinline__ void tile_map_add(TileMap& m, uint32_t part, uint32_t
     if (cur == part) break;
     if (cur == 0xFFFFFFFFu) {
       const uint32_t prev = atomicCAS(&m.key[h], 0xFFFFFFFFu, part);
-      if (prev == 0xFFFFFFFFu || prev == part) break;
+      if (prev == 0xFFFFFFFFu) {
+        m.used[atomicAdd(&m.nused, 1u)] = (uint16_t)h;
+        break;
+      }
+      if (prev == part) break;
     }
     h = (h + 1) & (kTileMap - 1);
   }
@@ -234,45 +255,38 @@ __device__ __forceinline__ void tile_map_add(TileMap& m, uint32_t part, uint32_t
   rank = atomicAdd(&m.cnt[h], 1u);
 }
 
-// After a barrier: counts -> global bases, and each slot's offset in the staging area
-// (exclusive scan of the counts: kPartThreads threads x kTileMap / kPartThreads slots).
+// After a barrier: counts -> global bases, and each used slot's offset in the staging
+// area (exclusive scan of the used slots' counts, 256 at a time).
 __device__ __forceinline__ void tile_map_claim(TileMap& m, uint32_t* cur, uint32_t* wsum) {
-  constexpr int PER = kTileMap / kPartThreads;
   const int t = threadIdx.x, lane = t & 31, w = t >> 5;
-  uint32_t c[PER], tot = 0;
-#pragma unroll
-  for (int i = 0; i < PER; ++i) {
-    c[i] = m.cnt[t * PER + i];
-    tot += c[i];
-  }
-  uint32_t incl = tot;
-#pragma unroll
-  for (int o = 1; o < 32; o <<= 1) {
-    const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
-    if (lane >= o) incl += y;
-  }
-  if (lane == 31) wsum[w] = incl;
-  __syncthreads();
-  if (w == 0) {
-    const uint32_t x = lane < kPartThreads / 32 ? wsum[lane] : 0u;
-    uint32_t xi = x;
+  const uint32_t nu = m.nused;
+  uint32_t run0 = 0;
+  for (uint32_t b0 = 0; b0 < nu; b0 += kPartThreads) {
+    const uint32_t i = b0 + t;
+    const uint32_t sl = i < nu ? m.used[i] : 0u;
+    const uint32_t c = i < nu ? m.cnt[sl] : 0u;
+    uint32_t incl = c;
 #pragma unroll
     for (int o = 1; o < 32; o <<= 1) {
-      const uint32_t y = __shfl_up_sync(0xffffffffu, xi, o);
-      if (lane >= o) xi += y;
+      const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+      if (lane >= o) incl += y;
     }
-    if (lane < kPartThreads / 32) wsum[lane] = xi - x;
-  }
-  __syncthreads();
-  uint32_t run = wsum[w] + incl - tot;
+    if (lane == 31) wsum[w] = incl;
+    __syncthreads();
+    uint32_t off = 0, tot = 0;
 #pragma unroll
-  for (int i = 0; i < PER; ++i) {
-    const int sl = t * PER + i;
-    m.off[sl] = run;
-    run += c[i];
-    if (c[i]) m.cnt[sl] = atomicAdd(&cur[m.key[sl]], c[i]);
+    for (int k = 0; k < kPartThreads / 32; ++k) {
+      off += k < w ? wsum[k] : 0u;
+      tot += wsum[k];
+    }
+    if (i < nu) {
+      m.off[sl] = run0 + off + incl - c;
+      m.cnt[sl] = atomicAdd(&cur[m.key[sl]], c);
+    }
+    run0 += tot;
+    __syncthreads();
   }
-  if (t == kPartThreads - 1) m.total = run;
+  if (t == 0) m.total = run0;
 }
 
 // Stage item (slot, rank) in the tile's partition-grouped order.
@@ -335,8 +349,10 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter(const __grid_cons
   bool nok[kPartILP];
   const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
   if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
+  tile_map_init(map);
+  __syncthreads();
   for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
-    tile_map_clear(map);
+    tile_map_reset(map);
     Row<Sh, NV, false> x[kPartILP];
     bool ok[kPartILP];
     uint32_t slot[kPartILP], rank[kPartILP];
@@ -399,8 +415,10 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter2(PartArgs a) {
     }
   };
   if (j0 < j1) fetch(j0);
+  tile_map_init(map);
+  __syncthreads();
   for (int64_t base = j0; base < j1; base += TILE) {
-    tile_map_clear(map);
+    tile_map_reset(map);
     uint64_t key[kPartILP];
     int32_t v[kPartILP][NV > 0 ? NV : 1];
     bool ok[kPartILP];
