@@ -319,8 +319,10 @@ ocl_status plan_preds(const ocl_column* pred_cols, const ocl_range* preds, int32
 
 // Shared-memory budget of one register-tier CTA (private records + mid-G table).
 constexpr size_t kRegTierSmem = 200 * 1024;
-// Auto selection of the hash-partitioned tier.
-constexpr int64_t kPartMinGroups = 4096;
+// Auto selection of the hash-partitioned tier: above 1024 expected groups
+// it beats the fused kernel's shared-memory CTA table (C5, 2^28 rows, sel 100 %: 2048
+// groups 10.6 -> 8.8 ms, 4096 groups 14.7 -> 8.5 ms; at 1024 the fused kernel wins).
+constexpr int64_t kPartMinGroups = 1024;
 constexpr int64_t kPartMinRows = 1 << 20;
 
 // Tier selection: 0 auto; 1 register tier (private slots + HBM);
@@ -385,7 +387,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   // High-cardinality tier: more groups than the shared-memory tiers hold, integer
   // column values, enough rows to amortise its five launches (tier 5 forces it).
   P->pbits = -1;
-  const bool many = a->tier == 0 && p.smem_cap == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
+  const bool many = a->tier == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
   if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
   P->sorted = a->key_sorted != 0;
   P->sortgrp = a->tier == 6;
