@@ -374,61 +374,74 @@ __device__ __forceinline__ void spec_row_scalar(const SpecPlan& p, int64_t r, SR
   spec_values<S>(p, c, x);
 }
 
-// Flush: each consumer warp reduces its lanes' private accumulators -> CTA entry ->
-// global table (one thread per slot).  Every thread of the CTA calls it (barriers);
-// threads tid >= T (a producer warp) only take part in the barriers.
+// Flush: the CTA's T private records of every (slot, field) are summed in parallel --
+// Q threads per (slot, field), each over T/Q records, then Q-lane shuffles -- and added
+// into the slot's global entry.  (A warp-by-warp shuffle tree per (slot, field) was a
+// serial chain of ~NV x 5 dependent shuffles per slot: on C1, one chunk per CTA, that
+// chain was most of the kernel.)  One thread per slot resolves the entry first.
+// Every thread of the CTA calls it (barriers); threads tid >= T (a producer warp) only
+// take part in the barriers.
 template <class S, int L, int T>
 __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm, const uint64_t* dir, uint64_t* blk,
                                            int tid) {
   using A = Acc<S>;
-  const int lane = tid & 31;
-  __syncthreads();
-  uint8_t* blkb = (uint8_t*)blk;
-  if (tid < T) {
-#pragma unroll
-    for (int s = 0; s < L; ++s) {
-      if (dir[s] == 0) continue;
-      uint8_t* be = blkb + s * 256;
-      const uint8_t* sb = sm + (size_t)s * A::slot_bytes(T);
-      uint32_t cw = __reduce_add_sync(0xffffffffu, ((const uint32_t*)sb)[tid]);
-      if (lane == 0) atomicAdd((unsigned long long*)(be + 8), (unsigned long long)cw);
-#pragma unroll
-      for (int v = 0; v < S::NV; ++v) {
-        const int off = p.g.vals[v].off_sum;
-        if constexpr (S::F64) {
-          double sum = ((const double*)(sb + A::f_dbl(v, T)))[tid];
-          for (int o = 16; o > 0; o >>= 1) sum += __shfl_xor_sync(0xffffffffu, sum, o);
-          if (lane == 0 && off >= 0) atomicAdd((double*)(be + off), sum);
-        } else {
-          I128 x;
-          if (vx_kind(S::OP(v)) == VX_COL) {
-            x = i128_from_i64(((const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)))[tid]);
-          } else {
-            x.lo = ((const uint64_t*)(sb + A::f_wlo(A::wide_idx(v), T)))[tid];
-            x.hi = (uint64_t)(int64_t)(int32_t)((const uint32_t*)(sb + A::f_whi(A::wide_idx(v), T)))[tid];
-          }
-          x = warp_sum_i128(x);
-          if (lane == 0 && off >= 0) atomic_add_i128((uint64_t*)(be + off), x.lo, x.hi);
-        }
-      }
-    }
-  }
+  (void)blk;
+  constexpr int Q = 4;                     // threads per (slot, field)
+  constexpr int PER = T / Q;               // records each of them sums
+  constexpr int F = 1 + S::NV;             // COUNT + the value sums
+  static_assert(T % (32 * Q) == 0 || 32 % Q == 0, "Q lanes of a group share a warp");
+  __shared__ uint8_t* ent[L];
   __syncthreads();
   if (tid < L) {
-    const int s = tid;
-    uint64_t sk = dir[s];
-    if (sk != 0) {
-      const uint8_t* be = blkb + s * 256;
-      uint8_t* e = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, ~sk, p.g.status);
-      if (e) {
-        atomicAdd((unsigned long long*)(e + 8), (unsigned long long)*(const uint64_t*)(be + 8));
-        for (int v = 0; v < S::NV; ++v) {
-          const int off = p.g.vals[v].off_sum;
-          if (off < 0) continue;
-          if constexpr (S::F64) atomicAdd((double*)(e + off), *(const double*)(be + off));
-          else atomic_add_i128((uint64_t*)(e + off), *(const uint64_t*)(be + off), *(const uint64_t*)(be + off + 8));
-        }
+    const uint64_t sk = dir[tid];
+    ent[tid] = sk != 0 ? table_find_or_insert(p.g.table, p.g.mask, p.g.stride, ~sk, p.g.status) : nullptr;
+  }
+  __syncthreads();
+  if (tid >= T) return;
+  const int sub = tid % Q;
+  const unsigned gmask = ((1u << Q) - 1) << ((tid & 31) & ~(Q - 1));
+  for (int i = tid / Q; i < L * F; i += T / Q) {   // uniform within a Q group
+    const int s = i / F, v = i % F - 1;
+    uint8_t* e = ent[s];
+    if (e == nullptr) continue;
+    const uint8_t* sb = sm + (size_t)s * A::slot_bytes(T);
+    const int j0 = sub * PER;
+    if (v < 0) {
+      const uint32_t* c = (const uint32_t*)sb + j0;
+      unsigned long long cw = 0;
+#pragma unroll 8
+      for (int j = 0; j < PER; ++j) cw += c[j];
+      for (int o = Q / 2; o > 0; o >>= 1) cw += __shfl_xor_sync(gmask, cw, o);
+      if (sub == 0 && cw) atomicAdd((unsigned long long*)(e + 8), cw);
+      continue;
+    }
+    const int off = p.g.vals[v].off_sum;
+    if constexpr (S::F64) {
+      const double* d = (const double*)(sb + A::f_dbl(v, T)) + j0;
+      double sum = 0.0;
+#pragma unroll 8
+      for (int j = 0; j < PER; ++j) sum += d[j];
+      for (int o = Q / 2; o > 0; o >>= 1) sum += __shfl_xor_sync(gmask, sum, o);
+      if (sub == 0 && off >= 0) atomicAdd((double*)(e + off), sum);
+    } else {
+      I128 x{0, 0};
+      if (vx_kind(S::OP(v)) == VX_COL) {
+        const int64_t* d = (const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)) + j0;
+#pragma unroll 8
+        for (int j = 0; j < PER; ++j) x = i128_add(x, i128_from_i64(d[j]));
+      } else {
+        const uint64_t* lo = (const uint64_t*)(sb + A::f_wlo(A::wide_idx(v), T)) + j0;
+        const uint32_t* hi = (const uint32_t*)(sb + A::f_whi(A::wide_idx(v), T)) + j0;
+#pragma unroll 8
+        for (int j = 0; j < PER; ++j) x = i128_add(x, I128{lo[j], (uint64_t)(int64_t)(int32_t)hi[j]});
       }
+      for (int o = Q / 2; o > 0; o >>= 1) {
+        I128 y;
+        y.lo = __shfl_xor_sync(gmask, x.lo, o);
+        y.hi = __shfl_xor_sync(gmask, x.hi, o);
+        x = i128_add(x, y);
+      }
+      if (sub == 0 && off >= 0) atomic_add_i128((uint64_t*)(e + off), x.lo, x.hi);
     }
   }
 }
