@@ -9,8 +9,8 @@
 // Two kernels: k_sga_priv loads the columns into registers (vector LDG, two units in
 // flight per warp); k_sga_bulk (default) streams them into shared memory with TMA
 // bulk copies (cp.async.bulk + mbarrier ring, one producer warp) so the consumer
-// warps only compute.  On B200 C4 (600M rows) k_sga_bulk runs in ~3.5-3.6 ms
-// (~6.4 TB/s, ~97 % of the measured copy bandwidth); the generic StaticShape
+// warps only compute.  On B200 C4 (600M rows) k_sga_bulk runs in ~3.45 ms
+// (~6.6 TB/s, ~101 % of the measured copy bandwidth); the generic StaticShape
 // instantiation of k_sga takes 5.1-5.5 ms.  launch_fused (fused.cu)
 // tries these kernels first for few-group plans; OCL_NO_SPEC=1 disables them.
 #include <type_traits>
