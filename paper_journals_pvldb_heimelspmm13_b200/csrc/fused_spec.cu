@@ -758,20 +758,23 @@ static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t
 // Pipeline configuration, OCL_BULK = 0: off (the register-load kernel k_sga_priv);
 // else <consumer threads, rows per stage, stages>: 1 = <256, 1024, 4>, 2 = <256, 512, 3>,
 // 3 = <256, 512, 2>, 4 = <256, 512, 1>, 5 = <128, 256, 2>, 6 = <128, 256, 3>,
-// 7 = <128, 512, 2> (default: 3 CTAs x 4 consumer warps per SM; measured on B200 C4,
-// profiles/r01_c4_bulk_configs.md).
+// 7 = <128, 512, 2>.  Default (OCL_BULK unset): 7 for int64 plans (3 CTAs x 4 consumer
+// warps per SM; measured on B200 C4, profiles/r01_c4_bulk_configs.md), 3 for fp64 plans
+// (C2: 51.0 -> 48.9 us, two sweeps agree, profiles/r01_c2_bulk_configs.md).
 static int bulk_config() {
-  static int cfg = -1;
-  if (cfg < 0) {
+  static int cfg = -2;
+  if (cfg == -2) {
     const char* e = getenv("OCL_BULK");
-    cfg = e ? atoi(e) : 7;
+    cfg = e ? atoi(e) : -1;
   }
   return cfg;
 }
 
 template <class S>
 static bool launch_bulk_cfg(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err) {
-  switch (bulk_config()) {
+  int cfg = bulk_config();
+  if (cfg < 0) cfg = S::F64 ? 3 : 7;
+  switch (cfg) {
     case 1: return launch_bulk<S, 256, 1024, 4>(sp, sms, s, err);
     case 2: return launch_bulk<S, 256, 512, 3>(sp, sms, s, err);
     case 3: return launch_bulk<S, 256, 512, 2>(sp, sms, s, err);
