@@ -21,7 +21,7 @@ $(OBJDIR)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 
 $(LIB): $(COBJ)
 	@mkdir -p $(PKG)/_lib
-	$(NVCC) $(ARCH) -shared -o $@ $(COBJ) -lcudart
+	$(NVCC) $(ARCH) -shared -o $@ $(COBJ) -lcudart -ldl
 	@cat $(OBJDIR)/*.ptxas.log > $(PKG)/_lib/ptxas.log
 
 # oracle: test infrastructure only; plain C++17, single-threaded, no FMA contraction

@@ -195,6 +195,34 @@ def profiled_traffic(workload, rows):
         return None
 
 
+class pinned_one_core:
+    """Run the oracle on ONE host core (sched_setaffinity; SURVEY §8(d) "single-threaded, pinned to 1
+    core"); restores the previous affinity."""
+
+    def __enter__(self):
+        self.prev = os.sched_getaffinity(0)
+        self.core = max(self.prev)
+        os.sched_setaffinity(0, {self.core})
+        return self.core
+
+    def __exit__(self, *exc):
+        os.sched_setaffinity(0, self.prev)
+
+
+def host_cpu(core):
+    model = "unknown"
+    try:
+        with open("/proc/cpuinfo") as f:
+            for line in f:
+                if line.startswith("model name"):
+                    model = line.split(":", 1)[1].strip()
+                    break
+    except OSError:
+        pass
+    return {"pinned_core": core, "host_cores": os.cpu_count(), "cpu_model": model,
+            "note": f"1 of {os.cpu_count()} host cores ({model}), pinned with sched_setaffinity"}
+
+
 def oracle_time(wl, cols, rows):
     import oracle
     p, k, v, a, _ = workload_columns(wl, {f: c[:rows] for f, c in cols.items()})
@@ -211,7 +239,8 @@ def run_reference(args, wl, rank):
     cols = gen_host(wl, sample, 0, wl["rows"])
     for _ in range(args.warmup):
         oracle_time(wl, cols, sample)
-    ts = [oracle_time(wl, cols, sample) for _ in range(args.steps)]
+    with pinned_one_core() as core:
+        ts = [oracle_time(wl, cols, sample) for _ in range(args.steps)]
     ms = 1e3 * statistics.mean(ts)
     value = sample / (ms / 1e3)
     desc = f"first {sample:,} rows of the {wl['rows']:,}-row workload per step, oracle.sga single-threaded"
@@ -220,7 +249,8 @@ def run_reference(args, wl, rank):
             "scaling": "strong", "vs_baseline": None, "dtype": "int64" if not wl["f64"] else "f64",
             "data": "synthetic (seeded lineitem-shaped generator, datagen/)",
             "config": {"workload": wl["desc"], "rows": wl["rows"], "sample_rows": sample},
-            "cpu_baseline": {"value": value, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": desc},
+            "cpu_baseline": {"value": value, "unit": "rows/s", "cores": 1, "kind": "oracle", "sample": desc,
+                             **host_cpu(core)},
             "e2e": {"value": value, "unit": "rows/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0}}
     print(json.dumps(line), flush=True)
 
@@ -306,6 +336,11 @@ def main():
     ap.add_argument("--c5-groups", type=int, default=1 << 10, help="C5: key cardinality G")
     ap.add_argument("--c5-zipf", type=float, default=0.0, help="C5: Zipf exponent s (0 = uniform)")
     ap.add_argument("--c5-sel", type=float, default=1.0, help="C5: selectivity (0.01, 0.5, 1.0)")
+    ap.add_argument("--dist", action="store_true",
+                    help="1 GPU: run the distributed path (partial -> NCCL exchange -> merge in the library) on a "
+                         "world-size-1 communicator, to measure its overhead (always on for N > 1)")
+    ap.add_argument("--dist-mode", default="auto", choices=["auto", "allgather", "alltoall"],
+                    help="exchange of the distributed path (auto: allgather for partial tables <= 1 MB)")
     args = ap.parse_args()
     wl = dict(WORKLOADS[args.workload])
     if args.no_sorted and wl.get("sorted"):
@@ -330,7 +365,7 @@ def main():
         import torch.distributed as dist
         dist.init_process_group("nccl", device_id=dev)
     import paper_journals_pvldb_heimelspmm13_b200 as ocl
-    from paper_journals_pvldb_heimelspmm13_b200.distributed import distributed_select_group_aggregate, shard_range
+    from paper_journals_pvldb_heimelspmm13_b200.distributed import shard_range
 
     n = wl["rows"]
     start, length = shard_range(n, rank, world)
@@ -338,11 +373,28 @@ def main():
     torch.cuda.synchronize()
     p, k, v, aggs, bpr = workload_columns(wl, cols)
     order = wl["kind"] == "q1"
-    eg = wl["groups"] if world == 1 else wl["groups"]
+    eg = wl["groups"]
     key_sorted = bool(wl.get("sorted"))
     tier = args.tier or wl.get("tier", 0)
+    # multi-GPU: the library exchanges the partial tables itself over an NCCL communicator
+    # (ocl_ctx_attach_nccl + ocl_sga_args.distributed; no host sync inside a step)
+    distributed = 0
+    dctx = None
+    if world > 1 or args.dist:
+        if world == 1:
+            import torch.distributed as dist
+            dctx = ocl.Context(local)
+            dctx.attach_nccl(ocl.nccl_unique_id(), 0, 1)
+        else:
+            dctx = ocl.attach_nccl(local)
+        probe = ocl.SgaCall(p, k, v, aggs, expected_groups=eg, out_capacity=max(16, 2 * eg), tier=tier,
+                            key_sorted=key_sorted)
+        small = max(16, 2 * eg) * ocl.partial_row_bytes(probe) <= (1 << 20)
+        del probe
+        distributed = {"allgather": 1, "alltoall": 2}.get(args.dist_mode, 1 if small else 2)
+        order = order and distributed == 1
     call = ocl.SgaCall(p, k, v, aggs, expected_groups=eg, out_capacity=max(16, 2 * eg), order_by_key=order,
-                       tier=tier, key_sorted=key_sorted)
+                       tier=tier, key_sorted=key_sorted, distributed=distributed, ctx=dctx)
     ctx = call.ctx
     # inputs smaller than 2x the 126 MB L2 are flushed before every step (a 512 MB write)
     flush = torch.empty(512 << 20, dtype=torch.uint8, device=dev) if bpr * length < (256 << 20) else None
@@ -357,10 +409,8 @@ def main():
     def step():
         if graph is not None:
             graph.replay()
-        elif world == 1:
-            call.launch()
         else:
-            distributed_select_group_aggregate(call)
+            call.launch()
 
     clk = ClockSampler(local).start()
     for _ in range(args.warmup):
@@ -376,6 +426,10 @@ def main():
         b.record()
     t0, t1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     sev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(K)]
+    xev = [(torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)) for _ in range(K)]
+    for a, b in xev:
+        a.record()
+        b.record()
     if world > 1:
         dist.barrier()
     torch.cuda.synchronize()
@@ -385,6 +439,8 @@ def main():
     for i in range(K):
         if graph is None:
             ocl.set_kernel_events(ctx, kev[i][0], kev[i][1])
+            if distributed:
+                ocl.set_phase_events(ctx, 1, xev[i][0], xev[i][1])
         if flush is not None:
             flush.zero_()
         sev[i][0].record()
@@ -396,6 +452,7 @@ def main():
     clk.window(h0, h1)
     clk.stop()
     ocl.set_kernel_events(ctx, None, None)
+    ocl.set_phase_events(ctx, 1, None, None)
     kernel_name = ocl.last_kernel(ctx)
     launches = ocl.launch_count() - launches0
     if world > 1:
@@ -406,10 +463,11 @@ def main():
     kms = statistics.mean(a.elapsed_time(b) for a, b in (kev if graph is None else sev))
     if graph is not None:
         launches = per_call * K
+    xms = statistics.mean(a.elapsed_time(b) for a, b in xev) if distributed and graph is None else None
     if world > 1:
-        tt = torch.tensor([ms, kms], dtype=torch.float64, device=dev)
+        tt = torch.tensor([ms, kms, xms or 0.0], dtype=torch.float64, device=dev)
         dist.all_reduce(tt, op=dist.ReduceOp.MAX)
-        ms, kms = tt.tolist()
+        ms, kms, xms = tt.tolist()
     value = n / (ms / 1e3)
     peak, peak_src = measured_peak_gbs()
     out_bytes = G * (8 + sum(o.element_size() * (o[0].numel() if o.dim() > 1 else 1) for o in outs))
@@ -423,57 +481,45 @@ def main():
         gen_host(wl, length, start, n, out={f: h.numpy() for f, h in host.items()})
         hp, hk, hv, haggs, _ = workload_columns(wl, host)
         h2d = sum(h.numel() * h.element_size() for h in host.values())
-        if world == 1:
-            hcall = ocl.SgaCall(hp, hk, hv, haggs, expected_groups=eg, out_capacity=max(16, 2 * eg),
-                                order_by_key=order, tier=args.tier, host=True, chunk_rows=1 << 24)
-            # (the host-buffer entry streams chunks through the one-pass hash kernel, also for sorted input)
-            hcall.launch()                                     # warm-up
-            ke = max(1, args.e2e_steps)
-            torch.cuda.synchronize()
-            te = time.perf_counter()
-            for _ in range(ke):
-                hcall.launch()                                 # blocks until results are on the host
-            e2e_s = (time.perf_counter() - te) / ke
-            hk_, ho_ = hcall.result()
-            d2h = 8 + 4 + len(hk_) * 8 + sum(o.numel() * o.element_size() for o in ho_)
-        else:
-            dcols = {f: torch.empty_like(c) for f, c in cols.items()}
-            dp, dk, dv, daggs, _ = workload_columns(wl, dcols)
-            dcall = ocl.SgaCall(dp, dk, dv, daggs, expected_groups=eg, out_capacity=max(16, 2 * eg),
-                                order_by_key=order, tier=args.tier)
-            ke = max(1, args.e2e_steps)
+        # ocl_select_group_aggregate_host: pinned host shard -> chunked H2D overlapped with the fused kernel
+        # (-> partial exchange + merge over NCCL when distributed) -> D2H of the result; blocking
+        hcall = ocl.SgaCall(hp, hk, hv, haggs, expected_groups=eg, out_capacity=max(16, 2 * eg),
+                            order_by_key=order, tier=args.tier, host=True, chunk_rows=1 << 24,
+                            distributed=distributed, ctx=dctx, device=dev)
+        # (the host-buffer entry streams chunks through the one-pass hash kernel, also for sorted input)
+        hcall.launch()                                     # warm-up
+        ke = max(1, args.e2e_steps)
+        if world > 1:
             dist.barrier()
-            torch.cuda.synchronize()
-            te = time.perf_counter()
-            for _ in range(ke):
-                for f in dcols:
-                    dcols[f].copy_(host[f], non_blocking=True)
-                distributed_select_group_aggregate(dcall)
-                hk_ = dcall.keys_out.cpu()
-                ho_ = [o.cpu() for o in dcall.outs]
-            torch.cuda.synchronize()
-            e2e_s = (time.perf_counter() - te) / ke
+        torch.cuda.synchronize()
+        te = time.perf_counter()
+        for _ in range(ke):
+            hcall.launch()                                 # blocks until results are on the host
+        e2e_s = (time.perf_counter() - te) / ke
+        if world > 1:
             tt = torch.tensor([e2e_s], dtype=torch.float64, device=dev)
             dist.all_reduce(tt, op=dist.ReduceOp.MAX)
             e2e_s = tt.item()
-            d2h = int(hk_.numel() * 8 + sum(o.numel() * o.element_size() for o in ho_))
+        hk_, ho_ = hcall.result()
+        d2h = 8 + 4 + len(hk_) * 8 + sum(o.numel() * o.element_size() for o in ho_)
         e2e = {"value": n / e2e_s, "unit": "rows/s", "h2d_bytes_per_step": int(h2d),
                "d2h_bytes_per_step": int(d2h), "steps": ke,
                # the host link is the bound end to end: H2D bytes / step time (PCIe Gen5 x16 ~55 GB/s)
                "h2d_gbs": h2d / e2e_s / 1e9,
                "path": "ocl_select_group_aggregate_host (pinned host columns, chunked H2D overlapped with the "
-                       "fused kernel, D2H of the result)" if world == 1 else
-                       "torch H2D copies + distributed fused step + D2H of the result"}
+                       "fused kernel" + (", NCCL partial exchange + merge" if distributed else "") +
+                       ", D2H of the result)"}
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu:
         sample = min(n, args.cpu_rows)
         hcols = {f: h.numpy()[:sample] for f, h in host.items()} if e2e is not None else \
             gen_host(wl, sample, 0, n)
-        dt = oracle_time(wl, hcols, sample)
+        with pinned_one_core() as core:
+            dt = oracle_time(wl, hcols, sample)
         cpu = {"value": sample / dt, "unit": "rows/s", "cores": 1, "kind": "oracle",
                "sample": f"first {sample:,} rows of the same workload, oracle.sga (C++17, single thread), "
-                         f"{dt:.1f} s"}
+                         f"{dt:.1f} s", **host_cpu(core)}
 
     if rank == 0:
         line = {
@@ -496,6 +542,10 @@ def main():
                          "achieved_with_output": (algo_bytes + out_bytes) / (kms / 1e3) / 1e9,
                          "output_bytes_per_launch": out_bytes},
             "hbm_frac_step": algo_bytes / (ms / 1e3) / 1e9 / peak,
+            "exchange": None if not distributed else {
+                "mode": "allgather" if distributed == 1 else "alltoall", "ms": xms,
+                "what": "NCCL exchange of partial tables + merge + finalise inside ocl_select_group_aggregate "
+                        "(phase-1 events, max over ranks)", "world": world},
             "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches, "clocks": clk.summary(),
         }
         print(json.dumps(line), flush=True)

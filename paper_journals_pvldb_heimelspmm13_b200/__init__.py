@@ -24,7 +24,8 @@ import torch
 _HERE = os.path.dirname(os.path.abspath(__file__))
 LIB_PATH = os.environ.get("OCL_LIB_PATH") or os.path.join(_HERE, "_lib", "libocelot_b200.so")
 
-OCL_OK, OCL_ERR_INVALID_ARG, OCL_ERR_UNSUPPORTED, OCL_ERR_CAPACITY, OCL_ERR_OUT_OF_MEMORY, OCL_ERR_CUDA = range(6)
+(OCL_OK, OCL_ERR_INVALID_ARG, OCL_ERR_UNSUPPORTED, OCL_ERR_CAPACITY, OCL_ERR_OUT_OF_MEMORY, OCL_ERR_CUDA,
+ OCL_ERR_NCCL) = range(7)
 _DTYPE = {torch.uint8: 1, torch.int32: 2, torch.int64: 3, torch.float64: 4}
 _OPS = {"count": 0, "sum": 1, "min": 2, "max": 3, "avg": 4}
 _EXPRS = {"col": 0, "mul_1minus": 1, "mul_1minus_1plus": 2}
@@ -38,7 +39,7 @@ class OcelotError(RuntimeError):
 
 
 _STATUS_NAMES = {0: "OCL_OK", 1: "OCL_ERR_INVALID_ARG", 2: "OCL_ERR_UNSUPPORTED", 3: "OCL_ERR_CAPACITY",
-                 4: "OCL_ERR_OUT_OF_MEMORY", 5: "OCL_ERR_CUDA"}
+                 4: "OCL_ERR_OUT_OF_MEMORY", 5: "OCL_ERR_CUDA", 6: "OCL_ERR_NCCL"}
 
 
 class Column(ctypes.Structure):
@@ -65,7 +66,7 @@ class SgaArgs(ctypes.Structure):
                 ("expected_groups", ctypes.c_int64), ("out_capacity", ctypes.c_int64),
                 ("keys_out", ctypes.c_void_p), ("ngroups_out", ctypes.c_void_p), ("bitmap_out", ctypes.c_void_p),
                 ("dev_status", ctypes.c_void_p), ("order_by_key", ctypes.c_int32), ("tier", ctypes.c_int32),
-                ("key_sorted", ctypes.c_int32), ("reserved_", ctypes.c_int32)]
+                ("key_sorted", ctypes.c_int32), ("distributed", ctypes.c_int32)]
 
 
 _lib = None
@@ -98,6 +99,12 @@ def lib():
             "ocl_group_aggregate": [P, P, P, P, I64, P, I64, P, I32, P, I32, P, SZ, P],
             "ocl_select_group_aggregate_workspace_size": [P, P, PSZ],
             "ocl_select_group_aggregate": [P, P, P, SZ, P],
+            "ocl_select_group_aggregate_sync_workspace_size": [P, P, PSZ],
+            "ocl_select_group_aggregate_sync": [P, P, P, SZ, P],
+            "ocl_ctx_set_phase_events": [P, I32, P, P],
+            "ocl_nccl_unique_id": [P],
+            "ocl_ctx_attach_nccl": [P, P, I32, I32],
+            "ocl_ctx_nccl_rank": [P, ctypes.POINTER(I32), ctypes.POINTER(I32)],
             "ocl_partial_row_bytes": [P, PSZ],
             "ocl_sga_partial": [P, P, P, I64, P, P, SZ, P],
             "ocl_merge_partials_workspace_size": [P, P, I32, I64, PSZ],
@@ -136,7 +143,10 @@ ABI_SYMBOLS = ("ocl_ctx_create", "ocl_ctx_destroy", "ocl_status_string", "ocl_la
                "ocl_group_build_sorted_workspace_size", "ocl_group_build_sorted",
                "ocl_group_build_paper_workspace_size", "ocl_group_build_paper",
                "ocl_group_aggregate_workspace_size", "ocl_group_aggregate",
-               "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate", "ocl_partial_row_bytes",
+               "ocl_select_group_aggregate_workspace_size", "ocl_select_group_aggregate",
+               "ocl_select_group_aggregate_sync_workspace_size", "ocl_select_group_aggregate_sync",
+               "ocl_ctx_set_phase_events", "ocl_nccl_unique_id", "ocl_ctx_attach_nccl", "ocl_ctx_nccl_rank",
+               "ocl_partial_row_bytes",
                "ocl_sga_partial", "ocl_merge_partials_workspace_size", "ocl_merge_partials",
                "ocl_route_partials_workspace_size", "ocl_route_partials",
                "ocl_join_build_workspace_size", "ocl_join_build", "ocl_join_probe_workspace_size", "ocl_join_probe",
@@ -165,6 +175,24 @@ class Context:
             _lib.ocl_ctx_destroy(self.handle)
             self.handle = None
 
+    def attach_nccl(self, unique_id, rank, nranks):
+        """ocl_ctx_attach_nccl: join an NCCL communicator (collective over the nranks ranks)."""
+        buf = ctypes.create_string_buffer(bytes(unique_id), 128)
+        _check(lib().ocl_ctx_attach_nccl(self.handle, buf, int(rank), int(nranks)))
+
+    @property
+    def nccl_rank(self):
+        r, n = ctypes.c_int32(), ctypes.c_int32()
+        _check(lib().ocl_ctx_nccl_rank(self.handle, ctypes.byref(r), ctypes.byref(n)))
+        return r.value, n.value
+
+
+def nccl_unique_id():
+    """ocl_nccl_unique_id: 128 bytes to hand to every rank (out of band)."""
+    buf = ctypes.create_string_buffer(128)
+    _check(lib().ocl_nccl_unique_id(buf))
+    return buf.raw
+
 
 _ctxs = {}
 
@@ -177,6 +205,12 @@ def launch_count():
 def last_kernel(ctx):
     """Name of the fused kernel instantiation the last fused call on ctx used."""
     return lib().ocl_ctx_last_kernel(ctx.handle).decode()
+
+
+def set_phase_events(ctx, phase, begin=None, end=None):
+    """Bracket phase 0 (fused kernel) or 1 (exchange + merge) of subsequent calls on ctx with events."""
+    _check(lib().ocl_ctx_set_phase_events(ctx.handle, int(phase), begin.cuda_event if begin is not None else None,
+                                          end.cuda_event if end is not None else None))
 
 
 def set_kernel_events(ctx, begin=None, end=None):
@@ -447,12 +481,16 @@ class SgaCall:
     across launches (the benchmark times only ``launch``)."""
 
     def __init__(self, preds, keys, vals, aggs, expected_groups=1024, out_capacity=None, order_by_key=False,
-                 bitmap=False, tier=0, host=False, chunk_rows=1 << 24, device=None, key_sorted=False):
+                 bitmap=False, tier=0, host=False, chunk_rows=1 << 24, device=None, key_sorted=False,
+                 distributed=0, ctx=None, sync=False):
+        """distributed: 0 local, 1 allgather (replicated result), 2 all-to-all (this rank's hash partition),
+        over ctx's NCCL communicator (ctx = a Context after attach_nccl, see distributed.attach_nccl).
+        sync: size the workspace for ocl_select_group_aggregate_sync (launch_sync, the restart ladder)."""
         cols = [p[0] for p in preds] + list(keys) + list(vals)
         self.host = host
         self.device = torch.device(device) if device is not None else (
             cols[0].device if cols and not host else torch.device("cuda", torch.cuda.current_device()))
-        self.ctx = context(self.device)
+        self.ctx = ctx if ctx is not None else context(self.device)
         n = cols[0].numel() if cols else 0
         self.n = n
         self.aggs_spec = aggs
@@ -485,10 +523,14 @@ class SgaCall:
         a.dev_status = self.status.data_ptr()
         a.order_by_key, a.tier = int(bool(order_by_key)), int(tier)
         a.key_sorted = int(bool(key_sorted))
+        a.distributed = int(distributed)
         self.args = a
         self.chunk_rows = int(chunk_rows)
         sz = ctypes.c_size_t()
-        if host:
+        if sync and not host:
+            _check(lib().ocl_select_group_aggregate_sync_workspace_size(self.ctx.handle, ctypes.byref(a),
+                                                                        ctypes.byref(sz)))
+        elif host:
             _check(lib().ocl_select_group_aggregate_host_workspace_size(self.ctx.handle, ctypes.byref(a),
                                                                         self.chunk_rows, ctypes.byref(sz)))
         else:
@@ -503,6 +545,12 @@ class SgaCall:
         else:
             _check(lib().ocl_select_group_aggregate(self.ctx.handle, ctypes.byref(self.args), self.ws.data_ptr(),
                                                     self.ws_bytes, _stream(stream)))
+
+    def launch_sync(self, stream=None):
+        """ocl_select_group_aggregate_sync: blocking, restarts with a larger table on overflow.
+        Needs sync=True at construction (workspace for the restart ladder)."""
+        _check(lib().ocl_select_group_aggregate_sync(self.ctx.handle, ctypes.byref(self.args), self.ws.data_ptr(),
+                                                     self.ws_bytes, _stream(stream)))
 
     def capture(self, stream=None):
         """Record launch() once into a CUDA graph (torch.cuda.CUDAGraph) and return it: replay() re-runs the
@@ -538,21 +586,22 @@ def select_group_aggregate(preds, keys, vals, aggs, expected_groups=4, out_capac
     key_sorted=True: the packed key column is sorted -> sort-based grouping, output in key
     order; an unsorted key column raises OcelotError(OCL_ERR_INVALID_ARG).
     Returns (keys_out[G], [outputs[G]], bitmap or None)."""
-    eg = expected_groups
+    # The table restart runs in the library (ocl_select_group_aggregate_sync); only the OUTPUT
+    # buffers (caller memory, sized by out_capacity) are re-allocated here when G exceeds them.
+    cap = out_capacity
     for _ in range(max_retries):
-        call = SgaCall(preds, keys, vals, aggs, expected_groups=eg, out_capacity=out_capacity,
-                       order_by_key=order_by_key, bitmap=bitmap, tier=tier, key_sorted=key_sorted)
-        call.launch(stream)
+        call = SgaCall(preds, keys, vals, aggs, expected_groups=expected_groups, out_capacity=cap,
+                       order_by_key=order_by_key, bitmap=bitmap, tier=tier, key_sorted=key_sorted, sync=True)
         try:
+            call.launch_sync(stream)
             k, o = call.result()
             return k, o, call.bitmap
         except OcelotError as e:
             if e.status != OCL_ERR_CAPACITY:
                 raise
-            G = int(call.ngroups.item())
-            eg = max(4 * eg, 2 * G)              # table full -> G reads as the capacity: grow geometrically
-            if out_capacity is not None and out_capacity < G:
-                out_capacity = G
+            G = int(call.ngroups.item())             # > out_capacity: G (or a lower bound while the table was full)
+            cap = max(4 * call.out_capacity, 2 * G)
+            expected_groups = max(expected_groups, G)
     raise OcelotError(OCL_ERR_CAPACITY, "hash table still full after retries")
 
 
@@ -572,12 +621,21 @@ def partial_row_bytes(call):
     return sz.value
 
 
-def sga_partial(call, partial_capacity, stream=None):
-    """Local fused pass -> (partial rows uint8[cap, row_bytes], count int64[1]) on the device."""
+def sga_partial(call, partial_capacity, stream=None, status=None, out=None):
+    """Local fused pass -> (partial rows uint8[cap, row_bytes], count int64[1]) on the device.
+    status: an int32[1] device tensor for this step's overflow flag (default: call.status); out: a
+    preallocated (rows, count) pair to write into."""
     rb = partial_row_bytes(call)
-    part = torch.zeros((max(partial_capacity, 1), rb), dtype=torch.uint8, device=call.device)
-    cnt = torch.zeros(1, dtype=torch.int64, device=call.device)
-    _check(lib().ocl_sga_partial(call.ctx.handle, ctypes.byref(call.args), part.data_ptr(), partial_capacity,
+    if out is None:
+        part = torch.empty((max(partial_capacity, 1), rb), dtype=torch.uint8, device=call.device)
+        cnt = torch.empty(1, dtype=torch.int64, device=call.device)
+    else:
+        part, cnt = out
+    args = call.args
+    if status is not None:
+        args = SgaArgs.from_buffer_copy(call.args)
+        args.dev_status = status.data_ptr()
+    _check(lib().ocl_sga_partial(call.ctx.handle, ctypes.byref(args), part.data_ptr(), partial_capacity,
                                  cnt.data_ptr(), call.ws.data_ptr(), call.ws_bytes, _stream(stream)))
     return part, cnt
 
@@ -607,4 +665,4 @@ def route_partials(part, cnt, nparts, stream=None):
     return out, counts
 
 
-from .distributed import distributed_select_group_aggregate, shard_range  # noqa: E402,F401
+from .distributed import attach_nccl, distributed_select_group_aggregate, shard_range  # noqa: E402,F401

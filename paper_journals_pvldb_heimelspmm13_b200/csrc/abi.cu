@@ -10,6 +10,8 @@
 
 #include <algorithm>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "launch.cuh"
 
 
@@ -21,6 +23,9 @@ std::atomic<unsigned long long> g_launches{0};
 
 struct ocl_ctx {
   cudaEvent_t prof_begin = nullptr, prof_end = nullptr;   // optional: bracket the fused kernel
+  cudaEvent_t xchg_begin = nullptr, xchg_end = nullptr;   // optional: bracket exchange + merge (distributed)
+  void* comm = nullptr;     // ncclComm_t (ocl_ctx_attach_nccl)
+  int rank = 0, nranks = 1;
   int last_kernel = 0;                                     // 0 generic, >0 specialised signature id
   int device;
   int sms;
@@ -45,6 +50,12 @@ ocl_status fail(ocl_status s, const char* fmt, ...) {
 ocl_status cuda_fail(cudaError_t e, const char* what) {
   return fail(OCL_ERR_CUDA, "%s: %s", what, cudaGetErrorString(e));
 }
+
+// NVTX range for the enclosing scope (host-side phase markers; free without a profiler).
+struct NvtxRange {
+  explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+  ~NvtxRange() { nvtxRangePop(); }
+};
 
 #define OCL_CUDA(call, what)                       \
   do {                                             \
@@ -511,6 +522,192 @@ ocl_status run_sortpath(ocl_ctx* ctx, const ocl_sga_args* args, const Planned& P
   return OCL_OK;
 }
 
+// Local fused pass that emits partial rows (ocl_sga_partial; the local step of a distributed
+// call): count -> *count_out, rows -> partial_out (capacity cap); overflow -> args->dev_status.
+ocl_status local_partial(ocl_ctx* ctx, const ocl_sga_args* args, Planned& P, void* ws, size_t ws_bytes,
+                         cudaStream_t st, uint8_t* partial_out, int64_t cap, int64_t* count_out) {
+  if (P.sorted || P.sortgrp) return run_sortpath(ctx, args, P, ws, ws_bytes, st, partial_out, cap, count_out);
+  void* ews = nullptr;
+  EmitArgs ea;
+  memset(&ea, 0, sizeof(ea));
+  ea.kind = EMIT_PARTIAL;
+  ea.out_capacity = cap;
+  ea.partial_out = partial_out;
+  ea.status = args->dev_status;
+  bool emitted = false;
+  ocl_status s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews, &ea, count_out, cap, &emitted);
+  if (s) return s;
+  if (!emitted)
+    OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, count_out, cap, args->dev_status, false, ews,
+                         ctx->grid, st), "partial export");
+  return OCL_OK;
+}
+
+// ---------------------------------------------------------------- distributed calls (distributed.cu)
+// Workspace of a distributed call: [local step (size `local`)] then the exchange region:
+// header (W int64: row count(s) + the local partial's status word), all ranks' headers,
+// the local partial table, the all-to-all send blocks, the receive buffer (P parts), the
+// per-part row counts, the merge table and its emit scratch.
+struct DistLayout {
+  int mode, P, W;
+  int64_t part_cap;   // partial rows of this rank (= out_capacity)
+  int64_t block;      // rows per destination block (all-to-all)
+  int64_t recv_cap;   // rows per received part
+  uint64_t mcap;      // merge table slots
+  size_t rb;          // partial row bytes
+  size_t off_hdr, off_hdr_all, off_pcount, off_part, off_send, off_recv, off_counts, off_mtable, off_mews, total;
+};
+
+ocl_status dist_layout(ocl_ctx* ctx, const ocl_sga_args* a, const Planned& P, size_t local, DistLayout* L) {
+  if (!ctx->comm)
+    return fail(OCL_ERR_INVALID_ARG, "distributed = %d but ctx has no NCCL communicator (ocl_ctx_attach_nccl)",
+                a->distributed);
+  if (a->distributed != 1 && a->distributed != 2)
+    return fail(OCL_ERR_INVALID_ARG, "distributed = %d (0 local, 1 allgather, 2 all-to-all)", a->distributed);
+  memset(L, 0, sizeof(*L));
+  L->mode = a->distributed;
+  L->P = ctx->nranks;
+  L->W = L->mode == 1 ? 2 : L->P + 1;
+  L->rb = (size_t)P.plan.stride;
+  L->part_cap = std::max<int64_t>(a->out_capacity, 1);
+  L->block = L->mode == 1 ? L->part_cap : (L->part_cap * 5 / 4 + L->P - 1) / L->P + 64;
+  L->recv_cap = L->block;
+  const int64_t gmax = std::min<int64_t>((int64_t)L->P * L->recv_cap, std::max<int64_t>(a->out_capacity, 1));
+  L->mcap = next_pow2((uint64_t)std::max<int64_t>(2 * gmax, 16));
+  if (a->order_by_key && !sorted_emit_supported(L->mcap))
+    return fail(OCL_ERR_UNSUPPORTED, "order_by_key on a distributed call needs out_capacity <= 1023 (merge table of %llu slots)",
+                (unsigned long long)L->mcap);
+  size_t o = align_up(local, 256);
+  L->off_hdr = o;
+  o += align_up((size_t)L->W * 8, 256);
+  L->off_hdr_all = o;
+  o += align_up((size_t)L->P * L->W * 8, 256);
+  L->off_pcount = o;
+  o += 256;
+  L->off_part = o;
+  o += align_up((size_t)L->part_cap * L->rb, 256);
+  L->off_send = o;
+  if (L->mode == 2) o += align_up((size_t)L->P * L->block * L->rb, 256);
+  L->off_recv = o;
+  o += align_up((size_t)L->P * L->recv_cap * L->rb, 256);
+  L->off_counts = o;
+  o += align_up((size_t)L->P * 8, 256);
+  L->off_mtable = o;
+  o += align_up((L->mcap + 1) * L->rb, 256);
+  L->off_mews = o;
+  o += align_up(emit_ws_bytes(ctx->grid), 256);
+  L->total = o;
+  return OCL_OK;
+}
+
+// Exchange this rank's partial table (already in the region, its row count in the header
+// (allgather) or at off_pcount (all-to-all)) and merge the received parts into fin's outputs.
+ocl_status dist_exchange_merge(ocl_ctx* ctx, const ocl_sga_args* a, const DistLayout& L, uint8_t* ws,
+                               const FinPlan& fin, int64_t* ngroups_out, int32_t* status, cudaStream_t st) {
+  int64_t* hdr = (int64_t*)(ws + L.off_hdr);
+  int64_t* hdr_all = (int64_t*)(ws + L.off_hdr_all);
+  uint8_t* part = ws + L.off_part;
+  uint8_t* recv = ws + L.off_recv;
+  int64_t* counts = (int64_t*)(ws + L.off_counts);
+  uint8_t* mtable = ws + L.off_mtable;
+  char err[256];
+  if (ctx->xchg_begin) OCL_CUDA(cudaEventRecord(ctx->xchg_begin, st), "phase event");
+  if (L.mode == 1) {
+    NvtxRange nv("ocl:allgather");
+    if (nccl_allgather2(hdr, hdr_all, (size_t)L.W * 8, part, recv, (size_t)L.part_cap * L.rb, ctx->comm, st, err,
+                        sizeof(err)))
+      return fail(OCL_ERR_NCCL, "%s", err);
+  } else {
+    NvtxRange nv("ocl:alltoall");
+    uint8_t* send = ws + L.off_send;
+    OCL_CUDA(launch_route_blocks(part, (const int64_t*)(ws + L.off_pcount), L.part_cap, (int32_t)L.rb, L.P, L.block,
+                                 send, hdr, ctx->sms, st), "route partial rows");
+    if (nccl_alltoall_blocks(hdr, hdr_all, (size_t)L.W * 8, send, recv, (size_t)L.block * L.rb, L.P, ctx->comm, st,
+                             err, sizeof(err)))
+      return fail(OCL_ERR_NCCL, "%s", err);
+  }
+  NvtxRange nv("ocl:merge");
+  const int64_t hcap = L.mode == 1 ? L.part_cap : L.block;
+  OCL_CUDA(launch_dist_headers(hdr_all, L.P, L.W, L.mode == 1 ? 0 : ctx->rank, hcap, counts, status, 0, nullptr, st),
+           "exchange headers");
+  OCL_CUDA(cudaMemsetAsync(mtable, 0, align_up((L.mcap + 1) * L.rb, 256), st), "merge table init");
+  OCL_CUDA(launch_merge_partials(recv, L.P, L.recv_cap, counts, fin, mtable, L.mcap - 1, status, ctx->grid, st),
+           "merge");
+  EmitArgs ea;
+  memset(&ea, 0, sizeof(ea));
+  ea.kind = EMIT_FINAL;
+  ea.fin = fin;
+  OCL_CUDA(launch_emit(mtable, L.mcap, (int32_t)L.rb, ea, ngroups_out, a->out_capacity, status, a->order_by_key != 0,
+                       ws + L.off_mews, ctx->grid, st), "merge finalize");
+  OCL_CUDA(launch_dist_headers(hdr_all, L.P, L.W, 0, hcap, nullptr, nullptr, 1, ngroups_out, st), "overflow report");
+  if (ctx->xchg_end) OCL_CUDA(cudaEventRecord(ctx->xchg_end, st), "phase event");
+  return OCL_OK;
+}
+
+// Local step of a distributed device call: the caller's plan with its own status word (the
+// header's, so a local overflow reaches every rank) and no ORDER BY (partial rows).
+ocl_status dist_local_plan(ocl_ctx* ctx, const ocl_sga_args* args, ocl_sga_args* la, Planned* PL, size_t* local) {
+  *la = *args;
+  la->distributed = 0;
+  la->order_by_key = 0;
+  la->dev_status = nullptr;
+  ocl_status s = plan_sga(la, PL, false);
+  if (s) return s;
+  *local = sga_ws_bytes(ctx, *PL);
+  return OCL_OK;
+}
+
+ocl_status dist_ws_bytes(ocl_ctx* ctx, const ocl_sga_args* args, const Planned& P, size_t* bytes) {
+  ocl_sga_args la;
+  Planned PL;
+  size_t local = 0;
+  ocl_status s = dist_local_plan(ctx, args, &la, &PL, &local);
+  if (s) return s;
+  DistLayout L;
+  if ((s = dist_layout(ctx, args, P, local, &L))) return s;
+  *bytes = L.total;
+  return OCL_OK;
+}
+
+ocl_status run_distributed(ocl_ctx* ctx, const ocl_sga_args* args, const Planned& P, void* ws, size_t ws_bytes,
+                           cudaStream_t st) {
+  ocl_sga_args la;
+  Planned PL;
+  size_t local = 0;
+  ocl_status s = dist_local_plan(ctx, args, &la, &PL, &local);
+  if (s) return s;
+  DistLayout L;
+  if ((s = dist_layout(ctx, args, P, local, &L))) return s;
+  if (!ws || ws_bytes < L.total) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, L.total);
+  uint8_t* w = (uint8_t*)ws;
+  int64_t* hdr = (int64_t*)(w + L.off_hdr);
+  la.dev_status = (int32_t*)&hdr[L.W - 1];
+  if ((s = plan_sga(&la, &PL, false))) return s;
+  OCL_CUDA(cudaMemsetAsync(hdr, 0, (size_t)L.W * 8, st), "header init");
+  if (args->dev_status) OCL_CUDA(cudaMemsetAsync(args->dev_status, 0, 4, st), "status init");
+  {
+    NvtxRange nv("ocl:select+aggregate (local shard)");
+    if ((s = local_partial(ctx, &la, PL, ws, local, st, w + L.off_part, L.part_cap,
+                           L.mode == 1 ? hdr : (int64_t*)(w + L.off_pcount))))
+      return s;
+  }
+  return dist_exchange_merge(ctx, args, L, w, P.fin, args->ngroups_out, args->dev_status, st);
+}
+
+// Restart ladder of ocl_select_group_aggregate_sync: expected_groups x 4 per step, capped at
+// max(out_capacity, expected_groups).  Its workspace is the largest over the ladder.
+int sync_ladder(const ocl_sga_args* a, int64_t* egs, int maxn) {
+  int64_t eg = std::max<int64_t>(a->expected_groups, 1);
+  const int64_t top = std::max<int64_t>(a->out_capacity, eg);
+  int n = 0;
+  egs[n++] = eg;
+  while (eg < top && n < maxn) {
+    eg = std::min<int64_t>(eg * 4, top);
+    egs[n++] = eg;
+  }
+  return n;
+}
+
 }  // namespace
 
 // ======================================================================== ABI
@@ -529,6 +726,45 @@ ocl_status ocl_ctx_set_kernel_events(ocl_ctx* ctx, void* begin_event, void* end_
   return OCL_OK;
 }
 
+ocl_status ocl_ctx_set_phase_events(ocl_ctx* ctx, int32_t phase, void* begin_event, void* end_event) {
+  if (!ctx) return fail(OCL_ERR_INVALID_ARG, "NULL ctx");
+  if (phase == 0) return ocl_ctx_set_kernel_events(ctx, begin_event, end_event);
+  if (phase != 1) return fail(OCL_ERR_INVALID_ARG, "phase %d (0 fused kernel, 1 exchange + merge)", phase);
+  ctx->xchg_begin = (cudaEvent_t)begin_event;
+  ctx->xchg_end = (cudaEvent_t)end_event;
+  return OCL_OK;
+}
+
+ocl_status ocl_nccl_unique_id(void* id_out) {
+  if (!id_out) return fail(OCL_ERR_INVALID_ARG, "NULL id_out");
+  char err[256];
+  if (nccl_unique_id(id_out, err, sizeof(err))) return fail(OCL_ERR_NCCL, "%s", err);
+  return OCL_OK;
+}
+
+ocl_status ocl_ctx_attach_nccl(ocl_ctx* ctx, const void* nccl_unique_id, int32_t rank, int32_t nranks) {
+  if (!ctx || !nccl_unique_id) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/unique id");
+  if (nranks < 1 || rank < 0 || rank >= nranks || nranks > 1024)
+    return fail(OCL_ERR_INVALID_ARG, "rank %d of %d", rank, nranks);
+  NvtxRange nv("ocl:nccl_init");
+  OCL_CUDA(cudaSetDevice(ctx->device), "cudaSetDevice");
+  char err[256];
+  void* comm = nullptr;
+  if (nccl_comm_init(&comm, nccl_unique_id, rank, nranks, err, sizeof(err))) return fail(OCL_ERR_NCCL, "%s", err);
+  nccl_comm_destroy(ctx->comm);
+  ctx->comm = comm;
+  ctx->rank = rank;
+  ctx->nranks = nranks;
+  return OCL_OK;
+}
+
+ocl_status ocl_ctx_nccl_rank(ocl_ctx* ctx, int32_t* rank, int32_t* nranks) {
+  if (!ctx || !rank || !nranks) return fail(OCL_ERR_INVALID_ARG, "NULL argument");
+  *rank = ctx->rank;
+  *nranks = ctx->nranks;
+  return OCL_OK;
+}
+
 const char* ocl_last_error(void) { return g_err; }
 
 const char* ocl_status_string(ocl_status s) {
@@ -539,6 +775,7 @@ const char* ocl_status_string(ocl_status s) {
     case OCL_ERR_CAPACITY: return "OCL_ERR_CAPACITY";
     case OCL_ERR_OUT_OF_MEMORY: return "OCL_ERR_OUT_OF_MEMORY";
     case OCL_ERR_CUDA: return "OCL_ERR_CUDA";
+    case OCL_ERR_NCCL: return "OCL_ERR_NCCL";
   }
   return "OCL_ERR_UNKNOWN";
 }
@@ -571,6 +808,7 @@ ocl_status ocl_ctx_create(int device, ocl_ctx** out) {
 
 ocl_status ocl_ctx_destroy(ocl_ctx* ctx) {
   if (!ctx) return OCL_OK;
+  nccl_comm_destroy(ctx->comm);
   cudaStreamDestroy(ctx->copy_stream);
   cudaStreamDestroy(ctx->comp_stream);
   for (int i = 0; i < 2; ++i) {
@@ -876,6 +1114,7 @@ ocl_status ocl_select_group_aggregate_workspace_size(ocl_ctx* ctx, const ocl_sga
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
+  if (args->distributed) return dist_ws_bytes(ctx, args, P, bytes);
   *bytes = sga_ws_bytes(ctx, P);
   return OCL_OK;
 }
@@ -886,6 +1125,8 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
   ocl_status s = plan_sga(args, &P);
   if (s) return s;
   cudaStream_t st = (cudaStream_t)stream;
+  if (args->distributed) return run_distributed(ctx, args, P, ws, ws_bytes, st);
+  NvtxRange nv("ocl:select+group+aggregate");
   if (P.sorted || P.sortgrp) return run_sortpath(ctx, args, P, ws, ws_bytes, st, nullptr, args->out_capacity,
                                                  args->ngroups_out);
   void* ews = nullptr;
@@ -901,6 +1142,57 @@ ocl_status ocl_select_group_aggregate(ocl_ctx* ctx, const ocl_sga_args* args, vo
     OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, args->ngroups_out, args->out_capacity,
                          args->dev_status, args->order_by_key != 0, ews, ctx->grid, st), "finalize");
   return OCL_OK;
+}
+
+ocl_status ocl_select_group_aggregate_sync_workspace_size(ocl_ctx* ctx, const ocl_sga_args* args, size_t* bytes) {
+  if (!ctx || !bytes || !args) return fail(OCL_ERR_INVALID_ARG, "NULL ctx/args/bytes");
+  int64_t egs[40];
+  const int n = sync_ladder(args, egs, 40);
+  ocl_sga_args a = *args;
+  size_t best = 0;
+  for (int i = 0; i < n; ++i) {
+    a.expected_groups = egs[i];
+    size_t b = 0;
+    ocl_status s = ocl_select_group_aggregate_workspace_size(ctx, &a, &b);
+    if (s) return s;
+    best = std::max(best, b);
+  }
+  *bytes = align_up(best, 256) + (args->dev_status ? 0 : 256);
+  return OCL_OK;
+}
+
+ocl_status ocl_select_group_aggregate_sync(ocl_ctx* ctx, const ocl_sga_args* args, void* ws, size_t ws_bytes,
+                                           void* stream) {
+  size_t need = 0;
+  ocl_status s = ocl_select_group_aggregate_sync_workspace_size(ctx, args, &need);
+  if (s) return s;
+  if (!ws || ws_bytes < need) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
+  cudaStream_t st = (cudaStream_t)stream;
+  ocl_sga_args a = *args;
+  if (!a.dev_status) a.dev_status = (int32_t*)((uint8_t*)ws + need - 256);
+  int64_t egs[40];
+  const int n = sync_ladder(args, egs, 40);
+  for (int i = 0; i < n;) {
+    a.expected_groups = egs[i];
+    if ((s = ocl_select_group_aggregate(ctx, &a, ws, ws_bytes, stream))) return s;
+    int32_t hs = 0;
+    int64_t G = 0;
+    OCL_CUDA(cudaMemcpyAsync(&hs, a.dev_status, 4, cudaMemcpyDeviceToHost, st), "status readback");
+    OCL_CUDA(cudaMemcpyAsync(&G, a.ngroups_out, 8, cudaMemcpyDeviceToHost, st), "group count readback");
+    OCL_CUDA(cudaStreamSynchronize(st), "sync");
+    if (hs == OCL_OK) return OCL_OK;
+    if (hs != OCL_ERR_CAPACITY) return fail((ocl_status)hs, "device status %d", hs);
+    if (G > a.out_capacity)
+      return fail(OCL_ERR_CAPACITY, "%lld groups > out_capacity %lld", (long long)G, (long long)a.out_capacity);
+    // the table overflowed: restart at the ladder step covering max(4 x, 2 G)
+    const int64_t want = std::max<int64_t>(4 * egs[i], 2 * G);
+    int j = i + 1;
+    while (j < n - 1 && egs[j] < want) ++j;
+    if (j >= n) return fail(OCL_ERR_CAPACITY, "hash table full at expected_groups=%lld (out_capacity %lld)",
+                            (long long)egs[i], (long long)a.out_capacity);
+    i = j;
+  }
+  return fail(OCL_ERR_CAPACITY, "hash table full");
 }
 
 // ---------------------------------------------------------------- a10 multi-GPU pieces
@@ -920,22 +1212,10 @@ ocl_status ocl_sga_partial(ocl_ctx* ctx, const ocl_sga_args* args, void* partial
   Planned P;
   ocl_status s = plan_sga(args, &P, false);
   if (s) return s;
-  cudaStream_t st = (cudaStream_t)stream;
-  if (P.sorted || P.sortgrp)
-    return run_sortpath(ctx, args, P, ws, ws_bytes, st, (uint8_t*)partial_out, partial_capacity, npartial_out);
-  void* ews = nullptr;
-  EmitArgs ea;
-  memset(&ea, 0, sizeof(ea));
-  ea.kind = EMIT_PARTIAL;
-  ea.out_capacity = partial_capacity;
-  ea.partial_out = (uint8_t*)partial_out;
-  ea.status = args->dev_status;
-  bool emitted = false;
-  if ((s = run_fused(ctx, args, P, ws, ws_bytes, st, &ews, &ea, npartial_out, partial_capacity, &emitted))) return s;
-  if (!emitted)
-    OCL_CUDA(launch_emit(P.plan.table, P.cap, P.plan.stride, ea, npartial_out, partial_capacity, args->dev_status,
-                         false, ews, ctx->grid, st), "partial export");
-  return OCL_OK;
+  if (args->distributed) return fail(OCL_ERR_INVALID_ARG, "ocl_sga_partial is the local step: distributed must be 0");
+  NvtxRange nv("ocl:partial");
+  return local_partial(ctx, args, P, ws, ws_bytes, (cudaStream_t)stream, (uint8_t*)partial_out, partial_capacity,
+                       npartial_out);
 }
 
 static uint64_t merge_cap(const ocl_sga_args* args, int32_t nparts, int64_t part_capacity) {
@@ -1098,6 +1378,11 @@ ocl_status ocl_select_group_aggregate_host_workspace_size(ocl_ctx* ctx, const oc
   HostCols h;
   collect_host_cols(P, h, chunk_rows);
   *bytes = sga_ws_bytes(ctx, P) + 2 * h.slot_bytes + host_out_bytes(args, P);
+  if (args->distributed) {         // + the exchange region after the host-path workspace
+    DistLayout L;
+    if ((s = dist_layout(ctx, args, P, *bytes, &L))) return s;
+    *bytes = L.total;
+  }
   return OCL_OK;
 }
 
@@ -1141,9 +1426,19 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
   OCL_CUDA(cudaMemsetAsync(d_status, 0, 4, ks), "status init");
   OCL_CUDA(cudaEventRecord(ctx->ev_consumed[0], ks), "event");
   OCL_CUDA(cudaEventRecord(ctx->ev_consumed[1], ks), "event");
+  // distributed: the exchange region follows the host-path workspace; the chunks' table
+  // overflow goes to the header's status word so that every rank sees it
+  DistLayout L;
+  memset(&L, 0, sizeof(L));
+  int64_t* hdr = nullptr;
+  if (args->distributed) {
+    if ((s = dist_layout(ctx, args, P, (size_t)(cur - base), &L))) return s;
+    hdr = (int64_t*)(base + L.off_hdr);
+    OCL_CUDA(cudaMemsetAsync(hdr, 0, (size_t)L.W * 8, ks), "header init");
+  }
   Plan p = P.plan;
   p.table = table;
-  p.status = d_status;
+  p.status = hdr ? (int32_t*)&hdr[L.W - 1] : d_status;
   p.bitmap_out = nullptr;
   const int mode = fused_mode(args);
   const int64_t n = P.plan.n;
@@ -1177,12 +1472,25 @@ ocl_status ocl_select_group_aggregate_host(ocl_ctx* ctx, const ocl_sga_args* arg
     OCL_CUDA(launch_fused(q, mode, P.values_f64, ctx->sms, ks, &kind), "fused kernel (chunk)");
     OCL_CUDA(cudaEventRecord(ctx->ev_consumed[sl], ks), "event");
   }
-  EmitArgs ea;
-  memset(&ea, 0, sizeof(ea));
-  ea.kind = EMIT_FINAL;
-  ea.fin = fin;
-  OCL_CUDA(launch_emit(table, P.cap, p.stride, ea, d_ngroups, args->out_capacity, d_status, args->order_by_key != 0,
-                       ews, ctx->grid, ks), "finalize");
+  if (args->distributed) {
+    EmitArgs pa;
+    memset(&pa, 0, sizeof(pa));
+    pa.kind = EMIT_PARTIAL;
+    pa.out_capacity = L.part_cap;
+    pa.partial_out = base + L.off_part;
+    pa.status = p.status;
+    int64_t* pcount = L.mode == 1 ? hdr : (int64_t*)(base + L.off_pcount);
+    OCL_CUDA(launch_emit(table, P.cap, p.stride, pa, pcount, L.part_cap, p.status, false, ews, ctx->grid, ks),
+             "partial export");
+    if ((s = dist_exchange_merge(ctx, args, L, base, fin, d_ngroups, d_status, ks))) return s;
+  } else {
+    EmitArgs ea;
+    memset(&ea, 0, sizeof(ea));
+    ea.kind = EMIT_FINAL;
+    ea.fin = fin;
+    OCL_CUDA(launch_emit(table, P.cap, p.stride, ea, d_ngroups, args->out_capacity, d_status,
+                         args->order_by_key != 0, ews, ctx->grid, ks), "finalize");
+  }
   // results back to the host
   OCL_CUDA(cudaMemcpyAsync(args->ngroups_out, d_ngroups, 8, cudaMemcpyDeviceToHost, ks), "D2H ngroups");
   if (args->dev_status) OCL_CUDA(cudaMemcpyAsync(args->dev_status, d_status, 4, cudaMemcpyDeviceToHost, ks), "D2H status");

@@ -28,6 +28,21 @@ __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.release.cta.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
 
+// Release a stage that this warp has finished READING with generic-proxy loads (LDS) so
+// that the producer may overwrite it with async-proxy (TMA) writes.  A plain
+// mbarrier.arrive is not enough on sm_100a: ptxas issues the SYNCS.ARRIVE without waiting
+// for the warp's outstanding LDS (empty wait mask in the SASS control bits), so the next
+// bulk copy can land before the loads have read the stage — rows of two chunks mixed
+// (seen as rare wrong group counts, most often with a 1-stage ring).  The cross-proxy
+// fence orders the warp's generic reads before the async-proxy writes that follow the
+// barrier (PTX: fence.proxy.async is required between generic and async proxy accesses
+// to the same shared memory); every lane fences its own loads, then lane 0 arrives.
+__device__ __forceinline__ void mbar_release_reads(uint64_t* bar, int lane) {
+  asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+  __syncwarp();
+  if (lane == 0) mbar_arrive(bar);
+}
+
 __device__ __forceinline__ bool mbar_try_wait(uint64_t* bar, uint32_t parity) {
   uint32_t ok;
   asm volatile(

@@ -382,12 +382,11 @@ __device__ __forceinline__ void spec_row_scalar(const SpecPlan& p, int64_t r, SR
 // Every thread of the CTA calls it (barriers); threads tid >= T (a producer warp) only
 // take part in the barriers.
 template <class S, int L, int T>
-__device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm, const uint64_t* dir, uint64_t* blk,
-                                           int tid) {
+__device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm, const uint64_t* dir, int tid) {
   using A = Acc<S>;
-  (void)blk;
   constexpr int Q = 4;                     // threads per (slot, field)
-  constexpr int PER = T / Q;               // records each of them sums
+  constexpr int PER = T / Q;               // records each of them sums (interleaved: j = sub + Q k,
+                                           // so the Q lanes of a group read Q different banks)
   constexpr int F = 1 + S::NV;             // COUNT + the value sums
   static_assert(T % (32 * Q) == 0 || 32 % Q == 0, "Q lanes of a group share a warp");
   __shared__ uint8_t* ent[L];
@@ -405,35 +404,34 @@ __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm,
     uint8_t* e = ent[s];
     if (e == nullptr) continue;
     const uint8_t* sb = sm + (size_t)s * A::slot_bytes(T);
-    const int j0 = sub * PER;
-    if (v < 0) {
-      const uint32_t* c = (const uint32_t*)sb + j0;
+        if (v < 0) {
+      const uint32_t* c = (const uint32_t*)sb + sub;
       unsigned long long cw = 0;
 #pragma unroll 8
-      for (int j = 0; j < PER; ++j) cw += c[j];
+      for (int j = 0; j < PER; ++j) cw += c[Q * j];
       for (int o = Q / 2; o > 0; o >>= 1) cw += __shfl_xor_sync(gmask, cw, o);
       if (sub == 0 && cw) atomicAdd((unsigned long long*)(e + 8), cw);
       continue;
     }
     const int off = p.g.vals[v].off_sum;
     if constexpr (S::F64) {
-      const double* d = (const double*)(sb + A::f_dbl(v, T)) + j0;
+      const double* d = (const double*)(sb + A::f_dbl(v, T)) + sub;
       double sum = 0.0;
 #pragma unroll 8
-      for (int j = 0; j < PER; ++j) sum += d[j];
+      for (int j = 0; j < PER; ++j) sum += d[Q * j];
       for (int o = Q / 2; o > 0; o >>= 1) sum += __shfl_xor_sync(gmask, sum, o);
       if (sub == 0 && off >= 0) atomicAdd((double*)(e + off), sum);
     } else {
       I128 x{0, 0};
       if (vx_kind(S::OP(v)) == VX_COL) {
-        const int64_t* d = (const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)) + j0;
+        const int64_t* d = (const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)) + sub;
 #pragma unroll 8
-        for (int j = 0; j < PER; ++j) x = i128_add(x, i128_from_i64(d[j]));
+        for (int j = 0; j < PER; ++j) x = i128_add(x, i128_from_i64(d[Q * j]));
       } else {
-        const uint64_t* lo = (const uint64_t*)(sb + A::f_wlo(A::wide_idx(v), T)) + j0;
-        const uint32_t* hi = (const uint32_t*)(sb + A::f_whi(A::wide_idx(v), T)) + j0;
+        const uint64_t* lo = (const uint64_t*)(sb + A::f_wlo(A::wide_idx(v), T)) + sub;
+        const uint32_t* hi = (const uint32_t*)(sb + A::f_whi(A::wide_idx(v), T)) + sub;
 #pragma unroll 8
-        for (int j = 0; j < PER; ++j) x = i128_add(x, I128{lo[j], (uint64_t)(int64_t)(int32_t)hi[j]});
+        for (int j = 0; j < PER; ++j) x = i128_add(x, I128{lo[Q * j], (uint64_t)(int64_t)(int32_t)hi[Q * j]});
       }
       for (int o = Q / 2; o > 0; o >>= 1) {
         I128 y;
@@ -495,14 +493,12 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
   extern __shared__ __align__(128) uint8_t sm[];
   uint8_t* stg = sm + bulk_acc_bytes<S>(L, T);
   __shared__ uint64_t dir[L];
-  __shared__ __align__(16) uint64_t blk[L * 32];
   __shared__ __align__(8) uint64_t full[NS], empty[NS];
   const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
   {
     uint4* z = (uint4*)sm;
     for (int i = tid; i < (int)(A::bytes(L, T) / 16); i += T + 32) z[i] = make_uint4(0, 0, 0, 0);
   }
-  for (int i = tid; i < L * 32; i += T + 32) blk[i] = 0;
   if (tid < L) dir[tid] = 0;
   if (tid == 0) {
     for (int s = 0; s < NS; ++s) {
@@ -558,8 +554,7 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
 #pragma unroll
         for (int i = 0; i < S::NC; ++i) lds2<8>(d + B::OFF_C + i * R * 8, j, cv[u][0][i], cv[u][1][i]);
       }
-      __syncwarp();
-      if (lane == 0) mbar_arrive(&empty[stage]);     // the stage's bytes are in registers now
+      mbar_release_reads(&empty[stage], lane);       // the stage's bytes are in registers now
       if (++stage == NS) {
         stage = 0;
         phase ^= 1;
@@ -593,7 +588,7 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
       }
     }
   }
-  priv_flush<S, L, T>(p, sm, dir, blk, tid);
+  priv_flush<S, L, T>(p, sm, dir, tid);
 }
 
 template <class S, int L>
@@ -602,13 +597,11 @@ __global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant
   constexpr int T = kPrivThreads;
   extern __shared__ __align__(16) uint8_t sm[];
   __shared__ uint64_t dir[L];
-  __shared__ __align__(16) uint64_t blk[L * 32];
   const int tid = threadIdx.x, lane = tid & 31;
   {
     uint4* z = (uint4*)sm;
     for (int i = tid; i < (int)(A::bytes(L, T) / 16); i += T) z[i] = make_uint4(0, 0, 0, 0);
   }
-  for (int i = tid; i < L * 32; i += T) blk[i] = 0;
   if (tid < L) dir[tid] = 0;
   __syncthreads();
   KeyT<S> rk[L];
@@ -660,7 +653,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant
       }
     }
   }
-  priv_flush<S, L, T>(p, sm, dir, blk, tid);
+  priv_flush<S, L, T>(p, sm, dir, tid);
 }
 
 // ------------------------------------------------------------------ signature table
@@ -740,11 +733,13 @@ static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t
     if (!a16(sp.col[i])) return false;
   auto fn = k_sga_bulk<S, L, T, R, NS>;
   const size_t smem = bulk_acc_bytes<S>(L, T) + (size_t)NS * BulkStage<S, R>::BYTES;
-  static int nb = -1;
-  if (nb < 0) {
-    if (cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem) != cudaSuccess) return false;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&nb, fn, T + 32, smem) != cudaSuccess || nb < 1) nb = 0;
-  }
+  static DevCache cache;
+  const int nb = cache.get([&]() -> int {
+    if (cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem) != cudaSuccess) return 0;
+    int b = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, fn, T + 32, smem) != cudaSuccess || b < 1) b = 0;
+    return b;
+  });
   if (nb < 1) return false;
   int64_t grid = (int64_t)sms * nb;
   const int64_t chunks = sp.g.n / R;
@@ -762,12 +757,8 @@ static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t
 // warps per SM; measured on B200 C4, profiles/r01_c4_bulk_configs.md), 3 for fp64 plans
 // (C2: 51.0 -> 48.9 us, two sweeps agree, profiles/r01_c2_bulk_configs.md).
 static int bulk_config() {
-  static int cfg = -2;
-  if (cfg == -2) {
-    const char* e = getenv("OCL_BULK");
-    cfg = e ? atoi(e) : -1;
-  }
-  return cfg;
+  const char* e = getenv("OCL_BULK");   // read per launch (tests switch it inside one process)
+  return e ? atoi(e) : -1;
 }
 
 template <class S>
@@ -798,12 +789,12 @@ bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err,
       return true;
     }
     const size_t smem = Acc<S>::bytes(kPrivSlots, kPrivThreads);
-    static bool attr = false;
-    if (!attr) {
+    static DevCache cache;
+    const int nb = cache.get([&]() -> int {
       cudaFuncSetAttribute(k_sga_priv<S, kPrivSlots>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-      attr = true;
-    }
-    int grid = sms * spec_blocks_per_sm<S>(smem);
+      return spec_blocks_per_sm<S>(smem);
+    });
+    int grid = sms * nb;
     int64_t need = (tiles + 7) / 8;
     if (need < grid) grid = (int)(need > 0 ? need : 1);
     count_launch();

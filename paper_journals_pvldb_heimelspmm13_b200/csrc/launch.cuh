@@ -10,6 +10,30 @@ namespace ocl {
 extern std::atomic<unsigned long long> g_launches;
 inline void count_launch(unsigned long long k = 1) { g_launches.fetch_add(k, std::memory_order_relaxed); }
 
+// Per-device cache of a kernel's launch setup (dynamic shared-memory attribute set,
+// resident CTAs per SM).  Attributes and occupancy belong to a device, not to the
+// process: one process may drive several GPUs.  Racing initialisations compute the
+// same value, so relaxed atomics suffice.
+constexpr int kMaxDevices = 64;
+struct DevCache {
+  std::atomic<int> v[kMaxDevices];
+  DevCache() {
+    for (auto& x : v) x.store(-1, std::memory_order_relaxed);
+  }
+  // value for the current device, computing it with f() on first use
+  template <class F>
+  int get(F f) {
+    int d = 0;
+    if (cudaGetDevice(&d) != cudaSuccess || d < 0 || d >= kMaxDevices) return f();
+    int x = v[d].load(std::memory_order_relaxed);
+    if (x < 0) {
+      x = f();
+      v[d].store(x, std::memory_order_relaxed);
+    }
+    return x;
+  }
+};
+
 struct SelParams {
   const void* col;
   int64_t n;
@@ -74,6 +98,21 @@ size_t route_ws_bytes(int32_t nparts);
 int route_max_parts();
 cudaError_t launch_route(const void* rows, const int64_t* nrows_dev, int64_t max_rows, int32_t row_bytes,
                          int32_t nparts, void* out, int64_t* part_counts, void* ws, int sms, cudaStream_t s);
+// Multi-GPU exchange over NCCL (distributed.cu; NCCL loaded at run time).  The int
+// functions return 0 on success, else 1 with a message in err.
+int nccl_unique_id(void* id128, char* err, size_t errlen);
+int nccl_comm_init(void** comm, const void* id128, int rank, int nranks, char* err, size_t errlen);
+void nccl_comm_destroy(void* comm);
+int nccl_allgather2(const void* a, void* a_all, size_t a_bytes, const void* b, void* b_all, size_t b_bytes,
+                    void* comm, cudaStream_t s, char* err, size_t errlen);
+int nccl_alltoall_blocks(const void* hdr, void* hdr_all, size_t hdr_bytes, const void* send, void* recv,
+                         size_t block_bytes, int nranks, void* comm, cudaStream_t s, char* err, size_t errlen);
+cudaError_t launch_dist_headers(const int64_t* hdr_all, int32_t nparts, int32_t hdr_words, int32_t col, int64_t cap,
+                                int64_t* counts_out, int32_t* status, int32_t report, int64_t* ngroups_out,
+                                cudaStream_t s);
+cudaError_t launch_route_blocks(const void* rows, const int64_t* nrows_dev, int64_t max_rows, int32_t row_bytes,
+                                int32_t nparts, int64_t block_rows, void* out, int64_t* counts, int sms,
+                                cudaStream_t s);
 // Equi hash join (join.cu).
 size_t join_build_ws_bytes(int64_t n_build);
 size_t join_probe_ws_bytes(int64_t max_rows);

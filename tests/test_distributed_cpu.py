@@ -60,7 +60,7 @@ def _worker(rank, world, port, n, q):
         rows[:G, 5] = outs[3]
         part = torch.from_numpy(rows.view(np.uint8).reshape(cap, 48).copy())
         cnt = torch.tensor([G], dtype=torch.int64)
-        allp, counts, cap_x = exchange_partials(part, cnt)
+        allp, counts, cap_x = exchange_partials(part, cnt, cap)
         assert allp.shape == (world, cap_x, 48)
         merged = {}
         for r in range(world):
@@ -104,6 +104,60 @@ def test_gloo_allgather_merge_equals_oracle():
         s = ((int(sums[i, 1]) & 0xFFFFFFFFFFFFFFFF) << 64) | (int(sums[i, 0]) & 0xFFFFFFFFFFFFFFFF)
         ref[k] = [int(outs[0][i]), s, int(outs[2][i]), int(outs[3][i])]
     assert merged == ref
+
+
+# ---------------------------------------------------------------- overflow agreement
+def _overflow_worker(rank, world, port, bad_rank, how, q):
+    """distributed_select_group_aggregate's host logic with the library steps stubbed (no GPU here): one
+    rank's partial overflows -> every rank raises OCL_ERR_CAPACITY before any exchange of truncated tables."""
+    os.environ["MASTER_ADDR"] = "127.0.0.1"
+    os.environ["MASTER_PORT"] = str(port)
+    dist.init_process_group("gloo", rank=rank, world_size=world)
+    try:
+        import paper_journals_pvldb_heimelspmm13_b200 as pkg
+        from paper_journals_pvldb_heimelspmm13_b200.distributed import distributed_select_group_aggregate
+        merged = []
+
+        def fake_partial(call, cap, stream=None, status=None, out=None):
+            cnt = torch.tensor([cap + 5 if (rank == bad_rank and how == "count") else 2], dtype=torch.int64)
+            if rank == bad_rank and how == "status":
+                status[0] = pkg.OCL_ERR_CAPACITY
+            return torch.zeros((cap, 48), dtype=torch.uint8), cnt
+
+        pkg.sga_partial = fake_partial
+        pkg.partial_row_bytes = lambda call: 48
+        pkg.merge_partials = lambda call, allp, counts, nparts, cap, stream=None: merged.append(counts.tolist())
+
+        class Call:
+            out_capacity = 16
+            device = torch.device("cpu")
+
+        try:
+            distributed_select_group_aggregate(Call(), mode="allgather")
+            q.put((rank, "ok", merged))
+        except pkg.OcelotError as e:
+            q.put((rank, "capacity" if e.status == pkg.OCL_ERR_CAPACITY else "other", merged))
+    finally:
+        dist.destroy_process_group()
+
+
+@pytest.mark.parametrize("bad_rank,how", [(-1, "none"), (1, "status"), (0, "count")])
+def test_gloo_overflow_agreement(bad_rank, how):
+    world = 2
+    ctx = mp.get_context("spawn")
+    q = ctx.Queue()
+    port = _free_port()
+    procs = [ctx.Process(target=_overflow_worker, args=(r, world, port, bad_rank, how, q)) for r in range(world)]
+    for p in procs:
+        p.start()
+    res = sorted(q.get(timeout=300) for _ in range(world))
+    for p in procs:
+        p.join(timeout=120)
+        assert p.exitcode == 0
+    if bad_rank < 0:
+        assert [r[1] for r in res] == ["ok", "ok"] and all(r[2] == [[2, 2]] for r in res)
+    else:
+        assert [r[1] for r in res] == ["capacity", "capacity"] and all(r[2] == [] for r in res)
 
 
 # ---------------------------------------------------------------- all-to-all (hash-routed) exchange, NEXT-2

@@ -186,10 +186,20 @@ def _lineitem(n, seed, f64=False, shuffled=False):
     return datagen.lineitem_host(n, seed, fields=fields, shuffled=shuffled)
 
 
-def _check_sga(preds, keys, vals, aggs, expected_groups=4, tier=0, order_by_key=False, bitmap=False, rtol=1e-9):
+def ran_kernel():
+    """Name of the fused kernel the last fused call on cuda:0 launched (ocl_ctx_last_kernel)."""
+    return ocl.last_kernel(ocl.context(DEV))
+
+
+def _check_sga(preds, keys, vals, aggs, expected_groups=4, tier=0, order_by_key=False, bitmap=False, rtol=1e-9,
+               kernel=None):
+    """Fused call vs oracle.sga; kernel (substring) asserts which fused kernel ran, so a dispatch change
+    cannot silently move a test away from the kernel it is meant to cover."""
     k, outs, bm = ocl.select_group_aggregate([(dev(c), s) for c, s in preds], [dev(c) for c in keys],
                                              [dev(c) for c in vals], aggs, expected_groups=expected_groups,
                                              tier=tier, order_by_key=order_by_key, bitmap=bitmap)
+    if kernel is not None:
+        assert kernel in ran_kernel(), (kernel, ran_kernel())
     rk, routs = oracle.sga(preds, keys, vals, aggs, order_by_key=order_by_key)
     dts = [c.dtype for c in vals]
     assert_results_equal(by_key(k.cpu().numpy(), [o.cpu().numpy() for o in outs], aggs, dts),
@@ -223,14 +233,15 @@ def test_fused_q1_int(tier, n):
     li = _lineitem(n, datagen.BASE_SEED + 1)
     p, k, v, a = _q1(li)
     _check_sga(p, k, v, a + [{"op": "sum", "a": 2}, {"op": "min", "a": 0}, {"op": "max", "a": 1}], tier=tier,
-               order_by_key=True, bitmap=True)
+               order_by_key=True, bitmap=True, kernel="k_sga<DynShape>" if tier == 1 else "k_sga_glb")
 
 
 @pytest.mark.parametrize("tier", [1, 2])
 def test_fused_q1_f64(tier):
     li = _lineitem(6000000 if tier == 1 else 300000, datagen.BASE_SEED + 2, f64=True)
     p, k, v, a = _q1(li, f64=True)
-    _check_sga(p, k, v, a + [{"op": "min", "a": 0}, {"op": "max", "a": 1}], tier=tier)
+    _check_sga(p, k, v, a + [{"op": "min", "a": 0}, {"op": "max", "a": 1}], tier=tier,
+               kernel="k_sga<DynShape>" if tier == 1 else "k_sga_glb")
 
 
 def test_fused_worked_example():
@@ -238,7 +249,7 @@ def test_fused_worked_example():
     c = golden_columns(load_golden())
     li = dict(c)
     p, k, v, a = _q1(li)
-    _check_sga(p, k, v, a, order_by_key=True, bitmap=True, rtol=0.0)
+    _check_sga(p, k, v, a, order_by_key=True, bitmap=True, rtol=0.0, kernel="k_sga_priv<Sig Q1 int64>")
 
 
 @pytest.mark.parametrize("G", [3, 5, 64, 5000, 200000])
@@ -299,11 +310,24 @@ def test_fused_edge_cases():
 
 @pytest.mark.parametrize("offset", [1, 3])
 def test_fused_unaligned_columns(offset):
+    """Device columns that start `offset` elements into their allocation (torch slices keep the offset, so
+    u8 / i32 / i64 columns are 1- / 4- / 8-byte but not 16-byte aligned): the scalar-load path."""
     n = 20000
     li = _lineitem(n + offset, 11)
-    li = {k: v[offset:] for k, v in li.items()}
     p, k, v, a = _q1(li)
-    _check_sga(p, k, v, a, tier=1, bitmap=True)
+    sl = lambda c: dev(c)[offset:]
+    assert sl(li["quantity"]).data_ptr() % 16 != 0
+    keys, outs, bm = ocl.select_group_aggregate([(sl(c), s) for c, s in p], [sl(c) for c in k], [sl(c) for c in v],
+                                                a, expected_groups=4, tier=1, order_by_key=True, bitmap=True)
+    assert "k_sga<DynShape>" in ran_kernel()                 # unaligned: no vector loads, no copy engine
+    p0 = [(c[offset:], s) for c, s in p]
+    k0, v0 = [c[offset:] for c in k], [c[offset:] for c in v]
+    rk, routs = oracle.sga(p0, k0, v0, a, order_by_key=True)
+    dts = [c.dtype for c in v0]
+    assert keys.cpu().numpy().tolist() == rk.tolist()
+    assert_results_equal(by_key(keys.cpu().numpy(), [o.cpu().numpy() for o in outs], a, dts),
+                         by_key(rk, routs, a, dts), a, dts)
+    assert np.array_equal(host_u32(bm), oracle.select(p0[0][0], p0[0][1]))
 
 
 def test_fused_c3_orderkey():
@@ -313,7 +337,8 @@ def test_fused_c3_orderkey():
         li = _lineitem(n, datagen.BASE_SEED + 3, shuffled=shuffled)
         aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
         for tier in (2, 5):
-            _check_sga([], [li["orderkey"]], [li["quantity"]], aggs, expected_groups=n // 4, tier=tier)
+            _check_sga([], [li["orderkey"]], [li["quantity"]], aggs, expected_groups=n // 4, tier=tier,
+                       kernel="k_sga_glb" if tier == 2 else "hash-partitioned")
 
 
 @pytest.mark.parametrize("n", [1, 1000, 70001, 1 << 20])
@@ -408,10 +433,10 @@ def test_fused_q1_unified_static_shape(monkeypatch):
     for n in (1000, 300001):
         li = _lineitem(n, datagen.BASE_SEED + 1)
         p, k, v, a = _q1(li)
-        _check_sga(p, k, v, a, tier=1, order_by_key=True, bitmap=True)
+        _check_sga(p, k, v, a, tier=1, order_by_key=True, bitmap=True, kernel="k_sga<StaticShape Q1 int64>")
         lf = _lineitem(n, datagen.BASE_SEED + 2, f64=True)
         p, k, v, a = _q1(lf, f64=True)
-        _check_sga(p, k, v, a, tier=1)
+        _check_sga(p, k, v, a, tier=1, kernel="k_sga<StaticShape Q1 fp64>")
 
 
 # ---------------------------------------------------------------- NEXT-2: hash-routed all-to-all merge (fake exchange)

@@ -1,0 +1,119 @@
+"""Parity of the exact kernels the benchmark times ("close the parity gaps").
+
+The C1 / C2 / C4 numbers come from the Q1-signature kernels of fused_spec.cu:
+``k_sga_bulk<Sig Q1 int64|fp64>`` (TMA bulk pipeline, default) and ``k_sga_priv<Sig ...>``
+(register loads; ``OCL_BULK=0`` or fewer rows than one pipeline stage).  Each test here runs
+the bench's own plan — the TPC-H Q1 aggregates with no MIN/MAX, so ``spec_match`` accepts it —
+compares every group with the oracle (SURVEY §8(c) rules: integers bit-exact, fp64 SUM / AVG
+within 1e-9 relative) and asserts the kernel that ran (``ocl_ctx_last_kernel``).
+
+Covered: every bulk pipeline configuration (``OCL_BULK`` 1-7, read per launch), ragged sizes
+around the stage size (n < R runs ``k_sga_priv``; n >= R the bulk kernel plus its scalar tail),
+the bitmap output of the bulk kernel, and rows outside the int32 fast path (the exact
+per-row int128 path inside the specialised kernels).  PAPER.md L562-568 (aggregation),
+L429-438 (bitmap).
+"""
+import numpy as np
+import pytest
+
+import datagen
+from tests._common import Q1_AGGS, Q1_AGGS_F64
+from tests.test_gpu_parity import _check_sga, _lineitem, ran_kernel
+
+pytestmark = pytest.mark.gpu
+
+# OCL_BULK -> rows per pipeline stage (fused_spec.cu launch_bulk_cfg); None = default (int 7, fp64 3)
+STAGE_ROWS = {None: 512, "0": 512, "1": 1024, "2": 512, "3": 512, "4": 512, "5": 256, "6": 256, "7": 512}
+
+
+def _q1_plan(li, f64):
+    if f64:
+        vals = [li["quantity_f"], li["extendedprice_f"], li["discount_f"], li["tax_f"]]
+        return [(li["shipdate"], {"hi": 10471})], [li["returnflag"], li["linestatus"]], vals, Q1_AGGS_F64
+    vals = [li["quantity"], li["extendedprice"], li["discount"], li["tax"]]
+    return [(li["shipdate"], {"hi": 10471})], [li["returnflag"], li["linestatus"]], vals, Q1_AGGS
+
+
+def _expect(f64, n, cfg):
+    sig = "fp64" if f64 else "int64"
+    if cfg == "0" or n < STAGE_ROWS[cfg]:
+        return f"k_sga_priv<Sig Q1 {sig}>"
+    return f"k_sga_bulk<Sig Q1 {sig}>"
+
+
+@pytest.mark.parametrize("n", [1, 100, 511, 512, 513, 1024 + 17, 4 * 512 * 148 + 333, 6_000_000])
+def test_c2_kernel_fp64_q1(n):
+    """C2's timed kernel: k_sga_bulk<SigQ1F> (default fp64 config <256, 512, 2>)."""
+    li = _lineitem(n, datagen.BASE_SEED + 2, f64=True)
+    p, k, v, a = _q1_plan(li, True)
+    _check_sga(p, k, v, a, order_by_key=True, kernel=_expect(True, n, None))
+
+
+@pytest.mark.parametrize("n", [1, 511, 512, 60_000, 1_000_003])
+def test_c1_c4_kernel_int_q1(n):
+    """C1 / C4's timed kernel: k_sga_bulk<SigQ1I> (default int config <128, 512, 2>)."""
+    li = _lineitem(n, datagen.BASE_SEED + 4)
+    p, k, v, a = _q1_plan(li, False)
+    _check_sga(p, k, v, a, order_by_key=True, kernel=_expect(False, n, None))
+
+
+@pytest.mark.parametrize("cfg", ["0", "1", "2", "3", "4", "5", "6", "7"])
+@pytest.mark.parametrize("f64", [False, True])
+def test_bulk_configs(monkeypatch, cfg, f64):
+    """Every pipeline configuration (OCL_BULK, read per launch) on a size with several chunks per CTA and a
+    ragged tail, plus one size below its stage.  Repeated: a stage-reuse race (the release of a stage before
+    the warp's shared-memory loads had read it, fixed with mbar_release_reads in bulk.cuh) showed up as a
+    few rows counted in the wrong group in some runs, most often with the 1-stage ring (cfg 4)."""
+    monkeypatch.setenv("OCL_BULK", cfg)
+    for n in (STAGE_ROWS[cfg] - 1, 3 * 148 * 2048 + 1000 + 17):   # cfg "0": k_sga_priv at both sizes
+        li = _lineitem(n, datagen.BASE_SEED + 2 + (n & 7), f64=f64)
+        p, k, v, a = _q1_plan(li, f64)
+        for _ in range(3 if n > 100_000 else 1):
+            _check_sga(p, k, v, a, order_by_key=True, kernel=_expect(f64, n, cfg))
+
+
+@pytest.mark.parametrize("cfg", [None, "0", "5"])
+@pytest.mark.parametrize("f64", [False, True])
+def test_spec_bitmap_out(monkeypatch, cfg, f64):
+    """bitmap_out emitted by the specialised kernels (bulk stages and the scalar tail), n >= R."""
+    if cfg is not None:
+        monkeypatch.setenv("OCL_BULK", cfg)
+    n = 1_000_003
+    li = _lineitem(n, datagen.BASE_SEED + 4, f64=f64)
+    p, k, v, a = _q1_plan(li, f64)
+    _check_sga(p, k, v, a, order_by_key=True, bitmap=True, kernel=_expect(f64, n, cfg))
+
+
+@pytest.mark.parametrize("cfg", [None, "0"])
+@pytest.mark.parametrize("n", [300, 700_001])
+def test_spec_values_beyond_int32(monkeypatch, cfg, n):
+    """Q1-signature plan whose rows leave the int32 fast path: quantities >= 2^31, prices whose products
+    exceed 2^62, negative values; those rows take the exact int128 per-row update of the HBM entry
+    (fused_spec.cu priv_slot -> update_entry_slow) while the rest stay in the private slots."""
+    if cfg is not None:
+        monkeypatch.setenv("OCL_BULK", cfg)
+    li = _lineitem(n, datagen.BASE_SEED + 4)
+    q, pr, d, t = (li[f].copy() for f in ("quantity", "extendedprice", "discount", "tax"))
+    q[::97] = 3 * (1 << 40) + 1                     # COL value beyond int32
+    pr[::101] = (1 << 35) + 7                       # product factor beyond int32
+    pr[5::211] = (1 << 62) - 3                      # products beyond int64 (int128 accumulation)
+    q[7::89] = -(1 << 33)                           # negative, beyond int32
+    d[3::53] = -(1 << 31)                           # S - b beyond int32
+    li.update(quantity=q, extendedprice=pr, discount=d, tax=t)
+    p, k, v, a = _q1_plan(li, False)
+    _check_sga(p, k, v, a, order_by_key=True, kernel=_expect(False, n, cfg))
+    assert "Sig Q1 int64" in ran_kernel()
+
+
+def test_spec_all_rows_filtered_and_one_group():
+    """Degenerate Q1-signature inputs: every row filtered out (G = 0) and a single group."""
+    n = 100_000
+    li = _lineitem(n, datagen.BASE_SEED + 4)
+    p, k, v, a = _q1_plan(li, False)
+    keys, _ = _check_sga([(li["shipdate"], {"hi": 0})], k, v, a, order_by_key=True,
+                         kernel="k_sga_bulk<Sig Q1 int64>")
+    assert len(keys) == 0
+    rf = np.full(n, ord("N"), np.uint8)
+    ls = np.full(n, ord("O"), np.uint8)
+    keys, _ = _check_sga(p, [rf, ls], v, a, order_by_key=True, kernel="k_sga_bulk<Sig Q1 int64>")
+    assert keys.cpu().numpy().tolist() == [(ord("N") << 8) | ord("O")]

@@ -65,6 +65,63 @@ def test_worked_example_f64_variant():
         assert abs(Fraction(v) - exact[k]) <= Fraction(1, 10**15) * exact[k]
 
 
+def test_worked_example_f64_all_branches():
+    """Every fp64 branch of the oracle's aggregation on the worked example (fp64 columns = decimals / 100,
+    S = 1.0): SUM of a column, SUM of a*(S-b) (MUL_1MINUS) and a*(S-b)*(S+c) (MUL_1MINUS_1PLUS), AVG = SUM /
+    COUNT.  Pinned to the hand-computed exact decimals of tests/golden (not to a re-typed formula): each
+    fp64 row value is within a few ulps of its exact decimal and every value is >= 0, so each output lies
+    within 1e-14 (relative) of the exact rational.  A dropped term, a sign error, a wrong operand index or
+    an AVG divided by the wrong count misses by far more than that."""
+    g = load_golden()
+    c = golden_columns(g)
+    names = ("quantity", "extendedprice", "discount", "tax")
+    vals = [c[k].astype(np.float64) / 100.0 for k in names]
+    aggs = [{"op": "sum", "a": 0}, {"op": "sum", "a": 1},
+            {"op": "sum", "expr": "mul_1minus", "a": 1, "b": 2, "scale": 0},
+            {"op": "sum", "expr": "mul_1minus_1plus", "a": 1, "b": 2, "c": 3, "scale": 0},
+            {"op": "avg", "a": 0}, {"op": "avg", "a": 1}, {"op": "avg", "a": 2},
+            {"op": "avg", "expr": "mul_1minus", "a": 1, "b": 2, "scale": 0}, {"op": "count"}]
+    keys, outs = oracle.sga([(c["shipdate"], Q1_PRED)], [c["returnflag"], c["linestatus"]], vals, aggs,
+                            order_by_key=True)
+    for i, k in enumerate(keys.tolist()):
+        row = next(r for r in g["groups"] if int(r[0], 16) == k)
+        cnt, sq, sp, sdp, sch, sd = (int(x) for x in row[1:7])
+        exact = [Fraction(sq, 100), Fraction(sp, 100), Fraction(sdp, 10**4), Fraction(sch, 10**6),
+                 Fraction(sq, 100 * cnt), Fraction(sp, 100 * cnt), Fraction(sd, 100 * cnt),
+                 Fraction(sdp, 10**4 * cnt)]
+        for j, e in enumerate(exact):
+            v = outs[j][i].item()
+            assert abs(Fraction(v) - e) <= Fraction(1, 10**14) * e, (hex(k), aggs[j], v, float(e))
+        assert outs[8][i] == cnt
+
+
+@pytest.mark.parametrize("scale", [0, 2])
+def test_f64_expressions_exact_decimal(scale):
+    """fp64 MUL_1MINUS / MUL_1MINUS_1PLUS sums and AVG on random decimals k/100 against exact rationals
+    (Python Fractions from the integers k), S = 10^scale, one and several groups."""
+    rng = np.random.default_rng(scale + 11)
+    n = 2000
+    ka, kb, kc = rng.integers(1, 10**6, n), rng.integers(0, 11, n), rng.integers(0, 9, n)
+    vals = [ka.astype(np.float64) / 100.0, kb.astype(np.float64) / 100.0, kc.astype(np.float64) / 100.0]
+    gk = (ka % 3).astype(np.int64)
+    aggs = [{"op": "sum", "expr": "mul_1minus", "a": 0, "b": 1, "scale": scale},
+            {"op": "sum", "expr": "mul_1minus_1plus", "a": 0, "b": 1, "c": 2, "scale": scale},
+            {"op": "avg", "expr": "mul_1minus", "a": 0, "b": 1, "scale": scale}, {"op": "avg", "a": 2}]
+    keys, outs = oracle.sga([], [gk], vals, aggs)
+    S = 10**scale
+    for i, k in enumerate(keys.tolist()):
+        sel = gk == k
+        a = [Fraction(int(x), 100) for x in ka[sel]]
+        b = [Fraction(int(x), 100) for x in kb[sel]]
+        cc = [Fraction(int(x), 100) for x in kc[sel]]
+        m1 = sum(x * (S - y) for x, y in zip(a, b))
+        m2 = sum(x * (S - y) * (S + z) for x, y, z in zip(a, b, cc))
+        exact = [m1, m2, m1 / len(a), sum(cc) / len(a)]
+        for j, e in enumerate(exact):
+            v = outs[j][i].item()
+            assert abs(Fraction(v) - e) <= Fraction(1, 10**13) * abs(e), (k, aggs[j], v, float(e))
+
+
 # ---------------------------------------------------------------- selection
 def _py_pred(x, spec):
     ok = True
