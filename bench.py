@@ -42,6 +42,10 @@ WORKLOADS = {
     "c4": dict(desc="C4: lineitem SF100, 600,000,000 rows; TPC-H-Q1-style fused select l_shipdate<=1998-09-02 "
                     "+ GROUP BY (l_returnflag, l_linestatus) = 4 groups; int64 decimal SUM/AVG (int128 exact) + COUNT",
                rows=600_000_000, seed=datagen.BASE_SEED + 4, kind="q1", f64=False, groups=4),
+    "c4mm": dict(desc="C4 + MIN/MAX: lineitem SF100, 600,000,000 rows; the Q1-style fused select + GROUP BY "
+                      "(l_returnflag, l_linestatus) with MIN(l_quantity) and MAX(l_extendedprice) added to the "
+                      "int64 decimal SUM/AVG/COUNT set",
+                 rows=600_000_000, seed=datagen.BASE_SEED + 4, kind="q1", f64=False, groups=4, minmax=True),
     "c2": dict(desc="C2: lineitem SF1, 6,000,000 rows; Q1-style 4-group aggregation on fp64 columns with AVG",
                rows=6_000_000, seed=datagen.BASE_SEED + 2, kind="q1", f64=True, groups=4),
     "c1": dict(desc="C1: lineitem SF0.01, 60,000 rows; Q1-style 4 groups, int64 decimals",
@@ -83,6 +87,8 @@ def workload_columns(wl, cols):
         if wl["f64"]:
             v = [x + "_f" for x in v]
         aggs = [dict(a, scale=0) if wl["f64"] and a.get("expr", "col") != "col" else a for a in Q1_AGGS]
+        if wl.get("minmax"):
+            aggs = aggs + [{"op": "min", "a": 0}, {"op": "max", "a": 1}]
         return ([(cols["shipdate"], Q1_PRED)], [cols["returnflag"], cols["linestatus"]], [cols[x] for x in v],
                 aggs, 4 + 1 + 1 + 4 * 8)
     aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]

@@ -121,6 +121,8 @@ def lib():
             "ocl_select_group_aggregate_host": [P, P, I64, P, SZ, P],
         }
         for name, args in sig.items():
+            if not hasattr(L, name):     # an older library build (A/B timing through OCL_LIB_PATH)
+                continue
             f = getattr(L, name)
             f.argtypes = args
             f.restype = ctypes.c_int

@@ -342,6 +342,7 @@ constexpr int64_t kPartMinRows = 1 << 20;
 int fused_mode(const ocl_sga_args* a) {
   if (a->tier == 2) return 2;
   if (a->tier == 3) return 1;
+  if (a->tier == 4) return 3;
   return 0;
 }
 
@@ -393,12 +394,13 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   P->table_bytes = align_up((P->cap + 1) * (size_t)p.stride, 256);
   p.status = a->dev_status;
   p.bitmap_out = a->bitmap_out;
+  p.expected = expected;
   p.smem_cap = plan_smem_cap(a, p);
   p.miss_agg = a->expected_groups > reg_tier_slots() ? 1 : 0;
   // High-cardinality tier: more groups than the shared-memory tiers hold, integer
   // column values, enough rows to amortise its five launches (tier 5 forces it).
   P->pbits = -1;
-  const bool many = a->tier == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows;
+  const bool many = a->tier == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows && !spec_takes(p);
   if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
   P->sorted = a->key_sorted != 0;
   P->sortgrp = a->tier == 6;

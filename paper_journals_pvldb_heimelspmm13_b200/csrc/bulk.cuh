@@ -60,6 +60,38 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t parity) {
   }
 }
 
+// try_wait with a suspend-time hint: the thread is suspended (not re-issued) until the
+// phase completes or `ns` nanoseconds pass.
+__device__ __forceinline__ bool mbar_try_wait_hint(uint64_t* bar, uint32_t parity, uint32_t ns) {
+  uint32_t ok;
+  asm volatile(
+      "{\n\t.reg .pred p;\n\t"
+      "mbarrier.try_wait.parity.acquire.cta.shared::cta.b64 p, [%1], %2, %3;\n\t"
+      "selp.u32 %0, 1, 0, p;\n\t}"
+      : "=r"(ok)
+      : "r"(smem_u32(bar)), "r"(parity), "r"(ns)
+      : "memory");
+  return ok != 0;
+}
+
+// Wait strategies (mode): 0 spin on try_wait; 1 back off with __nanosleep between tries
+// (a waiting warp stops taking issue slots from the warps that have work); 2 try_wait
+// with a suspend-time hint.
+__device__ __forceinline__ void mbar_wait_mode(uint64_t* bar, uint32_t parity, int mode) {
+  if (mode == 1) {
+    uint32_t ns = 32;
+    while (!mbar_try_wait(bar, parity)) {
+      __nanosleep(ns);
+      if (ns < 512) ns <<= 1;
+    }
+  } else if (mode == 2) {
+    while (!mbar_try_wait_hint(bar, parity, 100000)) {
+    }
+  } else {
+    mbar_wait(bar, parity);
+  }
+}
+
 // 1-D bulk copy of `bytes` (multiple of 16; both addresses 16-byte aligned) from global
 // to this CTA's shared memory, completing `bytes` transactions on `bar`.  Streamed
 // input is read once: evict-first keeps it from displacing reusable lines in L2.

@@ -167,6 +167,7 @@ struct Plan {
   const int32_t* gids;  // unfused aggregate: direct group ids (table indexed by gid)
   const uint32_t* oids; // unfused aggregate: row ids (null: identity)
   const int64_t* m_dev; // unfused aggregate: device row count (null: n)
+  int64_t expected;     // the caller's expected_groups (picks the accumulation tier of the bulk kernels)
 };
 
 struct OutAgg {

@@ -333,8 +333,9 @@ static cudaError_t launch_glb(const Plan& p, int sms, cudaStream_t s) {
 
 int reg_tier_slots() { return kRegSlots; }
 
-// mode 0: fused kernel (static shape if one matches); 1: fused kernel, DynShape only;
-// 2: HBM-only kernel.  values_f64: every value expression is fp64 (mixed plans use the
+// mode 0: plan-signature kernel if one matches, else the fused kernel (static shape if one
+// matches); 1: fused kernel, DynShape only; 2: HBM-only kernel; 3: the fused kernel (no
+// signature kernels: tier 4 forces its CTA shared-memory table).  values_f64: every value expression is fp64 (mixed plans use the
 // integer instantiation, whose exact slow path handles fp64 values).  *kind reports
 // the shape used (0 dynamic / HBM-only, 1.. static).
 cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cudaStream_t s, int* kind) {
@@ -344,14 +345,12 @@ cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cuda
     *kind = 20;
     return values_f64 ? launch_glb<true>(p, sms, s) : launch_glb<false>(p, sms, s);
   }
-  if (mode == 0 && p.vec_ok && !p.miss_agg && p.smem_cap == 0 && getenv("OCL_NO_SPEC") == nullptr) {
+  if (mode == 0 && p.vec_ok && getenv("OCL_NO_SPEC") == nullptr) {
     cudaError_t err = cudaSuccess;
-    if (launch_fused_spec(p, sms, s, &err, kind)) {
-      *kind += 10;                       // 11 / 12: Q1-signature kernel (int / fp64); 13 / 14: bulk pipeline
-      return err;
-    }
+    if (launch_fused_spec(p, sms, s, &err, kind)) return err;   // plan-signature kernels (fused_spec.cu)
+    *kind = 0;
   }
-  if (mode == 0 && p.vec_ok) {
+  if ((mode == 0 || mode == 3) && p.vec_ok) {
     if (shape_match<ShQ1I>(p)) {
       *kind = 1;
       return launch_k<ShQ1I, 5, false>(p, sms, s);
@@ -382,6 +381,12 @@ const char* fused_kernel_name(int kind) {
     case 12: return "k_sga_priv<Sig Q1 fp64>";
     case 13: return "k_sga_bulk<Sig Q1 int64> (TMA bulk pipeline)";
     case 14: return "k_sga_bulk<Sig Q1 fp64> (TMA bulk pipeline)";
+    case 15: return "k_sga_bulk<Sig Q1+MINMAX int64> (TMA bulk pipeline)";
+    case 16: return "k_sga_bulk<Sig Q1+MINMAX fp64> (TMA bulk pipeline)";
+    case 61: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
+    case 64: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; replicated tables>";
+    case 71: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
+    case 74: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; replicated tables>";
     case 20: return "k_sga_glb<DynShape>";
     case 30: return "k_part_count/scatter/agg<DynShape> (hash-partitioned)";
     case 31: return "k_part_count/scatter/agg<StaticShape key i64> (hash-partitioned)";

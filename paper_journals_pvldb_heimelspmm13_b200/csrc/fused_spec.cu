@@ -1,18 +1,34 @@
-// fused_spec.cu — the TPC-H Q1-signature fused kernel (few groups; SUM / COUNT /
-// AVG over a predicate column, two u8 key columns and int64 / fp64 decimals).
+// fused_spec.cu — plan-signature fused kernels: select -> group -> aggregate in one
+// pass over TMA-streamed columns, specialised at compile time for the plan shapes the
+// benchmark configurations use (TPC-H Q1, Q1 + MIN/MAX, and the GROUP BY key / COUNT,
+// SUM, MIN, MAX shape of C3 / C5).
 //
 // Same method, semantics and accumulation scheme as the unified kernel in fused.cu
-// (§4.1.1 selection, §4.1.6 grouping, §4.1.7 aggregation; private
-// per-thread accumulators in shared memory), specialised by hand for the
-// Q1 plan shape: accumulator arrays grouped by type ([type][slot][value][thread]),
-// narrow sums in 64 bits, products in 96 bits, compile-time layout and key packing.
-// Two kernels: k_sga_priv loads the columns into registers (vector LDG, two units in
-// flight per warp); k_sga_bulk (default) streams them into shared memory with TMA
-// bulk copies (cp.async.bulk + mbarrier ring, one producer warp) so the consumer
-// warps only compute.  On B200 C4 (600M rows) k_sga_bulk runs in ~3.45 ms
-// (~6.6 TB/s, ~101 % of the measured copy bandwidth); the generic StaticShape
-// instantiation of k_sga takes 5.1-5.5 ms.  launch_fused (fused.cu)
-// tries these kernels first for few-group plans; OCL_NO_SPEC=1 disables them.
+// (§4.1.1 selection, §4.1.6 grouping, §4.1.7 aggregation), specialised by hand:
+// compile-time column widths, key packing and accumulator layout.  The columns reach
+// shared memory through the copy engine (k_sga_bulk: cp.async.bulk + an mbarrier ring
+// fed by one producer warp) so the consumer warps only compute; k_sga_priv is the
+// register-load variant for inputs smaller than one pipeline stage.
+//
+// Accumulation tiers (§4.1.7: local accumulation, "multiple accumulators per
+// group, inversely proportional to the number of groups"), chosen by expected_groups:
+//  * private (<= 4 groups): every consumer thread owns one accumulator record per group slot
+//    in shared memory ([slot][field][thread]: lane t always hits the same banks); a row
+//    costs a register compare against the 4 slot keys and a non-atomic read-modify-write —
+//    the limit of the paper's accumulators ∝ 1/G.
+//  * replicated tables (<= 2048 groups, integer COL values): nrep copies of a shared-memory
+//    hash table per CTA (consumer warp w -> copy w % nrep; nrep = min(warps, 72 KB / table),
+//    so the copies multiply as G falls; stored field-major), native 32-bit shared atomics — count, biased 64-bit
+//    sums as a 32-bit add whose carry is taken from the returned value (exact, no periodic
+//    fold), order-encoded MIN / MAX — and a loop-free home-slot hit.
+// Rows outside the int32 fast path, the key ~0 and keys beyond the tier's capacity take
+// the exact per-row update of the HBM table.  At the end every CTA folds its records /
+// table into the HBM table (int128 sums).
+//
+// On B200, C4 (600M rows, Q1) runs in ~3.5 ms (~98-100 % of the measured copy bandwidth).
+// launch_fused (fused.cu) tries these kernels first; OCL_NO_SPEC=1 disables them.
+#include <stdio.h>
+
 #include <type_traits>
 
 #include "bulk.cuh"
@@ -22,13 +38,17 @@
 namespace ocl {
 
 enum : uint32_t { VX_COL = 0, VX_M1 = 1, VX_M1P = 2 };
-__host__ __device__ constexpr uint32_t vop(uint32_t kind, uint32_t a, uint32_t b = 0, uint32_t c = 0) {
-  return kind | (a << 2) | (b << 5) | (c << 8);
+enum : uint32_t { VS_SUM = 1, VS_MIN = 2, VS_MAX = 4 };
+// value descriptor: kind (2 bits) | a (3) | b (3) | c (3) | flags (3: SUM / MIN / MAX)
+__host__ __device__ constexpr uint32_t vop(uint32_t kind, uint32_t a, uint32_t b = 0, uint32_t c = 0,
+                                           uint32_t flags = VS_SUM) {
+  return kind | (a << 2) | (b << 5) | (c << 8) | (flags << 11);
 }
 __host__ __device__ constexpr uint32_t vx_kind(uint32_t o) { return o & 3; }
 __host__ __device__ constexpr uint32_t vx_a(uint32_t o) { return (o >> 2) & 7; }
 __host__ __device__ constexpr uint32_t vx_b(uint32_t o) { return (o >> 5) & 7; }
 __host__ __device__ constexpr uint32_t vx_c(uint32_t o) { return (o >> 8) & 7; }
+__host__ __device__ constexpr uint32_t vx_flags(uint32_t o) { return (o >> 11) & 7; }
 
 // PW: predicate column width (0 = no predicate); K0W/K1W: key widths (0 = absent);
 // NC: distinct value columns (all i64, or all f64 when F64); OPS: value expressions.
@@ -46,6 +66,13 @@ struct Sig {
   }
   static constexpr int KBITS = 8 * (K0W + K1W);
   static constexpr bool NARROW_KEY = KBITS < 32;   // 0xFFFFFFFF can never be a key
+  __host__ __device__ static constexpr bool has(int v, uint32_t f) { return (vx_flags(OP(v)) & f) != 0; }
+  // the CTA-table tier holds integer COL values (int32 fast path) only
+  __host__ __device__ static constexpr bool cta_ok() {
+    for (int v = 0; v < NV; ++v)
+      if (vx_kind(OP(v)) != VX_COL) return false;
+    return !F64;
+  }
 };
 
 struct SpecPlan {
@@ -55,6 +82,9 @@ struct SpecPlan {
   const void* k0;
   const void* k1;
   const void* col[4];
+  uint32_t tab_hb;            // replicated-table tier: log2 of the slots per replica (H)
+  uint32_t tab_nrep;          // replicated-table tier: replicas per CTA
+  int32_t pwait, cwait;       // barrier wait strategies of the producer / consumers (mbar_wait_mode)
 };
 
 template <class S>
@@ -108,6 +138,12 @@ __device__ __forceinline__ int64_t spec_mul_wide_s32(int32_t a, int32_t b) {
 __device__ __forceinline__ uint32_t spec_i32_bad(int64_t x) {
   return (uint32_t)((uint64_t)x >> 32) ^ (uint32_t)((int32_t)(uint32_t)x >> 31);
 }
+
+// order-preserving 32-bit encodings of int32 (zero-initialised = identity for a max)
+__device__ __forceinline__ uint32_t s_enc32_max(int32_t v) { return (uint32_t)v ^ 0x80000000u; }
+__device__ __forceinline__ uint32_t s_enc32_min(int32_t v) { return ~s_enc32_max(v); }
+__device__ __forceinline__ int32_t s_dec32_max(uint32_t e) { return (int32_t)(e ^ 0x80000000u); }
+__device__ __forceinline__ int32_t s_dec32_min(uint32_t e) { return s_dec32_max(~e); }
 
 template <class S>
 using KeyT = typename std::conditional<(S::KBITS <= 32), uint32_t, uint64_t>::type;
@@ -173,47 +209,90 @@ __device__ __forceinline__ void spec_values(const SpecPlan& p, const uint64_t (&
 }
 
 // ------------------------------------------------------------------ private accumulators
-// Low-G tier: every thread owns one accumulator set per group slot in shared memory
-// (conflict-free: lane t always hits the same banks whatever its slot).  A row costs
-// one slot-indexed read-modify-write per accumulator — no atomics, no per-slot
-// predication — the limit of the paper's "multiple accumulators per group" in local
-// memory.
-//   count      u32   (rows per thread < 2^32)
-//   COL value  i64   (fast path: the value fits int32, so < 2^32 of them fit)
-//   product    96-bit = u64 lo + u32 hi (fast-path products < 2^62)
-//   fp64       double
+// Every thread owns one accumulator set per group slot in shared memory (conflict-free:
+// lane t always hits the same banks whatever its slot).  Fields per (slot, thread):
+//   count       u32   (rows per thread < 2^32)
+//   SUM of COL  i64   (fast path: the value fits int32, so < 2^32 of them fit)
+//   SUM product 96-bit = u64 lo + u32 hi (fast-path products < 2^62)
+//   SUM fp64    double
+//   MIN / MAX   order-encoded u32 of the int32 value (int) / u64 of the double (fp64),
+//               updated with max(), so the zeroed record is the identity
 constexpr int kPrivThreads = 256;
 constexpr int kPrivSlots = 4;
 
 template <class S>
 struct Acc {
-  static constexpr int nnar() {
-    int c = 0;
-    for (int v = 0; v < S::NV; ++v) c += vx_kind(S::OP(v)) == VX_COL ? 1 : 0;
-    return c;
+  __host__ __device__ static constexpr bool is_nar(uint32_t o) {
+    return !S::F64 && vx_kind(o) == VX_COL && (vx_flags(o) & VS_SUM);
   }
-  static constexpr int NNAR = S::F64 ? 0 : nnar();
-  static constexpr int NWIDE = S::F64 ? 0 : S::NV - nnar();
-  static constexpr int NDBL = S::F64 ? S::NV : 0;
+  __host__ __device__ static constexpr bool is_wide(uint32_t o) {
+    return !S::F64 && vx_kind(o) != VX_COL && (vx_flags(o) & VS_SUM);
+  }
+  __host__ __device__ static constexpr bool is_dbl(uint32_t o) { return S::F64 && (vx_flags(o) & VS_SUM); }
+  __host__ __device__ static constexpr int nmm_of(uint32_t o) {
+    return ((vx_flags(o) & VS_MIN) ? 1 : 0) + ((vx_flags(o) & VS_MAX) ? 1 : 0);
+  }
   __host__ __device__ static constexpr int nar_idx(int v) {
     int c = 0;
-    for (int i = 0; i < v; ++i) c += vx_kind(S::OP(i)) == VX_COL ? 1 : 0;
+    for (int i = 0; i < v; ++i) c += is_nar(S::OP(i)) ? 1 : 0;
     return c;
   }
-  __host__ __device__ static constexpr int wide_idx(int v) { return v - nar_idx(v); }
-  // Slot-major layout: slot s owns slot_bytes(T) bytes; inside it one T-thread array
-  // per field: [count u32][narrow i64 x NNAR][wide lo u64 x NWIDE][fp64 x NDBL]
-  // [wide hi u32 x NWIDE].  A row addresses every field from two per-row bases
-  // (slot base + 4*tid, slot base + 8*tid) plus compile-time offsets.
+  __host__ __device__ static constexpr int wide_idx(int v) {
+    int c = 0;
+    for (int i = 0; i < v; ++i) c += is_wide(S::OP(i)) ? 1 : 0;
+    return c;
+  }
+  __host__ __device__ static constexpr int dbl_idx(int v) {
+    int c = 0;
+    for (int i = 0; i < v; ++i) c += is_dbl(S::OP(i)) ? 1 : 0;
+    return c;
+  }
+  __host__ __device__ static constexpr int mm_before(int v) {
+    int c = 0;
+    for (int i = 0; i < v; ++i) c += nmm_of(S::OP(i));
+    return c;
+  }
+  static constexpr int NNAR = nar_idx(S::NV);
+  static constexpr int NWIDE = wide_idx(S::NV);
+  static constexpr int NDBL = dbl_idx(S::NV);
+  static constexpr int NMM = mm_before(S::NV);
+  static constexpr int NMM64 = S::F64 ? NMM : 0;
+  static constexpr int NMM32 = S::F64 ? 0 : NMM;
+  // mm field index of value v's MIN (which = 0) or MAX (which = 1)
+  __host__ __device__ static constexpr int mm_idx(int v, int which) {
+    return mm_before(v) + ((which == 1 && (vx_flags(S::OP(v)) & VS_MIN)) ? 1 : 0);
+  }
+  // Slot-major layout: slot s owns slot_bytes(T) bytes; inside it one T-thread array per
+  // field: [count u32][narrow i64 x NNAR][wide lo u64 x NWIDE][fp64 x NDBL][mm u64 x NMM64]
+  // [wide hi u32 x NWIDE][mm u32 x NMM32].  A row addresses every field from two per-row
+  // bases (slot base + 4*tid, slot base + 8*tid) plus compile-time offsets.
   __host__ __device__ static constexpr size_t slot_bytes(int T) {
-    return ((size_t)T * (4 + 8 * NNAR + 12 * NWIDE + 8 * NDBL) + 15) / 16 * 16;
+    return ((size_t)T * (4 + 8 * (NNAR + NWIDE + NDBL + NMM64) + 4 * (NWIDE + NMM32)) + 15) / 16 * 16;
   }
   __host__ __device__ static constexpr int f_nar(int i, int T) { return 4 * T + 8 * T * i; }
   __host__ __device__ static constexpr int f_wlo(int i, int T) { return 4 * T + 8 * T * (NNAR + i); }
   __host__ __device__ static constexpr int f_dbl(int i, int T) { return 4 * T + 8 * T * (NNAR + NWIDE + i); }
-  __host__ __device__ static constexpr int f_whi(int i, int T) { return 4 * T + 8 * T * (NNAR + NWIDE + NDBL) + 4 * T * i; }
+  __host__ __device__ static constexpr int f_mm64(int i, int T) { return 4 * T + 8 * T * (NNAR + NWIDE + NDBL + i); }
+  __host__ __device__ static constexpr int f_whi(int i, int T) {
+    return 4 * T + 8 * T * (NNAR + NWIDE + NDBL + NMM64) + 4 * T * i;
+  }
+  __host__ __device__ static constexpr int f_mm32(int i, int T) { return f_whi(NWIDE, T) + 4 * T * i; }
   // L slots plus the trash record of the integer pair update
   __host__ __device__ static constexpr size_t bytes(int L, int T) { return (size_t)(L + (S::F64 ? 0 : 1)) * slot_bytes(T); }
+  // flush fields: count, then per value SUM / MIN / MAX as flagged
+  static constexpr int NF = 1 + NNAR + NWIDE + NDBL + NMM;
+  // field f -> (kind: 0 count, 1 sum, 2 min, 3 max) | v << 2
+  __host__ __device__ static constexpr int field(int f) {
+    if (f == 0) return 0;
+    int i = 1;
+    for (int v = 0; v < S::NV; ++v) {
+      const uint32_t fl = vx_flags(S::OP(v));
+      if (fl & VS_SUM) { if (i == f) return 1 | (v << 2); ++i; }
+      if (fl & VS_MIN) { if (i == f) return 2 | (v << 2); ++i; }
+      if (fl & VS_MAX) { if (i == f) return 3 | (v << 2); ++i; }
+    }
+    return -1;
+  }
 };
 
 template <class S>
@@ -229,7 +308,18 @@ __device__ __forceinline__ void priv_add_f64(uint8_t* sm, int slot, int tid, con
   uint8_t* b = sm + (size_t)slot * A::slot_bytes(T);
   *(uint32_t*)(b + 4 * tid) += 1u;
 #pragma unroll
-  for (int v = 0; v < S::NV; ++v) *(double*)(b + 8 * tid + A::f_dbl(v, T)) += x.vd[v];
+  for (int v = 0; v < S::NV; ++v) {
+    if constexpr (A::NDBL > 0)
+      if (S::has(v, VS_SUM)) *(double*)(b + 8 * tid + A::f_dbl(A::dbl_idx(v), T)) += x.vd[v];
+    if (S::has(v, VS_MIN)) {
+      uint64_t* m = (uint64_t*)(b + 8 * tid + A::f_mm64(A::mm_idx(v, 0), T));
+      *m = max(*m, enc_min_f(x.vd[v]));
+    }
+    if (S::has(v, VS_MAX)) {
+      uint64_t* m = (uint64_t*)(b + 8 * tid + A::f_mm64(A::mm_idx(v, 1), T));
+      *m = max(*m, enc_max_f(x.vd[v]));
+    }
+  }
 }
 
 __device__ __forceinline__ void add96(uint64_t& l, uint32_t& h, int64_t v) {
@@ -250,7 +340,7 @@ template <class S, int L, int T>
 __device__ __forceinline__ void priv_add2(uint8_t* sm, int s0, int s1, bool g0, bool g1, int tid, const SRow<S>& x0,
                                           const SRow<S>& x1) {
   using A = Acc<S>;
-  constexpr int NN = A::NNAR > 0 ? A::NNAR : 1, NW = A::NWIDE > 0 ? A::NWIDE : 1;
+  constexpr int NN = A::NNAR > 0 ? A::NNAR : 1, NW = A::NWIDE > 0 ? A::NWIDE : 1, NM = A::NMM32 > 0 ? A::NMM32 : 1;
   s0 = g0 ? s0 : L;
   s1 = g1 ? s1 : L;
   const bool same = s0 == s1;
@@ -262,7 +352,7 @@ __device__ __forceinline__ void priv_add2(uint8_t* sm, int s0, int s1, bool g0, 
   const uint32_t c0 = *c0p, c1 = *c1p;
   int64_t n0[NN], n1[NN];
   uint64_t wl0[NW], wl1[NW];
-  uint32_t wh0[NW], wh1[NW];
+  uint32_t wh0[NW], wh1[NW], m0[NM], m1[NM];
 #pragma unroll
   for (int i = 0; i < A::NNAR; ++i) {
     n0[i] = *(const int64_t*)(b0 + 8 * tid + A::f_nar(i, T));
@@ -275,23 +365,40 @@ __device__ __forceinline__ void priv_add2(uint8_t* sm, int s0, int s1, bool g0, 
     wh0[i] = *(const uint32_t*)(b0 + 4 * tid + A::f_whi(i, T));
     wh1[i] = *(const uint32_t*)(b1 + 4 * tid + A::f_whi(i, T));
   }
+#pragma unroll
+  for (int i = 0; i < A::NMM32; ++i) {
+    m0[i] = *(const uint32_t*)(b0 + 4 * tid + A::f_mm32(i, T));
+    m1[i] = *(const uint32_t*)(b1 + 4 * tid + A::f_mm32(i, T));
+  }
   // arithmetic: record 1 continues from record 0 when both are the same slot
   const uint32_t cn0 = c0 + 1u;
   const uint32_t cn1 = (same ? cn0 : c1) + 1u;
 #pragma unroll
   for (int v = 0; v < S::NV; ++v) {
-    if (vx_kind(S::OP(v)) == VX_COL) {
-      const int i = A::nar_idx(v);
-      n0[i] += (int64_t)(int32_t)x0.vi[v];
-      n1[i] = (same ? n0[i] : n1[i]) + (int64_t)(int32_t)x1.vi[v];
-    } else {
-      const int i = A::wide_idx(v);
-      add96(wl0[i], wh0[i], x0.vi[v]);
-      if (same) {
-        wl1[i] = wl0[i];
-        wh1[i] = wh0[i];
+    if (S::has(v, VS_SUM)) {
+      if (vx_kind(S::OP(v)) == VX_COL) {
+        const int i = A::nar_idx(v);
+        n0[i] += (int64_t)(int32_t)x0.vi[v];
+        n1[i] = (same ? n0[i] : n1[i]) + (int64_t)(int32_t)x1.vi[v];
+      } else {
+        const int i = A::wide_idx(v);
+        add96(wl0[i], wh0[i], x0.vi[v]);
+        if (same) {
+          wl1[i] = wl0[i];
+          wh1[i] = wh0[i];
+        }
+        add96(wl1[i], wh1[i], x1.vi[v]);
       }
-      add96(wl1[i], wh1[i], x1.vi[v]);
+    }
+    if (S::has(v, VS_MIN)) {
+      const int i = A::mm_idx(v, 0);
+      m0[i] = max(m0[i], s_enc32_min((int32_t)x0.vi[v]));
+      m1[i] = max(same ? m0[i] : m1[i], s_enc32_min((int32_t)x1.vi[v]));
+    }
+    if (S::has(v, VS_MAX)) {
+      const int i = A::mm_idx(v, 1);
+      m0[i] = max(m0[i], s_enc32_max((int32_t)x0.vi[v]));
+      m1[i] = max(same ? m0[i] : m1[i], s_enc32_max((int32_t)x1.vi[v]));
     }
   }
   // stores (record 1 last)
@@ -303,6 +410,8 @@ __device__ __forceinline__ void priv_add2(uint8_t* sm, int s0, int s1, bool g0, 
     *(uint64_t*)(b0 + 8 * tid + A::f_wlo(i, T)) = wl0[i];
     *(uint32_t*)(b0 + 4 * tid + A::f_whi(i, T)) = wh0[i];
   }
+#pragma unroll
+  for (int i = 0; i < A::NMM32; ++i) *(uint32_t*)(b0 + 4 * tid + A::f_mm32(i, T)) = m0[i];
   *c1p = cn1;
 #pragma unroll
   for (int i = 0; i < A::NNAR; ++i) *(int64_t*)(b1 + 8 * tid + A::f_nar(i, T)) = n1[i];
@@ -311,44 +420,56 @@ __device__ __forceinline__ void priv_add2(uint8_t* sm, int s0, int s1, bool g0, 
     *(uint64_t*)(b1 + 8 * tid + A::f_wlo(i, T)) = wl1[i];
     *(uint32_t*)(b1 + 4 * tid + A::f_whi(i, T)) = wh1[i];
   }
+#pragma unroll
+  for (int i = 0; i < A::NMM32; ++i) *(uint32_t*)(b1 + 4 * tid + A::f_mm32(i, T)) = m1[i];
 }
 
-// Slot of a row; resolves the rare cases (a key new to this CTA -> directory insert;
-// a slow value or a key beyond the slots -> exact per-row update of the HBM table).
-// Returns true iff the row accumulates in private slot `slot`.
+// ------------------------------------------------------------------ slot lookup
+// The slot keys are cached in registers (rk); a key new to the CTA is claimed in the
+// shared directory `dir` (64-bit CAS), then rk is refreshed.
+template <int L>
+struct DirState {
+  uint64_t* dir;      // the L slot keys (~key, 0 = free)
+};
+
+// Slot of a row; resolves the rare cases (a key new to this CTA; a slow value or a key
+// beyond the slots -> exact per-row update of the HBM table).  Returns true iff the row
+// accumulates in private slot `slot`.
 template <class S, int L>
-__device__ __forceinline__ bool priv_slot(const SpecPlan& p, uint64_t* dir, KeyT<S> (&rk)[L], const SRow<S>& x,
-                                          int64_t r, int& slot) {
+__device__ __forceinline__ bool priv_slot(const SpecPlan& p, const DirState<L>& d, KeyT<S> (&rk)[L],
+                                          const SRow<S>& x, int64_t r, int& slot) {
+  static_assert(L <= 4, "slot keys are compared in registers");
+  const bool special = spec_is_special<S>(x.key);
   slot = -1;
 #pragma unroll
   for (int s = L - 1; s >= 0; --s)
     if (x.key == rk[s]) slot = s;
-  const bool special = spec_is_special<S>(x.key);
   bool go = x.q && x.fast && slot >= 0 && !special;
-  if (x.q && !go) {                                    // rare: new key in this CTA, or slow value
-    slot = (x.fast && !special) ? dir_find_or_insert<L>(dir, (uint64_t)x.key) : -1;
+  if (x.q && !go && x.fast && !special) {            // rare: new key in this CTA
+    slot = dir_find_or_insert<L>(d.dir, (uint64_t)x.key);
     if (slot >= 0) {
 #pragma unroll
       for (int s = 0; s < L; ++s) {
-        uint64_t sk = *(volatile uint64_t*)&dir[s];
+        uint64_t sk = *(volatile uint64_t*)&d.dir[s];
         rk[s] = sk ? (KeyT<S>)~sk : (KeyT<S>)~0ULL;
       }
       go = true;
-    } else {
-      uint8_t* e = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, (uint64_t)x.key, p.g.status);
-      if (e) update_entry_slow(p.g, e, r);
     }
+  }
+  if (x.q && !go) {                                   // slow value, key ~0, or no slot left
+    uint8_t* e = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, (uint64_t)x.key, p.g.status);
+    if (e) update_entry_slow(p.g, e, r);
   }
   return go;
 }
 
 // Both rows (r, r + 1) of a lane.
-template <class S, int L, int T = kPrivThreads>
-__device__ __forceinline__ void priv_rows(const SpecPlan& p, uint64_t* dir, KeyT<S> (&rk)[L], uint8_t* sm, int tid,
-                                          const SRow<S>& x0, const SRow<S>& x1, int64_t r) {
+template <class S, int L, int T>
+__device__ __forceinline__ void priv_rows(const SpecPlan& p, const DirState<L>& d, KeyT<S> (&rk)[L], uint8_t* sm,
+                                          int tid, const SRow<S>& x0, const SRow<S>& x1, int64_t r) {
   int s0, s1;
-  const bool g0 = priv_slot<S, L>(p, dir, rk, x0, r, s0);
-  const bool g1 = priv_slot<S, L>(p, dir, rk, x1, r + 1, s1);
+  const bool g0 = priv_slot<S, L>(p, d, rk, x0, r, s0);
+  const bool g1 = priv_slot<S, L>(p, d, rk, x1, r + 1, s1);
   if constexpr (S::F64) {
     if (g0) priv_add_f64<S, L, T>(sm, s0, tid, x0);
     if (g1) priv_add_f64<S, L, T>(sm, s1, tid, x1);
@@ -374,25 +495,25 @@ __device__ __forceinline__ void spec_row_scalar(const SpecPlan& p, int64_t r, SR
   spec_values<S>(p, c, x);
 }
 
-// Flush: the CTA's T private records of every (slot, field) are summed in parallel --
-// Q threads per (slot, field), each over T/Q records, then Q-lane shuffles -- and added
+// Flush: the CTA's T private records of every (slot, field) are reduced in parallel --
+// Q threads per (slot, field), each over T/Q records, then Q-lane shuffles -- and merged
 // into the slot's global entry.  (A warp-by-warp shuffle tree per (slot, field) was a
 // serial chain of ~NV x 5 dependent shuffles per slot: on C1, one chunk per CTA, that
 // chain was most of the kernel.)  One thread per slot resolves the entry first.
 // Every thread of the CTA calls it (barriers); threads tid >= T (a producer warp) only
 // take part in the barriers.
 template <class S, int L, int T>
-__device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm, const uint64_t* dir, int tid) {
+__device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm, const DirState<L>& d, int tid) {
   using A = Acc<S>;
   constexpr int Q = 4;                     // threads per (slot, field)
   constexpr int PER = T / Q;               // records each of them sums (interleaved: j = sub + Q k,
                                            // so the Q lanes of a group read Q different banks)
-  constexpr int F = 1 + S::NV;             // COUNT + the value sums
+  constexpr int F = A::NF;
   static_assert(T % (32 * Q) == 0 || 32 % Q == 0, "Q lanes of a group share a warp");
   __shared__ uint8_t* ent[L];
   __syncthreads();
   if (tid < L) {
-    const uint64_t sk = dir[tid];
+    const uint64_t sk = d.dir[tid];
     ent[tid] = sk != 0 ? table_find_or_insert(p.g.table, p.g.mask, p.g.stride, ~sk, p.g.status) : nullptr;
   }
   __syncthreads();
@@ -400,11 +521,13 @@ __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm,
   const int sub = tid % Q;
   const unsigned gmask = ((1u << Q) - 1) << ((tid & 31) & ~(Q - 1));
   for (int i = tid / Q; i < L * F; i += T / Q) {   // uniform within a Q group
-    const int s = i / F, v = i % F - 1;
+    const int s = i / F;
+    const int fd = A::field(i % F);
+    const int kind = fd & 3, v = fd >> 2;
     uint8_t* e = ent[s];
     if (e == nullptr) continue;
     const uint8_t* sb = sm + (size_t)s * A::slot_bytes(T);
-        if (v < 0) {
+    if (kind == 0) {
       const uint32_t* c = (const uint32_t*)sb + sub;
       unsigned long long cw = 0;
 #pragma unroll 8
@@ -413,20 +536,44 @@ __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm,
       if (sub == 0 && cw) atomicAdd((unsigned long long*)(e + 8), cw);
       continue;
     }
+    if (kind >= 2) {                       // MIN / MAX: max over the encodings, then the HBM encoding
+      const int mi = A::mm_idx(v, kind - 2);
+      unsigned long long m = 0;
+      if constexpr (S::F64) {
+        const uint64_t* d64 = (const uint64_t*)(sb + A::f_mm64(mi, T)) + sub;
+#pragma unroll 8
+        for (int j = 0; j < PER; ++j) m = max(m, (unsigned long long)d64[Q * j]);
+      } else {
+        const uint32_t* d32 = (const uint32_t*)(sb + A::f_mm32(mi, T)) + sub;
+        uint32_t m32 = 0;
+#pragma unroll 8
+        for (int j = 0; j < PER; ++j) m32 = max(m32, d32[Q * j]);
+        m = m32;
+      }
+      for (int o = Q / 2; o > 0; o >>= 1) m = max(m, __shfl_xor_sync(gmask, m, o));
+      if (sub == 0) {
+        const int off = kind == 2 ? p.g.vals[v].off_min : p.g.vals[v].off_max;
+        unsigned long long enc = m;        // fp64: the HBM table uses the same encodings
+        if constexpr (!S::F64)
+          enc = kind == 2 ? enc_min_i((int64_t)s_dec32_min((uint32_t)m)) : enc_max_i((int64_t)s_dec32_max((uint32_t)m));
+        if (off >= 0) atomicMax((unsigned long long*)(e + off), enc);
+      }
+      continue;
+    }
     const int off = p.g.vals[v].off_sum;
     if constexpr (S::F64) {
-      const double* d = (const double*)(sb + A::f_dbl(v, T)) + sub;
+      const double* dd = (const double*)(sb + A::f_dbl(A::dbl_idx(v), T)) + sub;
       double sum = 0.0;
 #pragma unroll 8
-      for (int j = 0; j < PER; ++j) sum += d[Q * j];
+      for (int j = 0; j < PER; ++j) sum += dd[Q * j];
       for (int o = Q / 2; o > 0; o >>= 1) sum += __shfl_xor_sync(gmask, sum, o);
       if (sub == 0 && off >= 0) atomicAdd((double*)(e + off), sum);
     } else {
       I128 x{0, 0};
       if (vx_kind(S::OP(v)) == VX_COL) {
-        const int64_t* d = (const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)) + sub;
+        const int64_t* dn = (const int64_t*)(sb + A::f_nar(A::nar_idx(v), T)) + sub;
 #pragma unroll 8
-        for (int j = 0; j < PER; ++j) x = i128_add(x, i128_from_i64(d[Q * j]));
+        for (int j = 0; j < PER; ++j) x = i128_add(x, i128_from_i64(dn[Q * j]));
       } else {
         const uint64_t* lo = (const uint64_t*)(sb + A::f_wlo(A::wide_idx(v), T)) + sub;
         const uint32_t* hi = (const uint32_t*)(sb + A::f_whi(A::wide_idx(v), T)) + sub;
@@ -444,13 +591,159 @@ __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm,
   }
 }
 
+// ------------------------------------------------------------------ replicated-table tier
+// "Multiple accumulators per group, inversely proportional to the number of groups"
+// (§4.1.7): nrep replicas of a shared-memory hash table of H = pow2 >= 2G slots
+// per CTA, consumer warp w updating replica w % nrep, so cross-warp contention falls as G
+// falls (G = 16: one replica per warp).  A replica is stored field-major (SoA) so that the
+// 32 lanes of an atomic instruction on 32 different slots hit different banks: keys u64[H]
+// (~key, 0 = empty), count u32[H], then per value SUM -> biased sum lo u32[H], hi u32[H]
+// (the sum of (x + 2^31) over the rows, exact in 64 bits; sum = biased - count * 2^31; the
+// carry out of lo is taken from the atomic's return value), MIN / MAX -> order-encoded
+// u32[H]; all updated with native 32-bit shared atomics.  All-zero = empty / identity.
+// The home slot is read without a loop (one LDS.64 + compare); probing and claiming run
+// out of line for the warp's misses only.
+template <class S>
+struct TabL {
+  // u32 field index of count / value v's sum lo, sum hi, min, max (after the u64 keys)
+  __host__ __device__ static constexpr int nfield_before(int v) {
+    int o = 1;
+    for (int i = 0; i < v; ++i) {
+      const uint32_t f = vx_flags(S::OP(i));
+      o += ((f & VS_SUM) ? 2 : 0) + ((f & VS_MIN) ? 1 : 0) + ((f & VS_MAX) ? 1 : 0);
+    }
+    return o;
+  }
+  __host__ __device__ static constexpr int f_sum(int v) { return nfield_before(v); }
+  __host__ __device__ static constexpr int f_min(int v) { return nfield_before(v) + ((vx_flags(S::OP(v)) & VS_SUM) ? 2 : 0); }
+  __host__ __device__ static constexpr int f_max(int v) { return f_min(v) + ((vx_flags(S::OP(v)) & VS_MIN) ? 1 : 0); }
+  static constexpr int NF32 = nfield_before(S::NV);
+  static constexpr int BYTES_PER_SLOT = 8 + 4 * NF32;
+  // replica of H slots: keys at 0, u32 field f at 8H + 4H f
+  __device__ static uint32_t* fld(uint8_t* rep, uint32_t H, int f) { return (uint32_t*)(rep + 8 * (size_t)H + 4 * (size_t)H * f); }
+};
+
+constexpr uint64_t kTabMul = 0x9E3779B97F4A7C15ULL;   // multiplicative hash: home slot = top hb bits
+
+// A warp's replica: slot count and field arrays, resolved once per kernel (registers).
+template <class S>
+struct TabRef {
+  uint64_t* keys;
+  uint32_t* f[TabL<S>::NF32];
+  uint32_t hb, mask;
+};
+
+template <class S>
+__device__ __forceinline__ TabRef<S> tab_ref(uint8_t* rep, uint32_t hb) {
+  TabRef<S> t;
+  const uint32_t H = 1u << hb;
+  t.keys = (uint64_t*)rep;
+  t.hb = hb;
+  t.mask = H - 1;
+#pragma unroll
+  for (int i = 0; i < TabL<S>::NF32; ++i) t.f[i] = TabL<S>::fld(rep, H, i);
+  return t;
+}
+
+// Out-of-line probe / claim over whole buckets from the home bucket: slot, or -1 when the
+// replica is full.
+__device__ __noinline__ int tab_find_slow(uint64_t* keys, uint32_t hb, uint64_t key) {
+  const uint32_t nb = 1u << (hb - 2);
+  const uint64_t sk = ~key;
+  uint32_t b = (uint32_t)((key * kTabMul) >> (64 - (hb - 2)));
+  for (uint32_t probe = 0; probe < nb; ++probe) {
+    for (int j = 0; j < 4; ++j) {
+      uint64_t* kp = &keys[4 * b + j];
+      const uint64_t cur = *(volatile uint64_t*)kp;
+      if (cur == sk) return (int)(4 * b + j);
+      if (cur == 0) {
+        const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
+        if (prev == 0 || prev == sk) return (int)(4 * b + j);
+      }
+    }
+    b = (b + 1) & (nb - 1);
+  }
+  return -1;
+}
+
+// One row position of the warp (all 32 lanes call): the row into this warp's replica, or,
+// for a slow value / the key ~0 / a full replica, the exact HBM update.  Slots come in
+// buckets of 4 (32 bytes, read with two LDS.128); the home bucket is the top bits of
+// key * 2^64/phi.  A key present in its home bucket is found without a loop or a branch;
+// claims and bucket overflows go out of line, warp-uniformly, and only after warm-up rarely.
+template <class S>
+__device__ __forceinline__ void tab_row(const SpecPlan& p, const TabRef<S>& t, const SRow<S>& x, int64_t r) {
+  using TL = TabL<S>;
+  const uint64_t k = (uint64_t)x.key;
+  const uint64_t sk = ~k;
+  const bool ok = x.q && x.fast && !spec_is_special<S>(x.key);
+  const uint32_t b = (uint32_t)((k * kTabMul) >> (64 - (t.hb - 2)));
+  const ulonglong2* bp = (const ulonglong2*)(t.keys + 4 * b);
+  const ulonglong2 k01 = bp[0], k23 = bp[1];
+  int h = (int)(4 * b);
+  h = k01.x == sk ? h : (k01.y == sk ? h + 1 : (k23.x == sk ? h + 2 : (k23.y == sk ? h + 3 : -1)));
+  const bool miss = ok && h < 0;
+  if (__any_sync(0xffffffffu, miss))
+    if (miss) h = tab_find_slow(t.keys, t.hb, k);
+  if (x.q && (!ok || h < 0)) {                        // slow value, key ~0, or a full replica
+    uint8_t* g = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, k, p.g.status);
+    if (g) update_entry_slow(p.g, g, r);
+  }
+  if (!ok || h < 0) return;
+  atomicAdd(t.f[0] + h, 1u);
+#pragma unroll
+  for (int v = 0; v < S::NV; ++v) {
+    const int32_t xv = (int32_t)x.vi[v];
+    if (S::has(v, VS_SUM)) {                        // biased add, carry from the returned value
+      const uint32_t a = (uint32_t)xv ^ 0x80000000u;
+      const uint32_t old = atomicAdd(t.f[TL::f_sum(v)] + h, a);
+      if (old + a < old) atomicAdd(t.f[TL::f_sum(v) + 1] + h, 1u);
+    }
+    if (S::has(v, VS_MIN)) atomicMax(t.f[TL::f_min(v)] + h, s_enc32_min(xv));
+    if (S::has(v, VS_MAX)) atomicMax(t.f[TL::f_max(v)] + h, s_enc32_max(xv));
+  }
+}
+
+// Fold every replica into the HBM table (every thread of the CTA calls it).
+template <class S>
+__device__ __forceinline__ void tab_flush(const SpecPlan& p, uint8_t* tab, int tid, int nthreads) {
+  using TL = TabL<S>;
+  __syncthreads();
+  const uint32_t H = 1u << p.tab_hb;
+  const uint32_t slots = (uint32_t)p.tab_nrep * H;
+  for (uint32_t i = tid; i < slots; i += nthreads) {
+    uint8_t* rep = tab + (size_t)(i / H) * H * TL::BYTES_PER_SLOT;
+    const uint32_t h = i % H;
+    const uint64_t sk = ((const uint64_t*)rep)[h];
+    if (sk == 0) continue;
+    const uint32_t cnt = TL::fld(rep, H, 0)[h];
+    uint8_t* g = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, ~sk, p.g.status);
+    if (!g) continue;
+    atomicAdd((unsigned long long*)(g + 8), (unsigned long long)cnt);
+#pragma unroll
+    for (int v = 0; v < S::NV; ++v) {
+      const DevValue& d = p.g.vals[v];
+      if (S::has(v, VS_SUM) && d.off_sum >= 0) {
+        const uint64_t b = (uint64_t)TL::fld(rep, H, TL::f_sum(v))[h] | ((uint64_t)TL::fld(rep, H, TL::f_sum(v) + 1)[h] << 32);
+        const int64_t sum = (int64_t)(b - ((uint64_t)cnt << 31));
+        atomic_add_i128((uint64_t*)(g + d.off_sum), (uint64_t)sum, (uint64_t)(sum >> 63));
+      }
+      if (S::has(v, VS_MIN) && d.off_min >= 0)
+        atomicMax((unsigned long long*)(g + d.off_min),
+                  (unsigned long long)enc_min_i(s_dec32_min(TL::fld(rep, H, TL::f_min(v))[h])));
+      if (S::has(v, VS_MAX) && d.off_max >= 0)
+        atomicMax((unsigned long long*)(g + d.off_max),
+                  (unsigned long long)enc_max_i(s_dec32_max(TL::fld(rep, H, TL::f_max(v))[h])));
+    }
+  }
+}
+
 // ------------------------------------------------------------------ TMA bulk pipeline
-// Same rows, semantics and accumulators as k_sga_priv, but the columns reach shared
-// memory through the copy engine: one producer thread streams R-row chunks of every
-// column with cp.async.bulk into an NS-stage ring (mbarrier full/empty pairs); the T
-// consumer threads read their rows from shared memory.  Loads no longer occupy the
-// consumers' issue slots or registers, and the bytes in flight per SM (NS stages) do
-// not depend on where the consumer warps are in their row loop.
+// The columns reach shared memory through the copy engine: one producer thread streams
+// R-row chunks of every column with cp.async.bulk into an NS-stage ring (mbarrier
+// full/empty pairs); the T consumer threads read their rows from shared memory.  Loads
+// no longer occupy the consumers' issue slots or registers, and the bytes in flight per
+// SM (NS stages) do not depend on where the consumer warps are in their row loop.
 template <class S, int R>
 struct BulkStage {
   static constexpr int OFF_P = 0;
@@ -478,28 +771,38 @@ __device__ __forceinline__ void lds2(const uint8_t* base, int j, uint64_t& x0, u
   }
 }
 
-template <class S>
-__host__ __device__ constexpr size_t bulk_acc_bytes(int L, int T) {
-  return (Acc<S>::bytes(L, T) + 127) / 128 * 128;
+// Shared-memory bytes of the accumulation tier: L > 0 private records; L == 0 the replicated
+// tables (nrep x H slots, run time).
+template <class S, int L>
+__host__ __device__ constexpr size_t tier_bytes(int T, uint32_t tab_slots) {
+  return L > 0 ? (Acc<S>::bytes(L, T) + 127) / 128 * 128 : ((size_t)tab_slots * TabL<S>::BYTES_PER_SLOT + 127) / 128 * 128;
 }
 
+// minimum resident CTAs per SM for the register budget: without it ptxas capped the Q1
+// kernel at 72 registers and spilled two values per 64-row unit to local memory (+0.6 GB
+// of L2 traffic on C4, 3.56 -> 4.19 ms); the shared-memory footprint allows 2-3 CTAs anyway
+template <int T>
+constexpr int bulk_min_blocks() { return T <= 128 ? 3 : 2; }
+
 template <class S, int L, int T, int R, int NS>
-__global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ SpecPlan p) {
-  using A = Acc<S>;
+__global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const __grid_constant__ SpecPlan p) {
   using B = BulkStage<S, R>;
   constexpr int NW = T / 32;                 // consumer warps
   constexpr int UPW = R / 64 / NW;           // 64-row units per consumer warp per stage
   static_assert(UPW >= 1 && UPW * 64 * NW == R, "R must be 64 * consumer warps * units");
+  constexpr int LD = L > 0 ? L : 1;
   extern __shared__ __align__(128) uint8_t sm[];
-  uint8_t* stg = sm + bulk_acc_bytes<S>(L, T);
-  __shared__ uint64_t dir[L];
+  const uint32_t tab_slots = L > 0 ? 0u : ((uint32_t)p.tab_nrep << p.tab_hb);
+  const size_t tb = tier_bytes<S, L>(T, tab_slots);
+  uint8_t* stg = sm + tb;
+  __shared__ uint64_t dir[LD];
   __shared__ __align__(8) uint64_t full[NS], empty[NS];
   const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
   {
     uint4* z = (uint4*)sm;
-    for (int i = tid; i < (int)(A::bytes(L, T) / 16); i += T + 32) z[i] = make_uint4(0, 0, 0, 0);
+    for (int i = tid; i < (int)(tb / 16); i += T + 32) z[i] = make_uint4(0, 0, 0, 0);
   }
-  if (tid < L) dir[tid] = 0;
+  for (int i = tid; i < LD; i += T + 32) dir[i] = 0;
   if (tid == 0) {
     for (int s = 0; s < NS; ++s) {
       mbar_init(&full[s], 1);
@@ -508,6 +811,12 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
     mbar_fence_init();
   }
   __syncthreads();
+  const DirState<LD> d{dir};
+  // replicated-table tier: this warp's replica
+  const TabRef<S> mytab = tab_ref<S>(sm + (L > 0 ? 0 : (size_t)(wid % (p.tab_nrep ? p.tab_nrep : 1)) *
+                                                         ((size_t)1 << p.tab_hb) * TabL<S>::BYTES_PER_SLOT),
+                                     L > 0 ? 5u : p.tab_hb);
+  (void)lane;
   const int64_t n = p.g.n;
   const int64_t nfull = n / R;
   if (wid == NW) {
@@ -517,17 +826,17 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
       int stage = 0;
       uint32_t phase = 0;
       for (int64_t c = blockIdx.x; c < nfull; c += gridDim.x) {
-        mbar_wait(&empty[stage], phase ^ 1);
+        mbar_wait_mode(&empty[stage], phase ^ 1, p.pwait);
         uint64_t* fb = &full[stage];
         mbar_arrive_expect_tx(fb, B::BYTES);
-        uint8_t* d = stg + (size_t)stage * B::BYTES;
+        uint8_t* dst = stg + (size_t)stage * B::BYTES;
         const int64_t r0 = c * R;
-        if constexpr (S::PW > 0) bulk_g2s(d + B::OFF_P, (const uint8_t*)p.pcol + r0 * S::PW, R * S::PW, fb, pol);
-        if constexpr (S::K0W > 0) bulk_g2s(d + B::OFF_K0, (const uint8_t*)p.k0 + r0 * S::K0W, R * S::K0W, fb, pol);
-        if constexpr (S::K1W > 0) bulk_g2s(d + B::OFF_K1, (const uint8_t*)p.k1 + r0 * S::K1W, R * S::K1W, fb, pol);
+        if constexpr (S::PW > 0) bulk_g2s(dst + B::OFF_P, (const uint8_t*)p.pcol + r0 * S::PW, R * S::PW, fb, pol);
+        if constexpr (S::K0W > 0) bulk_g2s(dst + B::OFF_K0, (const uint8_t*)p.k0 + r0 * S::K0W, R * S::K0W, fb, pol);
+        if constexpr (S::K1W > 0) bulk_g2s(dst + B::OFF_K1, (const uint8_t*)p.k1 + r0 * S::K1W, R * S::K1W, fb, pol);
 #pragma unroll
         for (int i = 0; i < S::NC; ++i)
-          bulk_g2s(d + B::OFF_C + i * R * 8, (const uint8_t*)p.col[i] + r0 * 8, R * 8, fb, pol);
+          bulk_g2s(dst + B::OFF_C + i * R * 8, (const uint8_t*)p.col[i] + r0 * 8, R * 8, fb, pol);
         if (++stage == NS) {
           stage = 0;
           phase ^= 1;
@@ -536,23 +845,23 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
     }
   } else {
     // ---- consumers
-    KeyT<S> rk[L];
+    KeyT<S> rk[LD];
 #pragma unroll
-    for (int s = 0; s < L; ++s) rk[s] = (KeyT<S>)~0ULL;
+    for (int s = 0; s < LD; ++s) rk[s] = (KeyT<S>)~0ULL;
     int stage = 0;
     uint32_t phase = 0;
     for (int64_t c = blockIdx.x; c < nfull; c += gridDim.x) {
-      mbar_wait(&full[stage], phase);
-      const uint8_t* d = stg + (size_t)stage * B::BYTES;
+      mbar_wait_mode(&full[stage], phase, p.cwait);
+      const uint8_t* sd = stg + (size_t)stage * B::BYTES;
       uint64_t pr[UPW][2], k0[UPW][2], k1[UPW][2], cv[UPW][2][S::NC];
 #pragma unroll
       for (int u = 0; u < UPW; ++u) {
         const int j = (wid * UPW + u) * 64 + 2 * lane;
-        if constexpr (S::PW > 0) lds2<S::PW>(d + B::OFF_P, j, pr[u][0], pr[u][1]);
-        if constexpr (S::K0W > 0) lds2<S::K0W>(d + B::OFF_K0, j, k0[u][0], k0[u][1]);
-        if constexpr (S::K1W > 0) lds2<S::K1W>(d + B::OFF_K1, j, k1[u][0], k1[u][1]);
+        if constexpr (S::PW > 0) lds2<S::PW>(sd + B::OFF_P, j, pr[u][0], pr[u][1]);
+        if constexpr (S::K0W > 0) lds2<S::K0W>(sd + B::OFF_K0, j, k0[u][0], k0[u][1]);
+        if constexpr (S::K1W > 0) lds2<S::K1W>(sd + B::OFF_K1, j, k1[u][0], k1[u][1]);
 #pragma unroll
-        for (int i = 0; i < S::NC; ++i) lds2<8>(d + B::OFF_C + i * R * 8, j, cv[u][0][i], cv[u][1][i]);
+        for (int i = 0; i < S::NC; ++i) lds2<8>(sd + B::OFF_C + i * R * 8, j, cv[u][0][i], cv[u][1][i]);
       }
       mbar_release_reads(&empty[stage], lane);       // the stage's bytes are in registers now
       if (++stage == NS) {
@@ -573,7 +882,12 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
           spec_values<S>(p, cv[u][k], x[k]);
         }
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base, lane, x[0].q, x[1].q);
-        priv_rows<S, L, T>(p, dir, rk, sm, tid, x[0], x[1], r);
+        if constexpr (L > 0) {
+          priv_rows<S, LD, T>(p, d, rk, sm, tid, x[0], x[1], r);
+        } else {
+          tab_row<S>(p, mytab, x[0], r);
+          tab_row<S>(p, mytab, x[1], r + 1);
+        }
       }
     }
     // ragged tail (< R rows): one CTA, scalar loads straight from global memory
@@ -584,11 +898,17 @@ __global__ void __launch_bounds__(T + 32) k_sga_bulk(const __grid_constant__ Spe
         spec_row_scalar<S>(p, r, x0);
         spec_row_scalar<S>(p, r + 1, x1);
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base, lane, x0.q, x1.q);
-        priv_rows<S, L, T>(p, dir, rk, sm, tid, x0, x1, r);
+        if constexpr (L > 0) {
+          priv_rows<S, LD, T>(p, d, rk, sm, tid, x0, x1, r);
+        } else {
+          tab_row<S>(p, mytab, x0, r);
+          tab_row<S>(p, mytab, x1, r + 1);
+        }
       }
     }
   }
-  priv_flush<S, L, T>(p, sm, dir, tid);
+  if constexpr (L > 0) priv_flush<S, LD, T>(p, sm, d, tid);
+  else tab_flush<S>(p, sm, tid, T + 32);
 }
 
 template <class S, int L>
@@ -604,6 +924,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant
   }
   if (tid < L) dir[tid] = 0;
   __syncthreads();
+  const DirState<L> d{dir};
   KeyT<S> rk[L];
 #pragma unroll
   for (int s = 0; s < L; ++s) rk[s] = (KeyT<S>)~0ULL;
@@ -640,7 +961,7 @@ __global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant
           spec_values<S>(p, c[u][k], x[k]);
         }
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base + 64 * u, lane, x[0].q, x[1].q);
-        priv_rows<S, L>(p, dir, rk, sm, tid, x[0], x[1], r);
+        priv_rows<S, L, T>(p, d, rk, sm, tid, x[0], x[1], r);
       }
     } else {
       for (int u = 0; u < U; ++u) {
@@ -649,11 +970,11 @@ __global__ void __launch_bounds__(kPrivThreads) k_sga_priv(const __grid_constant
         spec_row_scalar<S>(p, r, x0);
         spec_row_scalar<S>(p, r + 1, x1);
         if (p.g.bitmap_out) emit_bitmap_unit(p.g, base + 64 * u, lane, x0.q, x1.q);
-        priv_rows<S, L>(p, dir, rk, sm, tid, x0, x1, r);
+        priv_rows<S, L, T>(p, d, rk, sm, tid, x0, x1, r);
       }
     }
   }
-  priv_flush<S, L, T>(p, sm, dir, tid);
+  priv_flush<S, L, T>(p, sm, d, tid);
 }
 
 // ------------------------------------------------------------------ signature table
@@ -663,10 +984,18 @@ using SigQ1I = Sig<4, false, 1, 1, 4, false, vop(VX_COL, 0), vop(VX_COL, 1), vop
                    vop(VX_COL, 2)>;
 using SigQ1F = Sig<4, false, 1, 1, 4, true, vop(VX_COL, 0), vop(VX_COL, 1), vop(VX_M1, 1, 2), vop(VX_M1P, 1, 2, 3),
                    vop(VX_COL, 2)>;
+// Q1 + MIN(qty) + MAX(price) (bench workload c4mm): the same columns, two more states.
+using SigQ1IMM = Sig<4, false, 1, 1, 4, false, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN),
+                     vop(VX_COL, 1, 0, 0, VS_SUM | VS_MAX), vop(VX_M1, 1, 2), vop(VX_M1P, 1, 2, 3), vop(VX_COL, 2)>;
+using SigQ1FMM = Sig<4, false, 1, 1, 4, true, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN),
+                     vop(VX_COL, 1, 0, 0, VS_SUM | VS_MAX), vop(VX_M1, 1, 2), vop(VX_M1P, 1, 2, 3), vop(VX_COL, 2)>;
+// C5: WHERE p (i32) GROUP BY key (i64): COUNT, SUM, MIN, MAX of v (i64).  C3: the same
+// without the predicate (GROUP BY l_orderkey: COUNT, SUM / MIN / MAX(l_quantity)).
+using SigC5 = Sig<4, false, 8, 0, 1, false, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN | VS_MAX)>;
+using SigC3 = Sig<0, false, 8, 0, 1, false, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN | VS_MAX)>;
 
 template <class S>
 static bool spec_match(const Plan& g, SpecPlan* sp) {
-  if (g.has_minmax) return false;
   if ((S::PW > 0) != (g.npreds == 1) || g.npreds > 1) return false;
   if (S::PW > 0 && (g.preds[0].col.width != S::PW || (bool)g.preds[0].is_f64 != S::PF64)) return false;
   if (g.nkeys != (S::K0W > 0) + (S::K1W > 0)) return false;
@@ -688,7 +1017,10 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
   for (int v = 0; v < g.nvals; ++v) {
     const DevValue& d = g.vals[v];
     uint32_t op = S::OP(v);
-    if ((int)vx_kind(op) != d.expr || (bool)d.is_f64 != S::F64 || d.off_sum < 0) return false;
+    if ((int)vx_kind(op) != d.expr || (bool)d.is_f64 != S::F64) return false;
+    if ((d.off_sum >= 0) != S::has(v, VS_SUM) || (d.off_min >= 0) != S::has(v, VS_MIN) ||
+        (d.off_max >= 0) != S::has(v, VS_MAX))
+      return false;
     if (idx(d.a) != (int)vx_a(op)) return false;
     if (d.expr >= OCL_EXPR_MUL_1MINUS && idx(d.b) != (int)vx_b(op)) return false;
     if (d.expr >= OCL_EXPR_MUL_1MINUS_1PLUS && idx(d.c) != (int)vx_c(op)) return false;
@@ -707,6 +1039,10 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
   sp->k0 = S::K0W > 0 ? g.keys[0].col.ptr : nullptr;
   sp->k1 = S::K1W > 0 ? g.keys[1].col.ptr : nullptr;
   for (int i = 0; i < 4; ++i) sp->col[i] = i < nc ? cols[i] : nullptr;
+  sp->tab_hb = 0;
+  sp->tab_nrep = 0;
+  sp->pwait = 1;
+  sp->cwait = 0;
   return true;
 }
 
@@ -721,9 +1057,8 @@ static int spec_blocks_per_sm(size_t smem) {
 
 // Launch the bulk-pipeline kernel <S, L, T, R, NS>; false if it cannot run this plan
 // (columns not 16-byte aligned for the copy engine, or fewer rows than one stage).
-template <class S, int T, int R, int NS>
+template <class S, int L, int T, int R, int NS>
 static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err) {
-  constexpr int L = kPrivSlots;
   auto a16 = [](const void* q) { return ((uintptr_t)q & 15) == 0; };
   if (sp.g.n < R) return false;
   if (S::PW > 0 && !a16(sp.pcol)) return false;
@@ -732,18 +1067,44 @@ static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t
   for (int i = 0; i < S::NC; ++i)
     if (!a16(sp.col[i])) return false;
   auto fn = k_sga_bulk<S, L, T, R, NS>;
-  const size_t smem = bulk_acc_bytes<S>(L, T) + (size_t)NS * BulkStage<S, R>::BYTES;
-  static DevCache cache;
-  const int nb = cache.get([&]() -> int {
-    if (cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem) != cudaSuccess) return 0;
+  const size_t smem = tier_bytes<S, L>(T, sp.tab_nrep << sp.tab_hb) + (size_t)NS * BulkStage<S, R>::BYTES;
+  // per device: the kernel's dynamic shared-memory attribute, raised to the largest size
+  // launched so far (an attribute far above the need changed the SM's carveout choice and
+  // cost ~15 % on C4); per device and table size: the resident CTAs per SM
+  static DevCache attr;
+  int have = attr.get([&]() -> int { return 0; });
+  if ((int)smem > have) {
+    if (cudaFuncSetAttribute(fn, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem) != cudaSuccess) {
+      cudaGetLastError();
+      return false;
+    }
+    int d = 0;
+    cudaGetDevice(&d);
+    if (d >= 0 && d < kMaxDevices) attr.v[d].store((int)smem, std::memory_order_relaxed);
+  }
+  static DevCache cache[8];
+  int ci = 0;
+  for (uint32_t c = sp.tab_nrep << sp.tab_hb; c > 128 && ci < 7; c >>= 1) ++ci;
+  const int nb = cache[ci].get([&]() -> int {
     int b = 0;
-    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, fn, T + 32, smem) != cudaSuccess || b < 1) b = 0;
+    if (cudaOccupancyMaxActiveBlocksPerMultiprocessor(&b, fn, T + 32, smem) != cudaSuccess || b < 1) {
+      cudaGetLastError();
+      b = 0;
+    }
     return b;
   });
   if (nb < 1) return false;
   int64_t grid = (int64_t)sms * nb;
   const int64_t chunks = sp.g.n / R;
   if (chunks < grid) grid = chunks;
+  if (const char* w = getenv("OCL_WAIT")) {        // "<producer><consumer>" digits, e.g. "10"
+    SpecPlan& q = const_cast<SpecPlan&>(sp);
+    q.pwait = w[0] ? w[0] - '0' : 0;
+    q.cwait = w[0] && w[1] ? w[1] - '0' : 0;
+  }
+  if (getenv("OCL_DEBUG"))
+    fprintf(stderr, "[ocl] k_sga_bulk L=%d T=%d R=%d NS=%d tab=%u x 2^%u smem=%zu blocks/SM=%d grid=%lld\n", L, T,
+            R, NS, sp.tab_nrep, sp.tab_hb, smem, nb, (long long)grid);
   count_launch();
   fn<<<(int)grid, T + 32, smem, s>>>(sp);
   *err = cudaGetLastError();
@@ -765,45 +1126,102 @@ template <class S>
 static bool launch_bulk_cfg(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err) {
   int cfg = bulk_config();
   if (cfg < 0) cfg = S::F64 ? 3 : 7;
+  constexpr int L = kPrivSlots;
   switch (cfg) {
-    case 1: return launch_bulk<S, 256, 1024, 4>(sp, sms, s, err);
-    case 2: return launch_bulk<S, 256, 512, 3>(sp, sms, s, err);
-    case 3: return launch_bulk<S, 256, 512, 2>(sp, sms, s, err);
-    case 4: return launch_bulk<S, 256, 512, 1>(sp, sms, s, err);
-    case 5: return launch_bulk<S, 128, 256, 2>(sp, sms, s, err);
-    case 6: return launch_bulk<S, 128, 256, 3>(sp, sms, s, err);
-    case 7: return launch_bulk<S, 128, 512, 2>(sp, sms, s, err);
+    case 1: return launch_bulk<S, L, 256, 1024, 4>(sp, sms, s, err);
+    case 2: return launch_bulk<S, L, 256, 512, 3>(sp, sms, s, err);
+    case 3: return launch_bulk<S, L, 256, 512, 2>(sp, sms, s, err);
+    case 4: return launch_bulk<S, L, 256, 512, 1>(sp, sms, s, err);
+    case 5: return launch_bulk<S, L, 128, 256, 2>(sp, sms, s, err);
+    case 6: return launch_bulk<S, L, 128, 256, 3>(sp, sms, s, err);
+    case 7: return launch_bulk<S, L, 128, 512, 2>(sp, sms, s, err);
     default: return false;
   }
 }
 
-// Try the specialised low-G kernels; returns false if no signature matches.
-// *kind: 1/2 = k_sga_priv (int / fp64), 3/4 = k_sga_bulk (int / fp64).
+// Few-group signatures (L = 4): the bulk pipeline (*kind + 2), else the register-load
+// kernel (fewer rows than one stage, or OCL_BULK=0).
+template <class S>
+static bool launch_few(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err, int* kind) {
+  if (launch_bulk_cfg<S>(sp, sms, s, err)) {
+    *kind += 2;
+    return true;
+  }
+  const size_t smem = Acc<S>::bytes(kPrivSlots, kPrivThreads);
+  static DevCache cache;
+  const int nb = cache.get([&]() -> int {
+    cudaFuncSetAttribute(k_sga_priv<S, kPrivSlots>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
+    return spec_blocks_per_sm<S>(smem);
+  });
+  int grid = sms * nb;
+  const int64_t tiles = (sp.g.n + 127) / 128;
+  const int64_t need = (tiles + 7) / 8;
+  if (need < grid) grid = (int)(need > 0 ? need : 1);
+  count_launch();
+  k_sga_priv<S, kPrivSlots><<<grid, kPrivThreads, smem, s>>>(sp);
+  *err = cudaGetLastError();
+  return true;
+}
+
+// Group-by signatures: the tier by expected groups — 4 private slots, or the replicated
+// tables (<= kSpecTabMaxGroups groups; replicas = min(consumer warps, 72 KB / table)).
+// false: no tier fits (the caller falls back).
+constexpr int64_t kSpecTabMaxGroups = 2048;
+constexpr size_t kTabBudget = 72 * 1024;   // + 2 stages of 20 KB: 2 CTAs per SM
+
+template <class S>
+static bool launch_grp(SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err, int* tier) {
+  const int64_t eg = sp.g.expected > 0 ? sp.g.expected : 1;
+  if (eg <= 4) { *tier = 1; return launch_bulk<S, 4, 128, 512, 2>(sp, sms, s, err); }
+  if constexpr (S::cta_ok()) {
+    if (eg <= kSpecTabMaxGroups) {
+      constexpr int T = 512;                          // 16 consumer warps: latency hiding at 2 CTAs / SM
+      uint32_t hb = 6;                                // load <= 1/4 up to 256 groups, <= 1/2 above
+      while (((int64_t)1 << hb) < (eg <= 256 ? 4 : 2) * eg) ++hb;
+      const size_t one = ((size_t)1 << hb) * TabL<S>::BYTES_PER_SLOT;
+      size_t nrep = kTabBudget / one;
+      if (nrep > T / 32) nrep = T / 32;
+      if (nrep < 1) nrep = 1;
+      sp.tab_hb = hb;
+      sp.tab_nrep = (uint32_t)nrep;
+      *tier = 4;
+      return launch_bulk<S, 0, T, 1024, 2>(sp, sms, s, err);
+    }
+  }
+  return false;
+}
+
+// Whether a group-by signature kernel takes this plan (the planner then keeps the one-pass
+// fused kernel instead of the hash-partitioned tier).
+bool spec_takes(const Plan& g) {
+  SpecPlan sp;
+  const int64_t eg = g.expected > 0 ? g.expected : 1;
+  if (eg > kSpecTabMaxGroups || getenv("OCL_NO_SPEC")) return false;
+  return spec_match<SigC5>(g, &sp) || spec_match<SigC3>(g, &sp);
+}
+
+// Try the specialised kernels; returns false if no signature matches.  *kind (see
+// fused_kernel_name): 11/12 = k_sga_priv Q1 (int / fp64), 13/14 = k_sga_bulk Q1, 15/16 =
+// k_sga_bulk Q1 + MIN/MAX, 60 + tier = C5 shape, 70 + tier = C3 shape (tier 1 = 4 private
+// slots, 4 = replicated tables).
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind) {
   SpecPlan sp;
-  int64_t tiles = (g.n + 127) / 128;
-  auto go = [&](auto sig) -> bool {
-    using S = decltype(sig);
-    if (launch_bulk_cfg<S>(sp, sms, s, err)) {
-      *kind += 2;
-      return true;
+  const int64_t eg = g.expected > 0 ? g.expected : 1;
+  if (eg <= kPrivSlots) {
+    if (spec_match<SigQ1I>(g, &sp)) { *kind = 11; return launch_few<SigQ1I>(sp, sms, s, err, kind); }
+    if (spec_match<SigQ1F>(g, &sp)) { *kind = 12; return launch_few<SigQ1F>(sp, sms, s, err, kind); }
+    if (spec_match<SigQ1IMM>(g, &sp)) {
+      *kind = 15;
+      return launch_bulk<SigQ1IMM, kPrivSlots, 128, 512, 2>(sp, sms, s, err);
     }
-    const size_t smem = Acc<S>::bytes(kPrivSlots, kPrivThreads);
-    static DevCache cache;
-    const int nb = cache.get([&]() -> int {
-      cudaFuncSetAttribute(k_sga_priv<S, kPrivSlots>, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem);
-      return spec_blocks_per_sm<S>(smem);
-    });
-    int grid = sms * nb;
-    int64_t need = (tiles + 7) / 8;
-    if (need < grid) grid = (int)(need > 0 ? need : 1);
-    count_launch();
-    k_sga_priv<S, kPrivSlots><<<grid, kPrivThreads, smem, s>>>(sp);
-    *err = cudaGetLastError();
-    return true;
-  };
-  if (spec_match<SigQ1I>(g, &sp)) { *kind = 1; return go(SigQ1I{}); }
-  if (spec_match<SigQ1F>(g, &sp)) { *kind = 2; return go(SigQ1F{}); }
+    if (spec_match<SigQ1FMM>(g, &sp)) {
+      *kind = 16;
+      return launch_bulk<SigQ1FMM, kPrivSlots, 256, 512, 2>(sp, sms, s, err);
+    }
+  }
+  int t = 0;
+  if (spec_match<SigC5>(g, &sp) && launch_grp<SigC5>(sp, sms, s, err, &t)) { *kind = 60 + t; return true; }
+  if (spec_match<SigC3>(g, &sp) && launch_grp<SigC3>(sp, sms, s, err, &t)) { *kind = 70 + t; return true; }
   return false;
 }
 

@@ -84,6 +84,8 @@ int reg_tier_slots();
 const char* fused_kernel_name(int kind);
 // Proven few-group Q1 kernel (fused_spec.cu) used while the unified kernel is tuned.
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
+// Whether a plan-signature kernel takes this group-by plan (the planner keeps the one-pass tier).
+bool spec_takes(const Plan& g);
 // High-cardinality tier (partition.cu): hash-partitioned two-pass aggregation.
 bool part_eligible(const Plan& p);
 int part_bits_for(int64_t expected_groups);

@@ -232,8 +232,10 @@ def _q1(li, f64=False):
 def test_fused_q1_int(tier, n):
     li = _lineitem(n, datagen.BASE_SEED + 1)
     p, k, v, a = _q1(li)
+    # tier 1: the Q1 + MIN/MAX signature kernel (the MIN/MAX pair matches it) when n fills a pipeline stage
+    want = ("k_sga_bulk<Sig Q1+MINMAX int64>" if n >= 512 else "k_sga<DynShape>") if tier == 1 else "k_sga_glb"
     _check_sga(p, k, v, a + [{"op": "sum", "a": 2}, {"op": "min", "a": 0}, {"op": "max", "a": 1}], tier=tier,
-               order_by_key=True, bitmap=True, kernel="k_sga<DynShape>" if tier == 1 else "k_sga_glb")
+               order_by_key=True, bitmap=True, kernel=want)
 
 
 @pytest.mark.parametrize("tier", [1, 2])
@@ -241,7 +243,7 @@ def test_fused_q1_f64(tier):
     li = _lineitem(6000000 if tier == 1 else 300000, datagen.BASE_SEED + 2, f64=True)
     p, k, v, a = _q1(li, f64=True)
     _check_sga(p, k, v, a + [{"op": "min", "a": 0}, {"op": "max", "a": 1}], tier=tier,
-               kernel="k_sga<DynShape>" if tier == 1 else "k_sga_glb")
+               kernel="k_sga_bulk<Sig Q1+MINMAX fp64>" if tier == 1 else "k_sga_glb")
 
 
 def test_fused_worked_example():

@@ -117,3 +117,95 @@ def test_spec_all_rows_filtered_and_one_group():
     ls = np.full(n, ord("O"), np.uint8)
     keys, _ = _check_sga(p, [rf, ls], v, a, order_by_key=True, kernel="k_sga_bulk<Sig Q1 int64>")
     assert keys.cpu().numpy().tolist() == [(ord("N") << 8) | ord("O")]
+
+
+# ---------------------------------------------------------------- Q1 + MIN/MAX (bench workload c4mm)
+Q1MM_EXTRA = [{"op": "min", "a": 0}, {"op": "max", "a": 1}]
+
+
+@pytest.mark.parametrize("f64", [False, True])
+@pytest.mark.parametrize("n", [511, 512, 100_003, 3_000_017])
+def test_c4mm_kernel(f64, n):
+    """Q1 + MIN(quantity) + MAX(extendedprice): the signature kernel with MIN/MAX private fields
+    (k_sga_bulk<Sig Q1+MINMAX>); n < 512 falls back to the unified kernel."""
+    li = _lineitem(n, datagen.BASE_SEED + 4, f64=f64)
+    p, k, v, a = _q1_plan(li, f64)
+    want = f"k_sga_bulk<Sig Q1+MINMAX {'fp64' if f64 else 'int64'}>" if n >= 512 else "k_sga<"
+    _check_sga(p, k, v, a + Q1MM_EXTRA, order_by_key=True, kernel=want)
+
+
+def test_c4mm_extremes():
+    """MIN/MAX fields at the int32 range ends (encodings 0 and ~0) and beyond int32 (exact slow path)."""
+    n = 200_000
+    li = _lineitem(n, datagen.BASE_SEED + 4)
+    q, pr = li["quantity"].copy(), li["extendedprice"].copy()
+    q[::1001] = 2**31 - 1
+    q[5::1003] = -(2**31)
+    pr[7::997] = 2**31 - 1
+    pr[9::991] = -(2**31)
+    q[11::5003] = 2**40                                  # beyond int32: HBM entry, exact
+    li.update(quantity=q, extendedprice=pr)
+    p, k, v, a = _q1_plan(li, False)
+    _check_sga(p, k, v, a + Q1MM_EXTRA, order_by_key=True, kernel="k_sga_bulk<Sig Q1+MINMAX int64>")
+
+
+# ---------------------------------------------------------------- C5 / C3 group-by signatures
+C5_AGGS = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+
+
+def _c5_tier(G):
+    return "4 private slots" if G <= 4 else "replicated tables"
+
+
+@pytest.mark.parametrize("G", [4, 16, 32, 64, 256, 1024, 2048])
+@pytest.mark.parametrize("zipf,sel", [(0.0, 10**6), (1.5, 5 * 10**5), (1.0, 10**4)])
+def test_c5_signature_tiers(G, zipf, sel):
+    """The C5 bench plan (WHERE p < T GROUP BY key: COUNT, SUM, MIN, MAX of v) on both accumulation tiers
+    of k_sga_bulk<Sig pred i32, key i64> (private slots, replicated tables with 8 / 4 / 1 replicas), uniform
+    and skewed keys (Zipf 1.5 puts ~38 % of the rows on one key), three selectivities."""
+    n = (1 << 21) + 77
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, G, s=zipf)
+    preds = [(sw["p"], {"hi": sel - 1})]
+    _check_sga(preds, [sw["key"]], [sw["v"]], C5_AGGS, expected_groups=G,
+               kernel=f"k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; {_c5_tier(G)}>")
+
+
+@pytest.mark.parametrize("G", [4, 16, 32, 1000])
+def test_c3_signature_tiers(G):
+    """No predicate (C3 shape): GROUP BY key, COUNT / SUM / MIN / MAX."""
+    n = 1_000_003
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 3, G, s=0.5)
+    _check_sga([], [sw["key"]], [sw["v"]], C5_AGGS, expected_groups=G,
+               kernel=f"k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; {_c5_tier(G)}>")
+
+
+@pytest.mark.parametrize("G,eg", [(40, 4), (100, 32), (3000, 2048), (3, 300)])
+def test_signature_tier_overflow(G, eg):
+    """More distinct keys than the tier holds (expected_groups underestimated): keys beyond the private
+    slots / a full table replica take the exact HBM update; the result is still exact (the HBM table is sized
+    by the restart of select_group_aggregate)."""
+    n = 600_001
+    rng = np.random.default_rng(G)
+    key = ((rng.integers(0, G, n).astype(np.uint64) * np.uint64(0x9E3779B97F4A7C15)) >> np.uint64(2)).astype(np.int64)
+    v = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    p = rng.integers(0, 100, n).astype(np.int32)
+    _check_sga([(p, {"hi": 89})], [key], [v], C5_AGGS, expected_groups=eg,
+               kernel="k_sga_bulk<Sig pred i32, key i64")
+
+
+def test_signature_exact_paths():
+    """C5 shape with values beyond int32 (exact int128 per-row path), the key ~0 (side entry), negative
+    values and int32 extremes, on the private and CTA tiers."""
+    n = 300_007
+    rng = np.random.default_rng(9)
+    for G in (8, 500):
+        key = rng.integers(0, G, n).astype(np.int64) * 7919 - 3
+        key[::97] = -1                                     # ~0
+        v = rng.integers(-2**31, 2**31, n).astype(np.int64)
+        v[::89] = 2**45 + 1
+        v[3::101] = -(2**40)
+        v[5::103] = 2**31 - 1
+        v[7::107] = -(2**31)
+        p = rng.integers(0, 10, n).astype(np.int32)
+        _check_sga([(p, {"lo": 1})], [key], [v], C5_AGGS, expected_groups=G,
+                   kernel="k_sga_bulk<Sig pred i32, key i64")

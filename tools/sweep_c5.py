@@ -35,6 +35,7 @@ def main():
     ap.add_argument("--out", default=os.path.join(ROOT, "profiles", "r01_c5_sweep.json"))
     ap.add_argument("--groups", default="2,4,6,8,10,12,14,16,18,20,22,24", help="log2 G values")
     ap.add_argument("--zipf", default="0,1.0,1.5")
+    ap.add_argument("--sel", default="0.01,0.5,1.0")
     args = ap.parse_args()
     dev = torch.device("cuda", 0)
     peak = json.load(open(os.path.join(ROOT, "MEASURED_PEAKS.json")))["hbm_gbs"] \
@@ -46,7 +47,8 @@ def main():
         for s in [float(x) for x in args.zipf.split(",")]:
             cols = datagen.sweep_device(n, datagen.BASE_SEED + 5, G, s=s, device=dev)
             torch.cuda.synchronize()
-            for T, sel in ((10**4, 0.01), (5 * 10**5, 0.5), (10**6, 1.0)):
+            for sel in [float(x) for x in args.sel.split(",")]:
+                T = int(round(sel * 10**6))
                 call = ocl.SgaCall([(cols["p"], {"hi": T - 1})], [cols["key"]], [cols["v"]], AGGS,
                                    expected_groups=G, out_capacity=max(16, 2 * G))
                 for _ in range(2):
@@ -83,7 +85,8 @@ def main():
                 f"{peak:.0f} GB/s.\n\n")
         f.write("| log2 G | zipf | sel | distinct | ms | G rows/s | HBM frac | path |\n|---|---|---|---|---|---|---|---|\n")
         for r in rows:
-            path = "partitioned" if "part" in r["kernel"] else r["kernel"].split("<")[0]
+            k = r["kernel"]
+            path = "partitioned" if "part" in k else (k.split(";")[1].strip(" >") if ";" in k else k.split("<")[0])
             f.write(f"| {r['log2_groups']} | {r['zipf']} | {r['selectivity']} | {r['distinct_groups']} | "
                     f"{r['ms_median']:.3f} | {r['rows_per_s'] / 1e9:.1f} | {r['hbm_frac']:.3f} | {path} |\n")
 
