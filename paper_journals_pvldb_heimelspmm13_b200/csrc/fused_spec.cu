@@ -445,8 +445,8 @@ __device__ __forceinline__ bool priv_slot(const SpecPlan& p, const DirState<L>& 
   for (int s = L - 1; s >= 0; --s)
     if (x.key == rk[s]) slot = s;
   bool go = x.q && x.fast && slot >= 0 && !special;
-  if (x.q && !go && x.fast && !special) {            // rare: new key in this CTA
-    slot = dir_find_or_insert<L>(d.dir, (uint64_t)x.key);
+  if (x.q && !go) {                                   // rare: new key in this CTA, or slow value
+    slot = (x.fast && !special) ? dir_find_or_insert<L>(d.dir, (uint64_t)x.key) : -1;
     if (slot >= 0) {
 #pragma unroll
       for (int s = 0; s < L; ++s) {
@@ -454,11 +454,10 @@ __device__ __forceinline__ bool priv_slot(const SpecPlan& p, const DirState<L>& 
         rk[s] = sk ? (KeyT<S>)~sk : (KeyT<S>)~0ULL;
       }
       go = true;
+    } else {                                          // slow value, key ~0, or no slot left
+      uint8_t* e = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, (uint64_t)x.key, p.g.status);
+      if (e) update_entry_slow(p.g, e, r);
     }
-  }
-  if (x.q && !go) {                                   // slow value, key ~0, or no slot left
-    uint8_t* e = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, (uint64_t)x.key, p.g.status);
-    if (e) update_entry_slow(p.g, e, r);
   }
   return go;
 }
@@ -1041,7 +1040,7 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
   for (int i = 0; i < 4; ++i) sp->col[i] = i < nc ? cols[i] : nullptr;
   sp->tab_hb = 0;
   sp->tab_nrep = 0;
-  sp->pwait = 1;
+  sp->pwait = 0;
   sp->cwait = 0;
   return true;
 }
