@@ -40,3 +40,15 @@ clean:
 	rm -f $(LIB) oracle/liboracle.so datagen/liboclgen_host.so datagen/liboclgen_dev.so
 
 .PHONY: all clean
+
+# compute-sanitizer over one small call of every kernel family (tools/sanitize_cases.py checks each
+# result against the oracle); needs a GPU.  Logs: profiles/sanitize_<tool>.log
+SANITIZER ?= /usr/local/cuda/bin/compute-sanitizer
+sanitize: all
+	@for t in memcheck racecheck synccheck; do \
+	  echo "== $$t"; \
+	  $(SANITIZER) --tool $$t --error-exitcode 1 --print-limit 20 python tools/sanitize_cases.py $(CASES) \
+	    > profiles/sanitize_$$t.log 2>&1; echo "rc=$$?"; tail -3 profiles/sanitize_$$t.log; \
+	done
+
+.PHONY: sanitize

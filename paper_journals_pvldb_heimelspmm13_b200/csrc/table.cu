@@ -293,8 +293,11 @@ __global__ void __launch_bounds__(256) k_group_build(const __grid_constant__ Pla
             g = (int64_t)v - 1;
           }
           gid = (int32_t)g;
+          // publish key -> gid in the CTA cache; a reader that sees the key before the gid
+          // still reads -1 and takes the miss path (correct, just not cached).  The gid is
+          // written with an atomic so the publication is race-free (compute-sanitizer racecheck)
           if (key[k] != ~0ULL && atomicCAS(&ck[h], 0ULL, (unsigned long long)~key[k]) == 0ULL)
-            *(volatile int32_t*)&cs[h] = gid;
+            atomicExch(&cs[h], gid);
         }
         gid = __shfl_sync(peers, gid, leader);
       }
