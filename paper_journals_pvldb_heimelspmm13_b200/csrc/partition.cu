@@ -553,25 +553,84 @@ __device__ __forceinline__ void update_entry_rec(const Plan& p, uint8_t* e, cons
   }
 }
 
-// A whole warp of records with the same key (heavy hitters): one combined update.
-template <int NV>
-__device__ __forceinline__ void cta_add_warp(const Plan& p, uint8_t* e, const int32_t (&v)[NV > 0 ? NV : 1], int lane) {
-  if (lane == 0) atomicAdd((unsigned int*)(e + 8), 32u);
+// ---- the pass-2 shared table, field-major: keys u64[kPartCap] (~key, 0 = empty), then one
+// u32[kPartCap] array per 4-byte field of the CTA-table entry layout the planner assigned
+// (count at entry offset 8, per value sum lo / hi, MIN, MAX at d.co_*): entry offset co ->
+// array (co - 8) / 4.  Lanes of an atomic instruction on different slots then hit different
+// banks (an AoS entry of 32 bytes put every entry's count field in 4 of the 32 banks:
+// ~16 wavefronts per atomic instruction on C3).  SUM: the biased sum of (x + 2^31) as a
+// 64-bit {lo, hi} pair; lo is added atomically and the carry out of it (seen in the value
+// the atomic returns) is added to hi, so one atomic per row (exact: sum = biased - count * 2^31).
+__device__ __forceinline__ int32_t dec32_max(uint32_t e) { return (int32_t)(e ^ 0x80000000u); }
+__device__ __forceinline__ int32_t dec32_min(uint32_t e) { return dec32_max(~e); }
+__device__ __forceinline__ uint64_t* pkey(uint8_t* tab, int slot) { return (uint64_t*)tab + slot; }
+__device__ __forceinline__ uint32_t* pf32(uint8_t* tab, int slot, int co) {
+  return (uint32_t*)(tab + 8 * (size_t)kPartCap + (size_t)kPartCap * (co - 8)) + slot;
+}
+__device__ __forceinline__ const uint32_t* pf32(const uint8_t* tab, int slot, int co) {
+  return (const uint32_t*)(tab + 8 * (size_t)kPartCap + (size_t)kPartCap * (co - 8)) + slot;
+}
+__device__ __forceinline__ int64_t part_sum(const uint8_t* tab, int slot, int co_lo, uint32_t cnt) {
+  const uint64_t b = (uint64_t)*pf32(tab, slot, co_lo) | ((uint64_t)*pf32(tab, slot, co_lo + 4) << 32);
+  return (int64_t)(b - ((uint64_t)cnt << 31));
+}
+__device__ __forceinline__ void part_add_sum(uint8_t* tab, int slot, int co_lo, uint64_t biased) {
+  const uint32_t a = (uint32_t)biased, hi = (uint32_t)(biased >> 32);
+  const uint32_t old = atomicAdd(pf32(tab, slot, co_lo), a);
+  const uint32_t c = hi + (uint32_t)(old + a < old);
+  if (c) atomicAdd(pf32(tab, slot, co_lo + 4), c);
+}
+
+// Field offsets of value i: from the plan, or (FIX: one value with SUM, MIN and MAX — the
+// C3 / C5 plans) the compile-time layout co_lo 12, co_hi 16, co_min 20, co_max 24, which
+// removes the per-record constant-bank loads and flag branches.
+template <bool FIX>
+__device__ __forceinline__ void part_cos(const Plan& p, int i, int& lo, int& mn, int& mx) {
+  if constexpr (FIX) {
+    lo = 12;
+    mn = 20;
+    mx = 24;
+  } else {
+    lo = p.vals[i].co_lo;
+    mn = p.vals[i].co_min;
+    mx = p.vals[i].co_max;
+  }
+}
+
+// One record into slot `slot`.
+template <int NV, bool FIX>
+__device__ __forceinline__ void part_add(const Plan& p, uint8_t* tab, int slot, const int32_t (&v)[NV > 0 ? NV : 1]) {
+  atomicAdd(pf32(tab, slot, 8), 1u);
 #pragma unroll
   for (int i = 0; i < NV; ++i) {
-    if (i >= p.nvals) break;
-    const DevValue& d = p.vals[i];
-    const uint32_t lo = __reduce_add_sync(0xffffffffu, (uint32_t)v[i] & 0xFFFFu);
-    const int32_t hi = (int32_t)__reduce_add_sync(0xffffffffu, (uint32_t)(v[i] >> 16));
+    if (!FIX && i >= p.nvals) break;
+    int lo, mn, mx;
+    part_cos<FIX>(p, i, lo, mn, mx);
+    if (lo >= 0) part_add_sum(tab, slot, lo, (uint64_t)((uint32_t)v[i] ^ 0x80000000u));
+    if (mn >= 0) atomicMax(pf32(tab, slot, mn), enc32_min(v[i]));
+    if (mx >= 0) atomicMax(pf32(tab, slot, mx), enc32_max(v[i]));
+  }
+}
+
+// A whole warp of records with the same key (heavy hitters): one combined update.
+template <int NV, bool FIX>
+__device__ __forceinline__ void part_add_warp(const Plan& p, uint8_t* tab, int slot, const int32_t (&v)[NV > 0 ? NV : 1],
+                                              int lane) {
+  if (lane == 0) atomicAdd(pf32(tab, slot, 8), 32u);
+#pragma unroll
+  for (int i = 0; i < NV; ++i) {
+    if (!FIX && i >= p.nvals) break;
+    int clo, cmn, cmx;
+    part_cos<FIX>(p, i, clo, cmn, cmx);
+    const uint32_t b = (uint32_t)v[i] ^ 0x80000000u;
+    const uint32_t lo = __reduce_add_sync(0xffffffffu, b & 0xFFFFu);
+    const uint32_t hi = __reduce_add_sync(0xffffffffu, b >> 16);
     const int32_t mn = __reduce_min_sync(0xffffffffu, v[i]);
     const int32_t mx = __reduce_max_sync(0xffffffffu, v[i]);
     if (lane == 0) {
-      if (d.co_lo >= 0) {
-        atomicAdd((unsigned int*)(e + d.co_lo), lo);
-        atomicAdd((int*)(e + d.co_hi), hi);
-      }
-      if (d.co_min >= 0) atomicMax((unsigned int*)(e + d.co_min), enc32_min(mn));
-      if (d.co_max >= 0) atomicMax((unsigned int*)(e + d.co_max), enc32_max(mx));
+      if (clo >= 0) part_add_sum(tab, slot, clo, (uint64_t)lo + ((uint64_t)hi << 16));
+      if (cmn >= 0) atomicMax(pf32(tab, slot, cmn), enc32_min(mn));
+      if (cmx >= 0) atomicMax(pf32(tab, slot, cmx), enc32_max(mx));
     }
   }
 }
@@ -589,14 +648,35 @@ __global__ void k_part_items(PartArgs a) {
   a.icnt[q] = (uint32_t)((n + kPartItem - 1) / kPartItem);
 }
 
-// Merge a shared-table entry into the HBM table when this CTA is the only one
-// aggregating its partition (a one-item partition): plain read-modify-write of the
-// entry's fields — no other thread updates them (the scatter's exact path and this
-// CTA's own overflow updates happened before the barrier).  The slot is still
-// claimed with atomicCAS: linear probing may run into a neighbour partition's range.
-__device__ __forceinline__ void cta_flush_entry_excl(const Plan& p, const uint8_t* ce) {
-  const uint64_t sk = *(const uint64_t*)ce;
-  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+// Merge shared slot `slot` into the HBM table (atomics: other CTAs share the partition).
+__device__ __forceinline__ void part_flush_slot(const Plan& p, const uint8_t* tab, int slot) {
+  const uint64_t sk = *pkey((uint8_t*)tab, slot);
+  const uint32_t cnt = *pf32(tab, slot, 8);
+  if (sk == 0 || cnt == 0) return;
+  uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
+  if (!e) return;
+  atomicAdd((unsigned long long*)(e + 8), (unsigned long long)cnt);
+  for (int v = 0; v < p.nvals; ++v) {
+    const DevValue& d = p.vals[v];
+    if (d.co_lo >= 0) {
+      const int64_t sum = part_sum(tab, slot, d.co_lo, cnt);
+      atomic_add_i128((uint64_t*)(e + d.off_sum), (uint64_t)sum, (uint64_t)(sum >> 63));
+    }
+    if (d.co_min >= 0)
+      atomicMax((unsigned long long*)(e + d.off_min), (unsigned long long)enc_min_i(dec32_min(*pf32(tab, slot, d.co_min))));
+    if (d.co_max >= 0)
+      atomicMax((unsigned long long*)(e + d.off_max), (unsigned long long)enc_max_i(dec32_max(*pf32(tab, slot, d.co_max))));
+  }
+}
+
+// Merge a shared slot into the HBM table when this CTA is the only one aggregating its
+// partition (a one-item partition): plain read-modify-write of the entry's fields — no
+// other thread updates them (the scatter's exact path and this CTA's own overflow updates
+// happened before the barrier).  The slot is still claimed with atomicCAS: linear probing
+// may run into a neighbour partition's range.
+__device__ __forceinline__ void part_flush_slot_excl(const Plan& p, const uint8_t* tab, int slot) {
+  const uint64_t sk = *pkey((uint8_t*)tab, slot);
+  const uint32_t cnt = *pf32(tab, slot, 8);
   if (sk == 0 || cnt == 0) return;
   uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, ~sk, p.status);
   if (!e) return;
@@ -604,80 +684,75 @@ __device__ __forceinline__ void cta_flush_entry_excl(const Plan& p, const uint8_
   for (int v = 0; v < p.nvals; ++v) {
     const DevValue& d = p.vals[v];
     if (d.co_lo >= 0) {
-      const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
       I128 x{*(const uint64_t*)(e + d.off_sum), *(const uint64_t*)(e + d.off_sum + 8)};
-      x = i128_add(x, i128_from_i64(sum));
+      x = i128_add(x, i128_from_i64(part_sum(tab, slot, d.co_lo, cnt)));
       *(uint64_t*)(e + d.off_sum) = x.lo;
       *(uint64_t*)(e + d.off_sum + 8) = x.hi;
     }
     if (d.co_min >= 0) {
-      const int32_t mn = (int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u);
       uint64_t* f = (uint64_t*)(e + d.off_min);
-      *f = max(*f, enc_min_i(mn));
+      *f = max(*f, enc_min_i(dec32_min(*pf32(tab, slot, d.co_min))));
     }
     if (d.co_max >= 0) {
-      const int32_t mx = (int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u);
       uint64_t* f = (uint64_t*)(e + d.off_max);
-      *f = max(*f, enc_max_i(mx));
+      *f = max(*f, enc_max_i(dec32_max(*pf32(tab, slot, d.co_max))));
     }
   }
 }
 
-// Shared-table find-or-insert for pass 2.  In direct mode the start slot and the
-// linear probing (wrapping inside the table) mirror the key's slot range in the HBM
-// table — the table's start slot is the top log2(cap) hash bits and a partition's
-// range has exactly kPartCap slots — so the entries can be stored to the HBM table
-// position by position, without probing it.
+// Shared-table find-or-insert for pass 2 -> slot, or -1 (probe limit).  In direct mode the
+// start slot and the linear probing (wrapping inside the table) mirror the key's slot range
+// in the HBM table — the table's start slot is the top log2(cap) hash bits and a partition's
+// range has exactly kPartCap slots — so the entries can be stored to the HBM table position
+// by position, without probing it.
 constexpr int kPartProbes = 64;
 
-__device__ __forceinline__ uint8_t* part_find(uint8_t* tab, int32_t cs, uint64_t key, bool direct, int pbits) {
+__device__ __forceinline__ int part_find(uint8_t* tab, uint64_t key, bool direct, int pbits) {
   const uint64_t sk = ~key;
   const uint64_t h = fmix64(key);
   uint32_t i = direct ? (uint32_t)((h << pbits) >> (64 - kPartCapBits)) : (uint32_t)h & (kPartCap - 1);
   for (int probe = 0; probe < kPartProbes; ++probe) {
-    uint64_t* kp = (uint64_t*)(tab + (size_t)i * cs);
+    uint64_t* kp = pkey(tab, (int)i);
     const uint64_t cur = *(volatile uint64_t*)kp;
-    if (cur == sk) return (uint8_t*)kp;
+    if (cur == sk) return (int)i;
     if (cur == 0) {
       const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
-      if (prev == 0 || prev == sk) return (uint8_t*)kp;
+      if (prev == 0 || prev == sk) return (int)i;
     }
     i = (i + 1) & (kPartCap - 1);
   }
-  return nullptr;
+  return -1;
 }
 
-// Direct merge: shared entry i -> HBM slot region + i (the region holds no entries yet).
-__device__ __forceinline__ void cta_store_entry(const Plan& p, const uint8_t* ce, uint8_t* e) {
-  const uint64_t sk = *(const uint64_t*)ce;
-  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+// Direct merge: shared slot -> HBM slot region + slot (the region holds no entries yet).
+__device__ __forceinline__ void part_store_slot(const Plan& p, const uint8_t* tab, int slot, uint8_t* e) {
+  const uint64_t sk = *pkey((uint8_t*)tab, slot);
+  const uint32_t cnt = *pf32(tab, slot, 8);
   if (sk == 0 || cnt == 0) return;
   *(uint64_t*)e = sk;
   *(uint64_t*)(e + 8) = cnt;
   for (int v = 0; v < p.nvals; ++v) {
     const DevValue& d = p.vals[v];
     if (d.co_lo >= 0) {
-      const int64_t sum = (int64_t)(*(const int32_t*)(ce + d.co_hi)) * 65536 + (int64_t)(*(const uint32_t*)(ce + d.co_lo));
+      const int64_t sum = part_sum(tab, slot, d.co_lo, cnt);
       *(uint64_t*)(e + d.off_sum) = (uint64_t)sum;
       *(uint64_t*)(e + d.off_sum + 8) = (uint64_t)(sum >> 63);
     }
-    if (d.co_min >= 0)
-      *(uint64_t*)(e + d.off_min) = enc_min_i((int32_t)(~*(const uint32_t*)(ce + d.co_min) ^ 0x80000000u));
-    if (d.co_max >= 0)
-      *(uint64_t*)(e + d.off_max) = enc_max_i((int32_t)(*(const uint32_t*)(ce + d.co_max) ^ 0x80000000u));
+    if (d.co_min >= 0) *(uint64_t*)(e + d.off_min) = enc_min_i(dec32_min(*pf32(tab, slot, d.co_min)));
+    if (d.co_max >= 0) *(uint64_t*)(e + d.off_max) = enc_max_i(dec32_max(*pf32(tab, slot, d.co_max)));
   }
 }
 
-// One output row from a CTA-table entry (32-bit fields: count, 16-bit split sums, enc32
-// MIN / MAX): final values or a partial row in the table-entry layout.
-__device__ __forceinline__ void cta_emit_row(const Plan& p, const PartArgs& a, const EmitArgs& ea, const uint8_t* ce,
-                                             int64_t g) {
-  const uint64_t key = ~*(const uint64_t*)ce;
-  const uint32_t cnt = *(const uint32_t*)(ce + 8);
+// One output row from a shared slot: final values or a partial row in the
+// table-entry layout.
+__device__ __forceinline__ void part_emit_row(const Plan& p, const PartArgs& a, const EmitArgs& ea, const uint8_t* tab,
+                                              int slot, int64_t g) {
+  const uint64_t key = ~*pkey((uint8_t*)tab, slot);
+  const uint32_t cnt = *pf32(tab, slot, 8);
   if (ea.kind != EMIT_FINAL) {
     if (g >= ea.out_capacity) return;
     uint8_t* row = ea.partial_out + g * (int64_t)p.stride;
-    cta_store_entry(p, ce, row);
+    part_store_slot(p, tab, slot, row);
     *(uint64_t*)row = key;
     return;
   }
@@ -685,26 +760,25 @@ __device__ __forceinline__ void cta_emit_row(const Plan& p, const PartArgs& a, c
   if (g >= f.out_capacity) return;
   if (f.keys_out) f.keys_out[g] = (int64_t)key;
   for (int i = 0; i < a.npo; ++i) {
-    const int kind = a.po[i].kind, f0 = a.po[i].f0, f1 = a.po[i].f1;
+    const int kind = a.po[i].kind, f0 = a.po[i].f0;
     void* out = a.po[i].out;
     if (kind == 0) {
       ((int64_t*)out)[g] = cnt;
     } else if (kind <= 2) {
-      const int64_t sum = (int64_t)(*(const int32_t*)(ce + f1)) * 65536 + (int64_t)(*(const uint32_t*)(ce + f0));
+      const int64_t sum = part_sum(tab, slot, f0, cnt);
       if (kind == 1) ((ulonglong2*)out)[g] = make_ulonglong2((uint64_t)sum, (uint64_t)(sum >> 63));
       else ((double*)out)[g] = __ddiv_rn(__ll2double_rn(sum), __ull2double_rn(cnt));
     } else if (kind == 3) {
-      ((int64_t*)out)[g] = (int32_t)(~*(const uint32_t*)(ce + f0) ^ 0x80000000u);
+      ((int64_t*)out)[g] = dec32_min(*pf32(tab, slot, f0));
     } else {
-      ((int64_t*)out)[g] = (int32_t)(*(const uint32_t*)(ce + f0) ^ 0x80000000u);
+      ((int64_t*)out)[g] = dec32_max(*pf32(tab, slot, f0));
     }
   }
 }
 
-template <int NV>
-__global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
-                                                           const __grid_constant__ EmitArgs ea) {
-  using Sh = DynShape;
+template <int NV, bool FIX>
+__global__ void __launch_bounds__(kPartThreads, 2) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
+                                                              const __grid_constant__ EmitArgs ea) {
   extern __shared__ __align__(16) uint8_t tab[];
   __shared__ int overflowed;
   __shared__ uint32_t wsum[kPartThreads / 32];
@@ -716,8 +790,9 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
   const int64_t P = 1LL << a.pbits;
   const int cs = p.cta_stride;
   for (int64_t item = blockIdx.x; item < nitems; item += gridDim.x) {
-    // the partition of this item: the largest q with ioff[q] <= item
-    int64_t lo = 0, hi = P - 1;
+    // the partition of this item: the largest q with ioff[q] <= item (= item when no
+    // partition is split into several items)
+    int64_t lo = nitems == P ? item : 0, hi = nitems == P ? item : P - 1;
     while (lo < hi) {
       const int64_t mid = (lo + hi + 1) >> 1;
       if ((int64_t)a.ioff[mid] <= item) lo = mid;
@@ -748,22 +823,16 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
       for (int k = 0; k < kPartILP; ++k) {
         const uint64_t k0 = __shfl_sync(0xffffffffu, key[k], 0);
         if (__all_sync(0xffffffffu, valid[k] && key[k] == k0)) {    // heavy hitter: one update per warp
-          uint8_t* te = lane == 0 ? part_find(tab, cs, k0, direct, a.pbits) : nullptr;
-          const unsigned long long tp = __shfl_sync(0xffffffffu, (unsigned long long)te, 0);
-          if (tp) {
-            cta_add_warp<NV>(p, (uint8_t*)tp, v[k], lane);
+          const int ts = __shfl_sync(0xffffffffu, lane == 0 ? part_find(tab, k0, direct, a.pbits) : -1, 0);
+          if (ts >= 0) {
+            part_add_warp<NV, FIX>(p, tab, ts, v[k], lane);
             continue;
           }
         }
         if (!valid[k]) continue;
-        uint8_t* te = part_find(tab, cs, key[k], direct, a.pbits);
-        if (te) {
-          Row<Sh, NV, false> x;
-          x.q = x.fast = true;
-          x.key = key[k];
-#pragma unroll
-          for (int i = 0; i < NV; ++i) x.vi[i] = v[k][i];
-          cta_add<Sh, NV, false>(p, te, x);
+        const int ts = part_find(tab, key[k], direct, a.pbits);
+        if (ts >= 0) {
+          part_add<NV, FIX>(p, tab, ts, v[k]);
         } else {
           overflowed = 1;
           uint8_t* ge = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
@@ -777,8 +846,8 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
       uint32_t occ = 0;
 #pragma unroll
       for (int k = 0; k < PER; ++k) {
-        const uint8_t* ce = tab + (size_t)(threadIdx.x + k * kPartThreads) * cs;
-        if (*(const uint64_t*)ce != 0 && *(const uint32_t*)(ce + 8) != 0) occ |= 1u << k;
+        const int slot = threadIdx.x + k * kPartThreads;
+        if (*pkey(tab, slot) != 0 && *pf32(tab, slot, 8) != 0) occ |= 1u << k;
       }
       // occupied slots listed in shared memory, then emitted by consecutive threads into
       // consecutive output rows (coalesced stores)
@@ -791,18 +860,15 @@ __global__ void __launch_bounds__(kPartThreads) k_part_agg(const __grid_constant
       uint32_t tot = 0;
       for (int w = 0; w < kPartThreads / 32; ++w) tot += wsum[w];
       __syncthreads();
-      for (uint32_t i = threadIdx.x; i < tot; i += kPartThreads) {
-        const uint8_t* ce = tab + (size_t)slot_list[i] * cs;
-        cta_emit_row(p, a, ea, ce, (int64_t)base_s + i);
-      }
+      for (uint32_t i = threadIdx.x; i < tot; i += kPartThreads)
+        part_emit_row(p, a, ea, tab, slot_list[i], (int64_t)base_s + i);
     } else if (direct && !overflowed) {
       uint8_t* region = p.table + ((size_t)lo << kPartCapBits) * p.stride;
-      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x)
-        cta_store_entry(p, tab + (size_t)i * cs, region + (size_t)i * p.stride);
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) part_store_slot(p, tab, i, region + (size_t)i * p.stride);
     } else if (exclusive) {
-      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry_excl(p, tab + (size_t)i * cs);
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) part_flush_slot_excl(p, tab, i);
     } else {
-      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) cta_flush_entry(p, tab + (size_t)i * cs);
+      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) part_flush_slot(p, tab, i);
     }
     if (a.direct_emit && !(direct && !overflowed) && threadIdx.x == 0) a.dirty[lo] = 1;   // rows in the HBM range
     __syncthreads();
@@ -883,7 +949,9 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   const size_t hsm = (size_t)4 << a.pbits;
   auto kc = k_part_count<Sh, NV>;
   auto ks = k_part_scatter<Sh, NV>;
-  auto ka = k_part_agg<NV>;
+  const bool fix = NV == 1 && p.nvals == 1 && p.vals[0].co_lo == 12 && p.vals[0].co_hi == 16 &&
+                   p.vals[0].co_min == 20 && p.vals[0].co_max == 24;
+  auto ka = fix ? k_part_agg<NV, NV == 1> : k_part_agg<NV, false>;
   cudaError_t e;
   if ((e = cudaFuncSetAttribute(kc, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)hsm))) return e;
   const size_t tsm = (size_t)kPartCap * p.cta_stride;
