@@ -1122,9 +1122,9 @@ static int bulk_config() {
 }
 
 template <class S>
-static bool launch_bulk_cfg(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err) {
+static bool launch_bulk_cfg(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err, int dflt = -1) {
   int cfg = bulk_config();
-  if (cfg < 0) cfg = S::F64 ? 3 : 7;
+  if (cfg < 0) cfg = dflt >= 0 ? dflt : (S::F64 ? 3 : 7);
   constexpr int L = kPrivSlots;
   switch (cfg) {
     case 1: return launch_bulk<S, L, 256, 1024, 4>(sp, sms, s, err);
@@ -1210,12 +1210,12 @@ bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err,
     if (spec_match<SigQ1I>(g, &sp)) { *kind = 11; return launch_few<SigQ1I>(sp, sms, s, err, kind); }
     if (spec_match<SigQ1F>(g, &sp)) { *kind = 12; return launch_few<SigQ1F>(sp, sms, s, err, kind); }
     if (spec_match<SigQ1IMM>(g, &sp)) {
-      *kind = 15;
-      return launch_bulk<SigQ1IMM, kPrivSlots, 128, 512, 2>(sp, sms, s, err);
+      *kind = 15;                           // <128, 256, 3>: 4.19 -> 4.07 ms on c4mm (vs <128, 512, 2>)
+      return launch_bulk_cfg<SigQ1IMM>(sp, sms, s, err, 6);
     }
     if (spec_match<SigQ1FMM>(g, &sp)) {
       *kind = 16;
-      return launch_bulk<SigQ1FMM, kPrivSlots, 256, 512, 2>(sp, sms, s, err);
+      return launch_bulk_cfg<SigQ1FMM>(sp, sms, s, err);
     }
   }
   int t = 0;
