@@ -124,13 +124,15 @@ Q1MM_EXTRA = [{"op": "min", "a": 0}, {"op": "max", "a": 1}]
 
 
 @pytest.mark.parametrize("f64", [False, True])
-@pytest.mark.parametrize("n", [511, 512, 100_003, 3_000_017])
+@pytest.mark.parametrize("n", [255, 511, 512, 100_003, 3_000_017])
 def test_c4mm_kernel(f64, n):
     """Q1 + MIN(quantity) + MAX(extendedprice): the signature kernel with MIN/MAX private fields
-    (k_sga_bulk<Sig Q1+MINMAX>); n < 512 falls back to the unified kernel."""
+    (k_sga_bulk<Sig Q1+MINMAX>; int64 on a 256-row stage ring, fp64 on 512); smaller inputs fall back to
+    the unified kernel."""
     li = _lineitem(n, datagen.BASE_SEED + 4, f64=f64)
     p, k, v, a = _q1_plan(li, f64)
-    want = f"k_sga_bulk<Sig Q1+MINMAX {'fp64' if f64 else 'int64'}>" if n >= 512 else "k_sga<"
+    stage = 512 if f64 else 256
+    want = f"k_sga_bulk<Sig Q1+MINMAX {'fp64' if f64 else 'int64'}>" if n >= stage else "k_sga<"
     _check_sga(p, k, v, a + Q1MM_EXTRA, order_by_key=True, kernel=want)
 
 
