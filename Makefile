@@ -19,6 +19,16 @@ $(OBJDIR)/%.o: $(PKG)/csrc/%.cu $(CHDR)
 	@mkdir -p $(OBJDIR)
 	$(NVCC) $(NVFLAGS) -Iinclude -c -o $@ $< 2> $(OBJDIR)/$*.ptxas.log || (cat $(OBJDIR)/$*.ptxas.log; exit 1)
 
+# NVRTC sources of the run-time specialised kernels (jit.cu): the device headers as strings
+JITHDR    := $(PKG)/csrc/spec_device.cuh $(PKG)/csrc/bulk.cuh $(PKG)/csrc/rowops.cuh $(PKG)/csrc/common.cuh include/ocelot_b200.h
+$(OBJDIR)/jit_src.inc: $(JITHDR) tools/embed_src.py
+	@mkdir -p $(OBJDIR)
+	python3 tools/embed_src.py $@ $(JITHDR)
+
+$(OBJDIR)/jit.o: $(PKG)/csrc/jit.cu $(CHDR) $(OBJDIR)/jit_src.inc
+	@mkdir -p $(OBJDIR)
+	$(NVCC) $(NVFLAGS) -Iinclude -I$(OBJDIR) -c -o $@ $< 2> $(OBJDIR)/jit.ptxas.log || (cat $(OBJDIR)/jit.ptxas.log; exit 1)
+
 $(LIB): $(COBJ)
 	@mkdir -p $(PKG)/_lib
 	$(NVCC) $(ARCH) -shared -o $@ $(COBJ) -lcudart -ldl

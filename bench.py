@@ -345,6 +345,9 @@ def main():
     ap.add_argument("--dist", action="store_true",
                     help="1 GPU: run the distributed path (partial -> NCCL exchange -> merge in the library) on a "
                          "world-size-1 communicator, to measure its overhead (always on for N > 1)")
+    ap.add_argument("--jit", action="store_true",
+                    help="run the plan through the run-time compiled (NVRTC) signature kernel even when a "
+                         "compiled-in signature matches (the path every other plan of the family takes)")
     ap.add_argument("--dist-mode", default="auto", choices=["auto", "allgather", "alltoall"],
                     help="exchange of the distributed path (auto: allgather for partial tables <= 1 MB)")
     args = ap.parse_args()
@@ -355,6 +358,8 @@ def main():
     if wl["kind"] == "sweep":
         wl.update(groups=args.c5_groups, zipf=args.c5_zipf, threshold=max(1, int(round(args.c5_sel * 10**6))))
         wl["desc"] += f" [G={args.c5_groups}, zipf={args.c5_zipf}, selectivity={args.c5_sel}]"
+    if args.jit:
+        os.environ["OCL_JIT_ALL"] = "1"
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))

@@ -2,7 +2,9 @@
 // libocelot_b200.so (sm_100a only).  Nothing here is shared with the oracle.
 #pragma once
 
+#ifndef __CUDACC_RTC__   // NVRTC (jit.cu) compiles the device headers without the runtime headers
 #include <cuda_runtime.h>
+#endif
 #include <stdint.h>
 
 #include "ocelot_b200.h"

@@ -347,7 +347,9 @@ cudaError_t launch_fused(const Plan& p, int mode, bool values_f64, int sms, cuda
   }
   if (mode == 0 && p.vec_ok && getenv("OCL_NO_SPEC") == nullptr) {
     cudaError_t err = cudaSuccess;
-    if (launch_fused_spec(p, sms, s, &err, kind)) return err;   // plan-signature kernels (fused_spec.cu)
+    const bool aot = getenv("OCL_JIT_ALL") == nullptr;           // (A/B: every signature through NVRTC)
+    if (aot && launch_fused_spec(p, sms, s, &err, kind)) return err;   // plan-signature kernels (fused_spec.cu)
+    if (launch_fused_jit(p, sms, s, &err, kind)) return err;    // the same kernels compiled for this plan (jit.cu)
     *kind = 0;
   }
   if ((mode == 0 || mode == 3) && p.vec_ok) {
@@ -386,6 +388,8 @@ const char* fused_kernel_name(int kind) {
     case 61: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
     case 64: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; replicated tables>";
     case 71: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
+    case 90: return "k_sga_bulk<Sig of the plan, run-time compiled (NVRTC); 4 private slots>";
+    case 91: return "k_sga_bulk<Sig of the plan, run-time compiled (NVRTC); replicated tables>";
     case 74: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; replicated tables>";
     case 20: return "k_sga_glb<DynShape>";
     case 30: return "k_part_count/scatter/agg<DynShape> (hash-partitioned)";

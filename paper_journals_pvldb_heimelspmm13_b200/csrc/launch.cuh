@@ -86,6 +86,8 @@ const char* fused_kernel_name(int kind);
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 // Whether a plan-signature kernel takes this group-by plan (the planner keeps the one-pass tier).
 bool spec_takes(const Plan& g);
+// The signature kernels compiled at run time for a plan no compiled-in signature matches (jit.cu).
+bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 // High-cardinality tier (partition.cu): hash-partitioned two-pass aggregation.
 bool part_eligible(const Plan& p);
 int part_bits_for(int64_t expected_groups);

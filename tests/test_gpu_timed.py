@@ -211,3 +211,55 @@ def test_signature_exact_paths():
         p = rng.integers(0, 10, n).astype(np.int32)
         _check_sga([(p, {"lo": 1})], [key], [v], C5_AGGS, expected_groups=G,
                    kernel="k_sga_bulk<Sig pred i32, key i64")
+
+
+# ---------------------------------------------------------------- run-time compiled signatures (jit.cu)
+JIT = "run-time compiled (NVRTC)"
+
+
+@pytest.mark.parametrize("case", ["q1_one_key", "q1_minmax_other", "q1_f64_max", "two_values_tables",
+                                  "i64_pred_tables", "no_pred_u8_key"])
+def test_jit_signatures(case):
+    """Plans no compiled-in signature matches get the same bulk kernel compiled by NVRTC for their
+    signature (Ocelot's run-time kernel compilation): parity with the oracle and the
+    kernel that ran."""
+    n = 700_001
+    li = _lineitem(n, datagen.BASE_SEED + 4, f64=True)
+    vi = [li["quantity"], li["extendedprice"], li["discount"], li["tax"]]
+    vf = [li["quantity_f"], li["extendedprice_f"], li["discount_f"], li["tax_f"]]
+    pred = [(li["shipdate"], {"hi": 10471})]
+    if case == "q1_one_key":             # GROUP BY l_returnflag only (3 groups)
+        _check_sga(pred, [li["returnflag"]], vi, Q1_AGGS, expected_groups=4, order_by_key=True,
+                   kernel=f"{JIT}; 4 private slots")
+    elif case == "q1_minmax_other":      # Q1 + MIN(tax) + MAX(discount)
+        _check_sga(pred, [li["returnflag"], li["linestatus"]], vi,
+                   Q1_AGGS + [{"op": "min", "a": 3}, {"op": "max", "a": 2}], expected_groups=4,
+                   order_by_key=True, kernel=f"{JIT}; 4 private slots")
+    elif case == "q1_f64_max":           # fp64 Q1 + MAX(tax)
+        _check_sga(pred, [li["returnflag"], li["linestatus"]], vf, Q1_AGGS_F64 + [{"op": "max", "a": 3}],
+                   expected_groups=4, order_by_key=True, kernel=f"{JIT}; 4 private slots")
+    elif case == "two_values_tables":    # C5-like with two value columns: replicated tables
+        sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, 300, s=1.0)
+        v2 = (sw["v"] * 3 - 7).astype(np.int64)
+        aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "max", "a": 1}, {"op": "min", "a": 1}]
+        _check_sga([(sw["p"], {"hi": 799_999})], [sw["key"]], [sw["v"], v2], aggs, expected_groups=300,
+                   kernel=f"{JIT}; replicated tables")
+    elif case == "i64_pred_tables":      # predicate on an int64 column, u8 x u8 keys, 12 groups
+        rng = np.random.default_rng(4)
+        k1, k2 = rng.integers(0, 4, n).astype(np.uint8), rng.integers(0, 3, n).astype(np.uint8)
+        aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "max", "a": 0}]
+        _check_sga([(li["extendedprice"], {"lo": 1_000_000, "hi": 6_000_000})], [k1, k2], [li["quantity"]], aggs,
+                   expected_groups=12, kernel=f"{JIT}; replicated tables")
+    else:                                # no predicate, one u8 key, fp64 values (private slots)
+        aggs = [{"op": "sum", "a": 1}, {"op": "avg", "a": 0}, {"op": "count"}]
+        _check_sga([], [li["linestatus"]], vf, aggs, expected_groups=2, kernel=f"{JIT}; 4 private slots")
+
+
+def test_jit_off(monkeypatch):
+    """OCL_NO_JIT: the same plan runs on the unified kernel (the fallback stays exact)."""
+    monkeypatch.setenv("OCL_NO_JIT", "1")
+    n = 100_003
+    li = _lineitem(n, datagen.BASE_SEED + 4)
+    vi = [li["quantity"], li["extendedprice"], li["discount"], li["tax"]]
+    _check_sga([(li["shipdate"], {"hi": 10471})], [li["returnflag"]], vi, Q1_AGGS, expected_groups=4,
+               kernel="k_sga<")
