@@ -386,11 +386,11 @@ const char* fused_kernel_name(int kind) {
     case 15: return "k_sga_bulk<Sig Q1+MINMAX int64> (TMA bulk pipeline)";
     case 16: return "k_sga_bulk<Sig Q1+MINMAX fp64> (TMA bulk pipeline)";
     case 61: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
-    case 64: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; replicated tables>";
+    case 64: return "k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; CTA table>";
     case 71: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; 4 private slots>";
     case 90: return "k_sga_bulk<Sig of the plan, run-time compiled (NVRTC); 4 private slots>";
-    case 91: return "k_sga_bulk<Sig of the plan, run-time compiled (NVRTC); replicated tables>";
-    case 74: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; replicated tables>";
+    case 91: return "k_sga_bulk<Sig of the plan, run-time compiled (NVRTC); CTA table>";
+    case 74: return "k_sga_bulk<Sig key i64, COUNT/SUM/MIN/MAX; CTA table>";
     case 20: return "k_sga_glb<DynShape>";
     case 30: return "k_part_count/scatter/agg<DynShape> (hash-partitioned)";
     case 31: return "k_part_count/scatter/agg<StaticShape key i64> (hash-partitioned)";

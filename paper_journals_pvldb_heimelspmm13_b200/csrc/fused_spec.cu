@@ -16,11 +16,11 @@
 //    in shared memory ([slot][field][thread]: lane t always hits the same banks); a row
 //    costs a register compare against the 4 slot keys and a non-atomic read-modify-write —
 //    the limit of the paper's accumulators ∝ 1/G.
-//  * replicated tables (<= 2048 groups, integer COL values): nrep copies of a shared-memory
-//    hash table per CTA (consumer warp w -> copy w % nrep; nrep = min(warps, 72 KB / table),
-//    so the copies multiply as G falls; stored field-major), native 32-bit shared atomics — count, biased 64-bit
-//    sums as a 32-bit add whose carry is taken from the returned value (exact, no periodic
-//    fold), order-encoded MIN / MAX — and a loop-free home-slot hit.
+//  * CTA table (<= 2048 groups, integer COL values): one shared-memory hash table per CTA,
+//    as large as fits (tab_policy: replicas did not pay on B200), stored field-major, native
+//    32-bit shared atomics — count, biased 64-bit sums as a 32-bit add whose carry is taken
+//    from the returned value (exact, no periodic fold), order-encoded MIN / MAX — and
+//    slot-granular linear probing (one LDS.64 for a home-slot hit).
 // Rows outside the int32 fast path, the key ~0 and keys beyond the tier's capacity take
 // the exact per-row update of the HBM table.  At the end every CTA folds its records /
 // table into the HBM table (int128 sums).
@@ -100,6 +100,7 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
   sp->tab_nrep = 0;
   sp->pwait = 0;
   sp->cwait = 0;
+  sp->mm_check = 0;
   return true;
 }
 
@@ -220,29 +221,77 @@ static bool launch_few(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t*
   return true;
 }
 
-// Group-by signatures: the tier by expected groups — 4 private slots, or the replicated
-// tables (<= kSpecTabMaxGroups groups; replicas = min(consumer warps, 72 KB / table)).
-// false: no tier fits (the caller falls back).
+// Group-by signatures: the tier by expected groups — 4 private slots, or one shared-memory
+// hash table per CTA (<= kSpecTabMaxGroups groups).  false: no tier fits (the caller falls back).
 constexpr int64_t kSpecTabMaxGroups = 2048;
-constexpr size_t kTabBudget = 72 * 1024;   // + 2 stages of 20 KB: 2 CTAs per SM
+
+// CTA table: read-before-atomic MIN / MAX (smem_max), on by default: +0-4 % on uniform keys,
+// -25..45 % with Zipf 1.5 (C5 G = 16 1.89 -> 1.16 ms, G = 256 1.79 -> 1.26 ms, G = 2048
+// 2.07 -> 1.52 ms).  OCL_MM_CHECK=0/1 forces it (A/B).
+int32_t spec_mm_check(int64_t eg) {
+  (void)eg;
+  if (const char* e = getenv("OCL_MM_CHECK")) return atoi(e) != 0;
+  return 1;
+}
+
+// CTA-table policy (shared with the run-time compiled kernels, jit.cu).  Measured on B200, C5
+// on 2^28 rows (profiles/r02_tab_policy.md):
+//  - one table per CTA, as large as fits: replicas per warp group (the paper's "multiple
+//    accumulators") never paid here — across warps, shared atomics on one
+//    address cost no more than on different ones, while every replica raises the load
+//    factor of a fixed budget (G = 512: 2 replicas x 1024 slots 3.11 ms, 1 x 2048 1.80 ms);
+//  - one CTA of 30 consumer warps per SM (<960, 1920, 2>) with a 4096-slot table beats two
+//    CTAs of 16 warps with 2048 slots each at every G (G = 256 1.51 -> 1.26 ms);
+//  - slot-granular probing (one LDS.64 per row) beat buckets of 4 slots (two LDS.128) at
+//    every load up to 1/2 except G = 1024 uniform (1.52 vs 1.60 ms), so only slots remain.
+// Rows wider than the 30-warp stages allow fall back to <512, 1024, 2> (run-time compiled
+// signatures only).  The table must keep the load <= 1/2.  OCL_TAB="<wide|narrow>,<log2
+// slots>,<tables>" overrides (A/B).
+bool tab_policy(int64_t eg, size_t slot_bytes, size_t row_bytes, TabPolicy* tp) {
+  constexpr size_t kSmem = 225 * 1024;            // per SM, minus the static / reserved bytes
+  auto fit = [&](size_t budget) -> uint32_t {     // log2 of the largest table within budget
+    uint32_t hb = 0;
+    while (((size_t)2 << hb) * slot_bytes <= budget && hb < 16) ++hb;
+    return hb;
+  };
+  *tp = TabPolicy{};
+  tp->nrep = 1;
+  tp->NS = 2;
+  for (int wide = 1; wide >= 0 && tp->T == 0; --wide) {
+    const int R = wide ? 1920 : 1024;
+    const size_t stages = 2 * (size_t)R * row_bytes;
+    if (stages >= kSmem) continue;
+    const uint32_t hb = fit(kSmem - stages);
+    if (hb >= 6 && ((int64_t)1 << hb) >= 2 * eg) tp->T = wide ? 960 : 512, tp->R = R, tp->hb = hb;
+  }
+  if (const char* e = getenv("OCL_TAB")) {
+    char kind[8] = {0};
+    int a = 0, b = 0;
+    if (sscanf(e, "%6[a-z],%d,%d", kind, &a, &b) == 3 && a >= 6 && b >= 1) {
+      const bool wide = kind[0] == 'w';
+      const size_t stages = 2 * (size_t)(wide ? 1920 : 1024) * row_bytes;
+      if (((size_t)b << a) * slot_bytes + stages <= kSmem)
+        tp->T = wide ? 960 : 512, tp->R = wide ? 1920 : 1024, tp->hb = (uint32_t)a, tp->nrep = (uint32_t)b;
+    }
+  }
+  if (tp->T == 0) return false;
+  tp->mm_check = spec_mm_check(eg);
+  return true;
+}
 
 template <class S>
 static bool launch_grp(SpecPlan& sp, int sms, cudaStream_t s, cudaError_t* err, int* tier) {
   const int64_t eg = sp.g.expected > 0 ? sp.g.expected : 1;
   if (eg <= 4) { *tier = 1; return launch_bulk<S, 4, 128, 512, 2>(sp, sms, s, err); }
   if constexpr (S::cta_ok()) {
-    if (eg <= kSpecTabMaxGroups) {
-      constexpr int T = 512;                          // 16 consumer warps: latency hiding at 2 CTAs / SM
-      uint32_t hb = 6;                                // load <= 1/4 up to 256 groups, <= 1/2 above
-      while (((int64_t)1 << hb) < (eg <= 256 ? 4 : 2) * eg) ++hb;
-      const size_t one = ((size_t)1 << hb) * TabL<S>::BYTES_PER_SLOT;
-      size_t nrep = kTabBudget / one;
-      if (nrep > T / 32) nrep = T / 32;
-      if (nrep < 1) nrep = 1;
-      sp.tab_hb = hb;
-      sp.tab_nrep = (uint32_t)nrep;
+    TabPolicy tp;
+    if (eg <= kSpecTabMaxGroups && tab_policy(eg, TabL<S>::BYTES_PER_SLOT, BulkStage<S, 64>::BYTES / 64, &tp) &&
+        tp.T == 960) {                            // (the C5 / C3 rows always fit the wide stages)
+      sp.tab_hb = tp.hb;
+      sp.tab_nrep = tp.nrep;
+      sp.mm_check = tp.mm_check;
       *tier = 4;
-      return launch_bulk<S, 0, T, 1024, 2>(sp, sms, s, err);
+      return launch_bulk<S, 0, 960, 1920, 2>(sp, sms, s, err);
     }
   }
   return false;
@@ -260,7 +309,7 @@ bool spec_takes(const Plan& g) {
 // Try the specialised kernels; returns false if no signature matches.  *kind (see
 // fused_kernel_name): 11/12 = k_sga_priv Q1 (int / fp64), 13/14 = k_sga_bulk Q1, 15/16 =
 // k_sga_bulk Q1 + MIN/MAX, 60 + tier = C5 shape, 70 + tier = C3 shape (tier 1 = 4 private
-// slots, 4 = replicated tables).
+// slots, 4 = CTA table).
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind) {
   SpecPlan sp;
   const int64_t eg = g.expected > 0 ? g.expected : 1;

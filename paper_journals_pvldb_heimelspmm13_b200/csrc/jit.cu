@@ -305,7 +305,7 @@ static bool jit_self_check() {
 
 // Run-time specialised bulk kernel for a plan no compiled-in signature took; false if the
 // plan does not fit the signature scheme, JIT is off, or compiling / launching failed.
-// *kind: 90 = private slots, 91 = replicated tables.
+// *kind: 90 = private slots, 91 = CTA table.
 bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind) {
   if (getenv("OCL_NO_JIT")) return false;
   static const bool sane = jit_self_check();
@@ -330,18 +330,16 @@ bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, 
     tier = rt_priv_bytes(sig, L, T);
     *kind = 90;
   } else if (rt_cta_ok(sig) && eg <= 2048) {
+    TabPolicy tp;
+    if (!tab_policy(eg, rt_tab_slot_bytes(sig), rt_stage_bytes(sig, 64) / 64, &tp)) return false;
     L = 0;
-    T = 512;
-    R = 1024;
-    uint32_t hb = 6;
-    while (((int64_t)1 << hb) < (eg <= 256 ? 4 : 2) * eg) ++hb;
-    const size_t one = ((size_t)1 << hb) * rt_tab_slot_bytes(sig);
-    size_t nrep = (72 * 1024) / one;
-    if (nrep > (size_t)T / 32) nrep = T / 32;
-    if (nrep < 1) nrep = 1;
-    sp.tab_hb = hb;
-    sp.tab_nrep = (uint32_t)nrep;
-    tier = (((size_t)nrep << hb) * rt_tab_slot_bytes(sig) + 127) / 128 * 128;
+    T = tp.T;
+    R = tp.R;
+    NS = tp.NS;
+    sp.tab_hb = tp.hb;
+    sp.tab_nrep = tp.nrep;
+    sp.mm_check = tp.mm_check;
+    tier = (((size_t)tp.nrep << tp.hb) * rt_tab_slot_bytes(sig) + 127) / 128 * 128;
     *kind = 91;
   } else {
     return false;

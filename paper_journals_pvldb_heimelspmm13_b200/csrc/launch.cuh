@@ -86,6 +86,15 @@ const char* fused_kernel_name(int kind);
 bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 // Whether a plan-signature kernel takes this group-by plan (the planner keeps the one-pass tier).
 bool spec_takes(const Plan& g);
+int32_t spec_mm_check(int64_t expected_groups);
+// CTA-table tier of the signature kernels (fused_spec.cu): consumer threads T, rows per
+// stage R, stages NS, 2^hb slots x nrep tables, MIN / MAX read-before-atomic
+struct TabPolicy {
+  int T, R, NS;
+  uint32_t hb, nrep;
+  int32_t mm_check;
+};
+bool tab_policy(int64_t expected_groups, size_t slot_bytes, size_t row_bytes, TabPolicy* tp);
 // The signature kernels compiled at run time for a plan no compiled-in signature matches (jit.cu).
 bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 // High-cardinality tier (partition.cu): hash-partitioned two-pass aggregation.

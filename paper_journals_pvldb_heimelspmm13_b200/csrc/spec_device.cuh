@@ -66,9 +66,10 @@ struct SpecPlan {
   const void* k0;
   const void* k1;
   const void* col[4];
-  uint32_t tab_hb;            // replicated-table tier: log2 of the slots per replica (H)
-  uint32_t tab_nrep;          // replicated-table tier: replicas per CTA
+  uint32_t tab_hb;            // CTA-table tier: log2 of the slots per table (H)
+  uint32_t tab_nrep;          // CTA-table tier: tables per CTA (1 by default)
   int32_t pwait, cwait;       // barrier wait strategies of the producer / consumers (mbar_wait_mode)
+  int32_t mm_check;           // CTA-table tier: MIN / MAX atomics only when the value improves
 };
 
 template <class S>
@@ -574,18 +575,17 @@ __device__ __forceinline__ void priv_flush(const SpecPlan& p, const uint8_t* sm,
   }
 }
 
-// ------------------------------------------------------------------ replicated-table tier
+// ------------------------------------------------------------------ CTA-table tier
 // "Multiple accumulators per group, inversely proportional to the number of groups"
-// (§4.1.7): nrep replicas of a shared-memory hash table of H = pow2 >= 2G slots
-// per CTA, consumer warp w updating replica w % nrep, so cross-warp contention falls as G
-// falls (G = 16: one replica per warp).  A replica is stored field-major (SoA) so that the
-// 32 lanes of an atomic instruction on 32 different slots hit different banks: keys u64[H]
-// (~key, 0 = empty), count u32[H], then per value SUM -> biased sum lo u32[H], hi u32[H]
-// (the sum of (x + 2^31) over the rows, exact in 64 bits; sum = biased - count * 2^31; the
-// carry out of lo is taken from the atomic's return value), MIN / MAX -> order-encoded
-// u32[H]; all updated with native 32-bit shared atomics.  All-zero = empty / identity.
-// The home slot is read without a loop (one LDS.64 + compare); probing and claiming run
-// out of line for the warp's misses only.
+// (§4.1.7) as a shared-memory hash table of H = 2^hb slots per CTA; the kernel
+// still supports nrep replicas (consumer warp w -> replica w % nrep) but the host policy
+// (fused_spec.cu tab_policy) uses one: on B200 a replica only raised the load factor.  The
+// table is stored field-major (SoA) so that the 32 lanes of an atomic instruction on 32
+// different slots hit different banks: keys u64[H] (~key, 0 = empty), count u32[H], then
+// per value SUM -> biased sum lo u32[H], hi u32[H] (the sum of (x + 2^31) over the rows,
+// exact in 64 bits; sum = biased - count * 2^31; the carry out of lo is taken from the
+// atomic's return value), MIN / MAX -> order-encoded u32[H]; all updated with native 32-bit
+// shared atomics.  All-zero = empty / identity.
 template <class S>
 struct TabL {
   // u32 field index of count / value v's sum lo, sum hi, min, max (after the u64 keys)
@@ -605,6 +605,19 @@ struct TabL {
   // replica of H slots: keys at 0, u32 field f at 8H + 4H f
   __device__ static uint32_t* fld(uint8_t* rep, uint32_t H, int f) { return (uint32_t*)(rep + 8 * (size_t)H + 4 * (size_t)H * f); }
 };
+
+// MIN / MAX into a shared u32.  With `check`, the atomic only when the value improves on
+// what the slot holds: the field only moves towards the extreme, so a stale read can cost an
+// unneeded atomic but never skip a needed one; after warm-up almost no row improves, and
+// equal-key lanes of a warp read one broadcast word instead of serialising on one address
+// (few groups / skewed keys).  Without it, one atomic (many groups: the read is extra work).
+__device__ __forceinline__ void smem_max(uint32_t* a, uint32_t e, int32_t check) {
+  if (check) {
+    if (e > *(volatile uint32_t*)a) atomicMax(a, e);
+  } else {
+    atomicMax(a, e);
+  }
+}
 
 constexpr uint64_t kTabMul = 0x9E3779B97F4A7C15ULL;   // multiplicative hash: home slot = top hb bits
 
@@ -628,46 +641,54 @@ __device__ __forceinline__ TabRef<S> tab_ref(uint8_t* rep, uint32_t hb) {
   return t;
 }
 
-// Out-of-line probe / claim over whole buckets from the home bucket: slot, or -1 when the
-// replica is full.
+// Slot-granular linear probing from the home slot, out of line (claims): slot, or -1 when
+// the table is full.
 static __device__ __noinline__ int tab_find_slow(uint64_t* keys, uint32_t hb, uint64_t key) {
-  const uint32_t nb = 1u << (hb - 2);
+  const uint32_t H = 1u << hb;
   const uint64_t sk = ~key;
-  uint32_t b = (uint32_t)((key * kTabMul) >> (64 - (hb - 2)));
-  for (uint32_t probe = 0; probe < nb; ++probe) {
-    for (int j = 0; j < 4; ++j) {
-      uint64_t* kp = &keys[4 * b + j];
-      const uint64_t cur = *(volatile uint64_t*)kp;
-      if (cur == sk) return (int)(4 * b + j);
-      if (cur == 0) {
-        const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
-        if (prev == 0 || prev == sk) return (int)(4 * b + j);
-      }
+  uint32_t h = (uint32_t)((key * kTabMul) >> (64 - hb));
+  for (uint32_t probe = 0; probe < H; ++probe) {
+    uint64_t* kp = &keys[h];
+    const uint64_t cur = *(volatile uint64_t*)kp;
+    if (cur == sk) return (int)h;
+    if (cur == 0) {
+      const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
+      if (prev == 0 || prev == sk) return (int)h;
     }
-    b = (b + 1) & (nb - 1);
+    h = (h + 1) & (H - 1);
   }
   return -1;
 }
 
-// One row position of the warp (all 32 lanes call): the row into this warp's replica, or,
-// for a slow value / the key ~0 / a full replica, the exact HBM update.  Slots come in
-// buckets of 4 (32 bytes, read with two LDS.128); the home bucket is the top bits of
-// key * 2^64/phi.  A key present in its home bucket is found without a loop or a branch;
-// claims and bucket overflows go out of line, warp-uniformly, and only after warm-up rarely.
+// One row position of the warp (all 32 lanes call): the row into this warp's table, or, for
+// a slow value / the key ~0 / a full table, the exact HBM update.  Slot-granular linear
+// probing from the home slot (the top bits of key * 2^64/phi): a home-slot hit costs one
+// LDS.64 and no branch; further probes run inline, warp-uniformly, while every probed slot
+// holds another key (no deletions: a present key lies before the first empty slot of its
+// sequence); an empty slot means a claim, out of line.
 template <class S>
 __device__ __forceinline__ void tab_row(const SpecPlan& p, const TabRef<S>& t, const SRow<S>& x, int64_t r) {
   using TL = TabL<S>;
   const uint64_t k = (uint64_t)x.key;
   const uint64_t sk = ~k;
   const bool ok = x.q && x.fast && !spec_is_special<S>(x.key);
-  const uint32_t b = (uint32_t)((k * kTabMul) >> (64 - (t.hb - 2)));
-  const ulonglong2* bp = (const ulonglong2*)(t.keys + 4 * b);
-  const ulonglong2 k01 = bp[0], k23 = bp[1];
-  int h = (int)(4 * b);
-  h = k01.x == sk ? h : (k01.y == sk ? h + 1 : (k23.x == sk ? h + 2 : (k23.y == sk ? h + 3 : -1)));
-  const bool miss = ok && h < 0;
-  if (__any_sync(0xffffffffu, miss))
-    if (miss) h = tab_find_slow(t.keys, t.hb, k);
+  uint32_t hh = (uint32_t)((k * kTabMul) >> (64 - t.hb));
+  uint64_t c = t.keys[hh];
+  int h = c == sk ? (int)hh : -1;
+  if (__any_sync(0xffffffffu, ok && h < 0)) {
+    bool pend = ok && h < 0 && c != 0;
+    bool claim = ok && h < 0 && c == 0;
+    while (__any_sync(0xffffffffu, pend)) {
+      if (pend) {
+        hh = (hh + 1) & t.mask;
+        c = t.keys[hh];
+        if (c == sk) { h = (int)hh; pend = false; }
+        else if (c == 0) { claim = true; pend = false; }
+      }
+    }
+    if (__any_sync(0xffffffffu, claim))
+      if (claim) h = tab_find_slow(t.keys, t.hb, k);
+  }
   if (x.q && (!ok || h < 0)) {                        // slow value, key ~0, or a full replica
     uint8_t* g = table_find_or_insert(p.g.table, p.g.mask, p.g.stride, k, p.g.status);
     if (g) update_entry_slow(p.g, g, r);
@@ -682,8 +703,8 @@ __device__ __forceinline__ void tab_row(const SpecPlan& p, const TabRef<S>& t, c
       const uint32_t old = atomicAdd(t.f[TL::f_sum(v)] + h, a);
       if (old + a < old) atomicAdd(t.f[TL::f_sum(v) + 1] + h, 1u);
     }
-    if (S::has(v, VS_MIN)) atomicMax(t.f[TL::f_min(v)] + h, s_enc32_min(xv));
-    if (S::has(v, VS_MAX)) atomicMax(t.f[TL::f_max(v)] + h, s_enc32_max(xv));
+    if (S::has(v, VS_MIN)) smem_max(t.f[TL::f_min(v)] + h, s_enc32_min(xv), p.mm_check);
+    if (S::has(v, VS_MAX)) smem_max(t.f[TL::f_max(v)] + h, s_enc32_max(xv), p.mm_check);
   }
 }
 
@@ -754,7 +775,7 @@ __device__ __forceinline__ void lds2(const uint8_t* base, int j, uint64_t& x0, u
   }
 }
 
-// Shared-memory bytes of the accumulation tier: L > 0 private records; L == 0 the replicated
+// Shared-memory bytes of the accumulation tier: L > 0 private records; L == 0 the CTA
 // tables (nrep x H slots, run time).
 template <class S, int L>
 __host__ __device__ constexpr size_t tier_bytes(int T, uint32_t tab_slots) {
@@ -765,7 +786,7 @@ __host__ __device__ constexpr size_t tier_bytes(int T, uint32_t tab_slots) {
 // kernel at 72 registers and spilled two values per 64-row unit to local memory (+0.6 GB
 // of L2 traffic on C4, 3.56 -> 4.19 ms); the shared-memory footprint allows 2-3 CTAs anyway
 template <int T>
-__host__ __device__ constexpr int bulk_min_blocks() { return T <= 128 ? 3 : 2; }
+__host__ __device__ constexpr int bulk_min_blocks() { return T <= 128 ? 3 : (T <= 512 ? 2 : 1); }
 
 template <class S, int L, int T, int R, int NS>
 __global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const __grid_constant__ SpecPlan p) {
@@ -795,7 +816,7 @@ __global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const
   }
   __syncthreads();
   const DirState<LD> d{dir};
-  // replicated-table tier: this warp's replica
+  // CTA-table tier: this warp's table
   const TabRef<S> mytab = tab_ref<S>(sm + (L > 0 ? 0 : (size_t)(wid % (p.tab_nrep ? p.tab_nrep : 1)) *
                                                          ((size_t)1 << p.tab_hb) * TabL<S>::BYTES_PER_SLOT),
                                      L > 0 ? 5u : p.tab_hb);

@@ -156,14 +156,14 @@ C5_AGGS = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op":
 
 
 def _c5_tier(G):
-    return "4 private slots" if G <= 4 else "replicated tables"
+    return "4 private slots" if G <= 4 else "CTA table"
 
 
 @pytest.mark.parametrize("G", [4, 16, 32, 64, 256, 1024, 2048])
 @pytest.mark.parametrize("zipf,sel", [(0.0, 10**6), (1.5, 5 * 10**5), (1.0, 10**4)])
 def test_c5_signature_tiers(G, zipf, sel):
     """The C5 bench plan (WHERE p < T GROUP BY key: COUNT, SUM, MIN, MAX of v) on both accumulation tiers
-    of k_sga_bulk<Sig pred i32, key i64> (private slots, replicated tables with 8 / 4 / 1 replicas), uniform
+    of k_sga_bulk<Sig pred i32, key i64> (private slots, CTA table), uniform
     and skewed keys (Zipf 1.5 puts ~38 % of the rows on one key), three selectivities."""
     n = (1 << 21) + 77
     sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, G, s=zipf)
@@ -238,18 +238,18 @@ def test_jit_signatures(case):
     elif case == "q1_f64_max":           # fp64 Q1 + MAX(tax)
         _check_sga(pred, [li["returnflag"], li["linestatus"]], vf, Q1_AGGS_F64 + [{"op": "max", "a": 3}],
                    expected_groups=4, order_by_key=True, kernel=f"{JIT}; 4 private slots")
-    elif case == "two_values_tables":    # C5-like with two value columns: replicated tables
+    elif case == "two_values_tables":    # C5-like with two value columns: CTA table
         sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, 300, s=1.0)
         v2 = (sw["v"] * 3 - 7).astype(np.int64)
         aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "max", "a": 1}, {"op": "min", "a": 1}]
         _check_sga([(sw["p"], {"hi": 799_999})], [sw["key"]], [sw["v"], v2], aggs, expected_groups=300,
-                   kernel=f"{JIT}; replicated tables")
+                   kernel=f"{JIT}; CTA table")
     elif case == "i64_pred_tables":      # predicate on an int64 column, u8 x u8 keys, 12 groups
         rng = np.random.default_rng(4)
         k1, k2 = rng.integers(0, 4, n).astype(np.uint8), rng.integers(0, 3, n).astype(np.uint8)
         aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "max", "a": 0}]
         _check_sga([(li["extendedprice"], {"lo": 1_000_000, "hi": 6_000_000})], [k1, k2], [li["quantity"]], aggs,
-                   expected_groups=12, kernel=f"{JIT}; replicated tables")
+                   expected_groups=12, kernel=f"{JIT}; CTA table")
     else:                                # no predicate, one u8 key, fp64 values (private slots)
         aggs = [{"op": "sum", "a": 1}, {"op": "avg", "a": 0}, {"op": "count"}]
         _check_sga([], [li["linestatus"]], vf, aggs, expected_groups=2, kernel=f"{JIT}; 4 private slots")

@@ -103,7 +103,7 @@ def _():
 def _():
     p = [(sw["p"], {"hi": 699_999})]
     assert "4 private slots" in check_sga(p, [sw["key"] % 3], [sw["v"]], C5AGGS, expected_groups=4)
-    assert "replicated tables" in check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=300)
+    assert "CTA table" in check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=300)
     for tier in (1, 2, 3, 4):          # generic register tier, HBM tier, dynamic shape, CTA table
         check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=300, tier=tier)
     check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=2000, tier=5)   # hash-partitioned
