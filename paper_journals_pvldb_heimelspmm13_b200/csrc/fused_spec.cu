@@ -51,6 +51,23 @@ using SigQ1FMM = Sig<4, false, 1, 1, 4, true, vop(VX_COL, 0, 0, 0, VS_SUM | VS_M
 using SigC5 = Sig<4, false, 8, 0, 1, false, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN | VS_MAX)>;
 using SigC3 = Sig<0, false, 8, 0, 1, false, vop(VX_COL, 0, 0, 0, VS_SUM | VS_MIN | VS_MAX)>;
 
+// Select-compact-gather threshold (k_sga_bulk): CTAs whose predicate sample selects less
+// than this many percent of the rows stream the predicate column only and gather the
+// qualifying rows' key / value sectors.  Off below 2^24 rows, where the sample's latency at
+// kernel start is not amortised.  OCL_SPARSE_PCT overrides (0 = off).
+int32_t spec_sparse_pct(int64_t n) {
+  if (const char* e = getenv("OCL_SPARSE_PCT")) return atoi(e);
+  return n >= ((int64_t)1 << 24) ? 8 : 0;
+}
+
+// The threshold a launch uses: 0 without a predicate; on the private tier (<= 4 groups) 0
+// unless OCL_SPARSE_PCT is set — the twin's early exit costs its 3 x 148 CTAs ~16 us
+// (C4 3.46 -> 3.49 ms), more than the mode is worth there (C5 G = 4 at 1 %: 0.86 -> 0.74 ms).
+int32_t spec_twin_pct(int32_t pct, bool has_pred, bool private_tier) {
+  if (!has_pred || (private_tier && !getenv("OCL_SPARSE_PCT"))) return 0;
+  return pct;
+}
+
 template <class S>
 static bool spec_match(const Plan& g, SpecPlan* sp) {
   if ((S::PW > 0) != (g.npreds == 1) || g.npreds > 1) return false;
@@ -101,6 +118,7 @@ static bool spec_match(const Plan& g, SpecPlan* sp) {
   sp->pwait = 0;
   sp->cwait = 0;
   sp->mm_check = 0;
+  sp->sparse_pct = spec_sparse_pct(g.n);
   return true;
 }
 
@@ -155,16 +173,36 @@ static bool launch_bulk(const SpecPlan& sp, int sms, cudaStream_t s, cudaError_t
   int64_t grid = (int64_t)sms * nb;
   const int64_t chunks = sp.g.n / R;
   if (chunks < grid) grid = chunks;
+  SpecPlan q = sp;
   if (const char* w = getenv("OCL_WAIT")) {        // "<producer><consumer>" digits, e.g. "10"
-    SpecPlan& q = const_cast<SpecPlan&>(sp);
     q.pwait = w[0] ? w[0] - '0' : 0;
     q.cwait = w[0] && w[1] ? w[1] - '0' : 0;
   }
+  q.sparse_pct = spec_twin_pct(q.sparse_pct, S::PW > 0, L > 0);
   if (getenv("OCL_DEBUG"))
-    fprintf(stderr, "[ocl] k_sga_bulk L=%d T=%d R=%d NS=%d tab=%u x 2^%u smem=%zu blocks/SM=%d grid=%lld\n", L, T,
-            R, NS, sp.tab_nrep, sp.tab_hb, smem, nb, (long long)grid);
+    fprintf(stderr, "[ocl] k_sga_bulk L=%d T=%d R=%d NS=%d tab=%u x 2^%u smem=%zu blocks/SM=%d grid=%lld sparse<%d%%\n",
+            L, T, R, NS, q.tab_nrep, q.tab_hb, smem, nb, (long long)grid, q.sparse_pct);
+  if constexpr (S::PW > 0) {
+    // select-compact-gather twin first: exactly one of the two kernels runs past its sample
+    if (q.sparse_pct > 0) {
+      auto fs = k_sga_sparse<S, L, T, R, NS>;
+      static DevCache sattr;
+      if ((int)smem > sattr.get([&]() -> int { return 0; })) {
+        if (cudaFuncSetAttribute(fs, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)smem) != cudaSuccess) {
+          cudaGetLastError();
+          return false;
+        }
+        int d = 0;
+        cudaGetDevice(&d);
+        if (d >= 0 && d < kMaxDevices) sattr.v[d].store((int)smem, std::memory_order_relaxed);
+      }
+      count_launch();
+      fs<<<(int)grid, T + 32, smem, s>>>(q);
+      if ((*err = cudaGetLastError()) != cudaSuccess) return true;
+    }
+  }
   count_launch();
-  fn<<<(int)grid, T + 32, smem, s>>>(sp);
+  fn<<<(int)grid, T + 32, smem, s>>>(q);
   *err = cudaGetLastError();
   return true;
 }

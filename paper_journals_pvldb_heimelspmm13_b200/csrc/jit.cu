@@ -191,9 +191,9 @@ constexpr RtSig kQ1Check = [] {
 using Q1CheckSig = Sig<4, false, 1, 1, 4, false, vop(VX_COL, 0), vop(VX_COL, 1), vop(VX_M1, 1, 2),
                        vop(VX_M1P, 1, 2, 3), vop(VX_COL, 2)>;
 
-std::string sig_expr(const RtSig& s, int L, int T, int R, int NS) {
+std::string sig_expr(const RtSig& s, int L, int T, int R, int NS, const char* kernel = "k_sga_bulk") {
   char buf[512];
-  int n = snprintf(buf, sizeof(buf), "ocl::k_sga_bulk<ocl::Sig<%d, %s, %d, %d, %d, %s", s.PW, s.PF64 ? "true" : "false",
+  int n = snprintf(buf, sizeof(buf), "ocl::%s<ocl::Sig<%d, %s, %d, %d, %d, %s", kernel, s.PW, s.PF64 ? "true" : "false",
                    s.K0W, s.K1W, s.NC, s.F64 ? "true" : "false");
   for (int v = 0; v < s.NV; ++v) n += snprintf(buf + n, sizeof(buf) - n, ", %uu", s.ops[v]);
   snprintf(buf + n, sizeof(buf) - n, ">, %d, %d, %d, %d>", L, T, R, NS);
@@ -313,6 +313,7 @@ bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, 
   RtSig sig;
   SpecPlan sp;
   if (!rt_sig_of(g, &sig, &sp)) return false;
+  sp.sparse_pct = spec_sparse_pct(g.n);
   auto a16 = [](const void* q) { return ((uintptr_t)q & 15) == 0; };
   if ((sig.PW > 0 && !a16(sp.pcol)) || (sig.K0W > 0 && !a16(sp.k0)) || (sig.K1W > 0 && !a16(sp.k1))) return false;
   for (int i = 0; i < sig.NC; ++i)
@@ -347,9 +348,17 @@ bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, 
   if (sp.g.n < R) return false;
   JitKernel* jk = jit_get(sig_expr(sig, L, T, R, NS));
   if (!jk) return false;
+  sp.sparse_pct = spec_twin_pct(sp.sparse_pct, sig.PW > 0, L > 0);
+  JitKernel* jks = nullptr;                      // the select-compact-gather twin (k_sga_sparse)
+  if (sig.PW > 0 && sp.sparse_pct > 0 && !(jks = jit_get(sig_expr(sig, L, T, R, NS, "k_sga_sparse"))))
+    sp.sparse_pct = 0;
   const size_t smem = tier + (size_t)NS * rt_stage_bytes(sig, R);
   int sc = 0;
   for (uint32_t c = sp.tab_nrep << sp.tab_hb; c > 128 && sc < 7; c >>= 1) ++sc;
+  if (jks) {
+    if (!jit_launch(jks, sp, smem, T, R, sms, s, err, sc)) return false;
+    if (*err != cudaSuccess) return true;
+  }
   return jit_launch(jk, sp, smem, T, R, sms, s, err, sc);
 }
 

@@ -87,6 +87,8 @@ bool launch_fused_spec(const Plan& g, int sms, cudaStream_t s, cudaError_t* err,
 // Whether a plan-signature kernel takes this group-by plan (the planner keeps the one-pass tier).
 bool spec_takes(const Plan& g);
 int32_t spec_mm_check(int64_t expected_groups);
+int32_t spec_sparse_pct(int64_t n);
+int32_t spec_twin_pct(int32_t pct, bool has_pred, bool private_tier);
 // CTA-table tier of the signature kernels (fused_spec.cu): consumer threads T, rows per
 // stage R, stages NS, 2^hb slots x nrep tables, MIN / MAX read-before-atomic
 struct TabPolicy {

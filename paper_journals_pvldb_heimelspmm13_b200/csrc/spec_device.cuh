@@ -70,6 +70,7 @@ struct SpecPlan {
   uint32_t tab_nrep;          // CTA-table tier: tables per CTA (1 by default)
   int32_t pwait, cwait;       // barrier wait strategies of the producer / consumers (mbar_wait_mode)
   int32_t mm_check;           // CTA-table tier: MIN / MAX atomics only when the value improves
+  int32_t sparse_pct;         // select-compact-gather below this sampled selectivity (%); 0 = off
 };
 
 template <class S>
@@ -788,20 +789,151 @@ __host__ __device__ constexpr size_t tier_bytes(int T, uint32_t tab_slots) {
 template <int T>
 __host__ __device__ constexpr int bulk_min_blocks() { return T <= 128 ? 3 : (T <= 512 ? 2 : 1); }
 
-template <class S, int L, int T, int R, int NS>
-__global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const __grid_constant__ SpecPlan p) {
-  using B = BulkStage<S, R>;
-  constexpr int NW = T / 32;                 // consumer warps
-  constexpr int UPW = R / 64 / NW;           // 64-row units per consumer warp per stage
-  static_assert(UPW >= 1 && UPW * 64 * NW == R, "R must be 64 * consumer warps * units");
+// Select-compact-gather stages: the ring's stage buffers carry RS rows of the predicate
+// column only — US 64-row units per consumer warp (at most 5: the warp keeps 2 ballot masks
+// per unit in registers).
+template <class S, class B, int NW>
+struct SparseStage {
+  static constexpr int PWB = S::PW > 0 ? S::PW : 1;
+  static constexpr int FIT = B::BYTES / PWB / (64 * NW);
+  static constexpr int US = FIT < 1 ? 1 : (FIT > 5 ? 5 : FIT);
+  static constexpr int RS = 64 * NW * US;
+  static_assert(S::PW == 0 || RS * S::PW <= B::BYTES, "sparse stage must fit a dense stage buffer");
+};
+
+// Consumers of the select-compact-gather mode (the paper's select -> prefix-sum compaction
+// -> grouping, §4.1.1-4.1.2, per stage and per warp): a warp evaluates the
+// predicate on its US units of kSparseBatch consecutive stages of its CTA, releasing each
+// stage as soon as its ballots are taken, then turns the ballot masks (shared memory, one
+// word per unit and row parity) into a compacted list of qualifying rows (n-th set bit)
+// and gathers key and value columns for those rows only, 32 at a time, from global
+// memory.  Batching stages doubles the gathers in flight per warp (latency-bound at 1 %).
+constexpr int kSparseBatch = 2;
+
+template <class S, int L, int LD, int T, class B, int NS>
+__device__ __forceinline__ void sparse_consume(const SpecPlan& p, const DirState<LD>& d, KeyT<S> (&rk)[LD],
+                                               uint8_t* sm, const TabRef<S>& mytab, const uint8_t* stg,
+                                               uint64_t* full, uint64_t* empty, int64_t nfull, int tid) {
+  constexpr int NW = T / 32;
+  constexpr int US = SparseStage<S, B, NW>::US;
+  constexpr int RS = SparseStage<S, B, NW>::RS;
+  constexpr int NM = 2 * US * kSparseBatch;               // masks per warp and batch
+  __shared__ uint32_t smk[NW][NM];
+  const int lane = tid & 31, wid = tid >> 5;
+  uint32_t* mk = smk[wid];
+  int stage = 0;
+  uint32_t phase = 0;
+  for (int64_t c0 = blockIdx.x; c0 < nfull; c0 += (int64_t)kSparseBatch * gridDim.x) {
+    int tot = 0;
+#pragma unroll
+    for (int g = 0; g < kSparseBatch; ++g) {
+      const int64_t c = c0 + (int64_t)g * gridDim.x;
+      if (c >= nfull) {                                    // (warp-uniform) no stage: empty masks
+        if (lane < 2 * US) mk[g * 2 * US + lane] = 0u;
+        continue;
+      }
+      mbar_wait_mode(&full[stage], phase, p.cwait);
+      const uint8_t* sd = stg + (size_t)stage * B::BYTES;
+#pragma unroll
+      for (int u = 0; u < US; ++u) {
+        uint64_t a0, a1;
+        lds2<S::PW>(sd, (wid * US + u) * 64 + 2 * lane, a0, a1);
+        const bool q0 = spec_pred<S>(p, a0), q1 = spec_pred<S>(p, a1);
+        if (p.g.bitmap_out) emit_bitmap_unit(p.g, c * RS + (wid * US + u) * 64, lane, q0, q1);
+        const uint32_t m0 = __ballot_sync(0xffffffffu, q0), m1 = __ballot_sync(0xffffffffu, q1);
+        if (lane == 0) {
+          mk[(g * US + u) * 2] = m0;
+          mk[(g * US + u) * 2 + 1] = m1;
+        }
+        tot += __popc(m0) + __popc(m1);
+      }
+      mbar_release_reads(&empty[stage], lane);
+      if (++stage == NS) {
+        stage = 0;
+        phase ^= 1;
+      }
+    }
+    __syncwarp();
+    for (int b0 = 0; b0 < tot; b0 += 32) {              // warp-uniform rounds of 32 rows
+      int t = b0 + lane;
+      const bool valid = t < tot;
+      int64_t r = 0;                                     // the t-th qualifying row of the batch
+#pragma unroll 4
+      for (int m = 0; m < NM; ++m) {
+        const uint32_t w = mk[m];
+        const int cm = __popc(w);
+        if (t >= 0 && t < cm) {
+          const int g = m / (2 * US), u = (m / 2) % US;
+          r = (c0 + (int64_t)g * gridDim.x) * RS + (wid * US + u) * 64 + 2 * (int)__fns(w, 0, t + 1) + (m & 1);
+        }
+        t -= cm;
+      }
+      SRow<S> x;
+      x.q = valid;
+      x.fast = true;
+      uint64_t k0 = 0, k1 = 0, cv[S::NC];
+#pragma unroll
+      for (int i = 0; i < S::NC; ++i) cv[i] = 0;
+      if (valid) {
+        if constexpr (S::K0W > 0) k0 = ld1<S::K0W>(p.k0, r);
+        if constexpr (S::K1W > 0) k1 = ld1<S::K1W>(p.k1, r);
+#pragma unroll
+        for (int i = 0; i < S::NC; ++i) cv[i] = ld1<8>(p.col[i], r);
+      }
+      x.key = spec_key<S>(k0, k1);
+      spec_values<S>(p, cv, x);
+      if constexpr (L > 0) {
+        SRow<S> none = x;                                // second row position unused
+        none.q = false;
+        priv_rows<S, LD, T>(p, d, rk, sm, tid, x, none, r);
+      } else {
+        tab_row<S>(p, mytab, x, r);
+      }
+    }
+    __syncwarp();                                        // masks are rewritten by the next batch
+  }
+}
+
+// Select-compact-gather decision, identical in every CTA of both kernels (k_sga_sparse runs
+// iff k_sga_bulk exits): the predicate on kSparseSample rows at fixed positions spread
+// over the input, against p.sparse_pct %.  Every thread of the CTA calls it.
+constexpr int kSparseSample = 1024;
+
+template <class S, int NT>
+__device__ __forceinline__ bool spec_sparse(const SpecPlan& p) {
+  if constexpr (S::PW == 0) {
+    return false;
+  } else {
+    constexpr int PER = (kSparseSample + NT - 1) / NT;
+    __shared__ int s_cnt;
+    const int64_t span = p.g.n / kSparseSample;
+    int q = 0;
+    if (span > 0) {
+      uint64_t raw[PER];
+#pragma unroll
+      for (int k = 0; k < PER; ++k) {                   // all loads in flight, then the predicates
+        const int i = threadIdx.x + k * NT;
+        raw[k] = i < kSparseSample ? ld1<S::PW>(p.pcol, (int64_t)i * span) : 0;
+      }
+#pragma unroll
+      for (int k = 0; k < PER; ++k) q += (threadIdx.x + k * NT < kSparseSample && spec_pred<S>(p, raw[k])) ? 1 : 0;
+    }
+    if (threadIdx.x == 0) s_cnt = 0;
+    __syncthreads();
+    if (q) atomicAdd(&s_cnt, q);
+    __syncthreads();
+    return span > 0 && 100 * s_cnt < p.sparse_pct * kSparseSample;
+  }
+}
+
+// Shared-memory setup of both bulk kernels: zeroed accumulation tier, directory, barriers.
+template <class S, int L, int T, int NS>
+__device__ __forceinline__ size_t bulk_setup(const SpecPlan& p, uint8_t* sm, uint64_t* dir, uint64_t* full,
+                                             uint64_t* empty, int tid) {
+  constexpr int NW = T / 32;
   constexpr int LD = L > 0 ? L : 1;
-  extern __shared__ __align__(128) uint8_t sm[];
   const uint32_t tab_slots = L > 0 ? 0u : ((uint32_t)p.tab_nrep << p.tab_hb);
   const size_t tb = tier_bytes<S, L>(T, tab_slots);
-  uint8_t* stg = sm + tb;
-  __shared__ uint64_t dir[LD];
-  __shared__ __align__(8) uint64_t full[NS], empty[NS];
-  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
   {
     uint4* z = (uint4*)sm;
     for (int i = tid; i < (int)(tb / 16); i += T + 32) z[i] = make_uint4(0, 0, 0, 0);
@@ -815,12 +947,56 @@ __global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const
     mbar_fence_init();
   }
   __syncthreads();
+  return tb;
+}
+
+// CTA-table tier: this warp's table
+template <class S, int L>
+__device__ __forceinline__ TabRef<S> bulk_tab(const SpecPlan& p, uint8_t* sm, int wid) {
+  return tab_ref<S>(sm + (L > 0 ? 0 : (size_t)(wid % (p.tab_nrep ? p.tab_nrep : 1)) * ((size_t)1 << p.tab_hb) *
+                                           TabL<S>::BYTES_PER_SLOT),
+                    L > 0 ? 5u : p.tab_hb);
+}
+
+// Ragged tail (< one chunk of `crows` rows after nfull chunks): one CTA, scalar loads
+// straight from global memory.
+template <class S, int L, int LD, int T>
+__device__ __forceinline__ void bulk_tail(const SpecPlan& p, const DirState<LD>& d, KeyT<S> (&rk)[LD], uint8_t* sm,
+                                          const TabRef<S>& mytab, int64_t nfull, int64_t crows, int tid) {
+  constexpr int NW = T / 32;
+  const int lane = tid & 31, wid = tid >> 5;
+  if (blockIdx.x != (int)(nfull % gridDim.x)) return;
+  for (int64_t base = nfull * crows + (int64_t)wid * 64; base < p.g.n; base += 64 * NW) {
+    const int64_t r = base + 2 * lane;
+    SRow<S> x0, x1;
+    spec_row_scalar<S>(p, r, x0);
+    spec_row_scalar<S>(p, r + 1, x1);
+    if (p.g.bitmap_out) emit_bitmap_unit(p.g, base, lane, x0.q, x1.q);
+    if constexpr (L > 0) {
+      priv_rows<S, LD, T>(p, d, rk, sm, tid, x0, x1, r);
+    } else {
+      tab_row<S>(p, mytab, x0, r);
+      tab_row<S>(p, mytab, x1, r + 1);
+    }
+  }
+}
+
+template <class S, int L, int T, int R, int NS>
+__global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const __grid_constant__ SpecPlan p) {
+  using B = BulkStage<S, R>;
+  constexpr int NW = T / 32;                 // consumer warps
+  constexpr int UPW = R / 64 / NW;           // 64-row units per consumer warp per stage
+  static_assert(UPW >= 1 && UPW * 64 * NW == R, "R must be 64 * consumer warps * units");
+  constexpr int LD = L > 0 ? L : 1;
+  extern __shared__ __align__(128) uint8_t sm[];
+  __shared__ uint64_t dir[LD];
+  __shared__ __align__(8) uint64_t full[NS], empty[NS];
+  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+  if constexpr (S::PW > 0)
+    if (p.sparse_pct > 0 && spec_sparse<S, T + 32>(p)) return;   // k_sga_sparse took this call
+  uint8_t* stg = sm + bulk_setup<S, L, T, NS>(p, sm, dir, full, empty, tid);
   const DirState<LD> d{dir};
-  // CTA-table tier: this warp's table
-  const TabRef<S> mytab = tab_ref<S>(sm + (L > 0 ? 0 : (size_t)(wid % (p.tab_nrep ? p.tab_nrep : 1)) *
-                                                         ((size_t)1 << p.tab_hb) * TabL<S>::BYTES_PER_SLOT),
-                                     L > 0 ? 5u : p.tab_hb);
-  (void)lane;
+  const TabRef<S> mytab = bulk_tab<S, L>(p, sm, wid);
   const int64_t n = p.g.n;
   const int64_t nfull = n / R;
   if (wid == NW) {
@@ -894,22 +1070,54 @@ __global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_bulk(const
         }
       }
     }
-    // ragged tail (< R rows): one CTA, scalar loads straight from global memory
-    if (blockIdx.x == (int)(nfull % gridDim.x)) {
-      for (int64_t base = nfull * R + (int64_t)wid * 64; base < n; base += 64 * NW) {
-        const int64_t r = base + 2 * lane;
-        SRow<S> x0, x1;
-        spec_row_scalar<S>(p, r, x0);
-        spec_row_scalar<S>(p, r + 1, x1);
-        if (p.g.bitmap_out) emit_bitmap_unit(p.g, base, lane, x0.q, x1.q);
-        if constexpr (L > 0) {
-          priv_rows<S, LD, T>(p, d, rk, sm, tid, x0, x1, r);
-        } else {
-          tab_row<S>(p, mytab, x0, r);
-          tab_row<S>(p, mytab, x1, r + 1);
+    bulk_tail<S, L, LD, T>(p, d, rk, sm, mytab, nfull, R, tid);
+  }
+  if constexpr (L > 0) priv_flush<S, LD, T>(p, sm, d, tid);
+  else tab_flush<S>(p, sm, tid, T + 32);
+}
+
+// The select-compact-gather twin of k_sga_bulk (same accumulation tiers and shared-memory
+// layout; launched before it, exactly one of the two runs past its sample): the ring
+// carries the predicate column only, RS rows per stage, and the consumers gather key and
+// value sectors for the qualifying rows (sparse_consume).
+template <class S, int L, int T, int R, int NS>
+__global__ void __launch_bounds__(T + 32, bulk_min_blocks<T>()) k_sga_sparse(const __grid_constant__ SpecPlan p) {
+  static_assert(S::PW > 0, "select-compact-gather needs a predicate");
+  using B = BulkStage<S, R>;
+  constexpr int NW = T / 32;
+  constexpr int RS = SparseStage<S, B, NW>::RS;
+  constexpr int LD = L > 0 ? L : 1;
+  extern __shared__ __align__(128) uint8_t sm[];
+  __shared__ uint64_t dir[LD];
+  __shared__ __align__(8) uint64_t full[NS], empty[NS];
+  const int tid = threadIdx.x, lane = tid & 31, wid = tid >> 5;
+  if (p.sparse_pct <= 0 || !spec_sparse<S, T + 32>(p)) return;   // k_sga_bulk takes this call
+  uint8_t* stg = sm + bulk_setup<S, L, T, NS>(p, sm, dir, full, empty, tid);
+  const DirState<LD> d{dir};
+  const TabRef<S> mytab = bulk_tab<S, L>(p, sm, wid);
+  const int64_t nfull = p.g.n / RS;
+  if (wid == NW) {
+    if (lane == 0) {
+      const uint64_t pol = policy_evict_first();
+      int stage = 0;
+      uint32_t phase = 0;
+      for (int64_t c = blockIdx.x; c < nfull; c += gridDim.x) {
+        mbar_wait_mode(&empty[stage], phase ^ 1, p.pwait);
+        uint64_t* fb = &full[stage];
+        mbar_arrive_expect_tx(fb, RS * S::PW);
+        bulk_g2s(stg + (size_t)stage * B::BYTES, (const uint8_t*)p.pcol + c * RS * S::PW, RS * S::PW, fb, pol);
+        if (++stage == NS) {
+          stage = 0;
+          phase ^= 1;
         }
       }
     }
+  } else {
+    KeyT<S> rk[LD];
+#pragma unroll
+    for (int s = 0; s < LD; ++s) rk[s] = (KeyT<S>)~0ULL;
+    sparse_consume<S, L, LD, T, B, NS>(p, d, rk, sm, mytab, stg, full, empty, nfull, tid);
+    bulk_tail<S, L, LD, T>(p, d, rk, sm, mytab, nfull, RS, tid);
   }
   if constexpr (L > 0) priv_flush<S, LD, T>(p, sm, d, tid);
   else tab_flush<S>(p, sm, tid, T + 32);

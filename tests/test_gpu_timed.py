@@ -263,3 +263,64 @@ def test_jit_off(monkeypatch):
     vi = [li["quantity"], li["extendedprice"], li["discount"], li["tax"]]
     _check_sga([(li["shipdate"], {"hi": 10471})], [li["returnflag"]], vi, Q1_AGGS, expected_groups=4,
                kernel="k_sga<")
+
+
+# ---------------------------------------------------------------- select-compact-gather (k_sga_sparse)
+@pytest.mark.parametrize("G", [4, 16, 300, 2000])
+@pytest.mark.parametrize("zipf,sel", [(0.0, 0.001), (1.0, 0.01), (1.5, 0.05), (0.0, 0.3)])
+def test_c5_select_compact_gather(monkeypatch, G, zipf, sel):
+    """k_sga_sparse: the ring carries the predicate column only; each warp compacts its qualifying rows from
+    the ballot masks and gathers their key / value sectors (select -> prefix-sum
+    compaction -> grouping, per stage).  OCL_SPARSE_PCT=100 forces it whenever the sample selects < 100 %."""
+    monkeypatch.setenv("OCL_SPARSE_PCT", "100")
+    n = (1 << 21) + 77                               # several batches per CTA and a ragged tail
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 7, G, s=zipf)
+    preds = [(sw["p"], {"hi": int(round(sel * 10**6)) - 1})]
+    _check_sga(preds, [sw["key"]], [sw["v"]], C5_AGGS, expected_groups=G,
+               kernel=f"k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; {_c5_tier(G)}>")
+
+
+@pytest.mark.parametrize("G", [4, 300])
+def test_sparse_bitmap_and_exact_paths(monkeypatch, G):
+    """Select-compact-gather with the bitmap output, values beyond int32 (exact per-row path), the key ~0
+    and an empty selection."""
+    monkeypatch.setenv("OCL_SPARSE_PCT", "100")
+    n = 1_500_011
+    rng = np.random.default_rng(G + 5)
+    key = rng.integers(0, G, n).astype(np.int64) * 7919 - 3
+    key[::1013] = -1
+    v = rng.integers(-2**31, 2**31, n).astype(np.int64)
+    v[::997] = 2**45 + 1
+    p = rng.integers(0, 1000, n).astype(np.int32)
+    for hi in (9, -1):                               # ~1 %, and nothing selected
+        _check_sga([(p, {"hi": hi})], [key], [v], C5_AGGS, expected_groups=G, bitmap=True,
+                   kernel="k_sga_bulk<Sig pred i32, key i64")
+
+
+@pytest.mark.parametrize("f64", [False, True])
+def test_q1_select_compact_gather(monkeypatch, f64):
+    """The Q1 signatures (private tier) at ~2 % selectivity through the twin."""
+    monkeypatch.setenv("OCL_SPARSE_PCT", "100")
+    li = _lineitem(1_200_007, datagen.BASE_SEED + 8, f64=f64)
+    p, k, v, a = _q1_plan(li, f64)
+    p = [(li["shipdate"], {"hi": 8200})]
+    _check_sga(p, k, v, a, order_by_key=True, kernel=f"k_sga_bulk<Sig Q1 {'fp64' if f64 else 'int64'}>")
+
+
+def test_jit_select_compact_gather(monkeypatch):
+    """A run-time compiled signature (two value columns, CTA table) through its compiled twin."""
+    monkeypatch.setenv("OCL_SPARSE_PCT", "100")
+    n = 900_001
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 5, 300, s=1.0)
+    v2 = (sw["v"] * 3 - 7).astype(np.int64)
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "max", "a": 1}, {"op": "min", "a": 1}]
+    _check_sga([(sw["p"], {"hi": 19_999})], [sw["key"]], [sw["v"], v2], aggs, expected_groups=300,
+               kernel=f"{JIT}; CTA table")
+
+
+def test_c5_sparse_default_threshold():
+    """At 2^24 rows the default threshold (8 %) takes the twin for a 1 % predicate: full oracle compare."""
+    n = (1 << 24) + 77
+    sw = datagen.sweep_host(n, datagen.BASE_SEED + 9, 256, s=1.0)
+    _check_sga([(sw["p"], {"hi": 9_999})], [sw["key"]], [sw["v"]], C5_AGGS, expected_groups=256,
+               kernel="k_sga_bulk<Sig pred i32, key i64, COUNT/SUM/MIN/MAX; CTA table>")

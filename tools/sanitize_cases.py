@@ -109,6 +109,19 @@ def _():
     check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=2000, tier=5)   # hash-partitioned
 
 
+@case("fused_select_compact_gather")
+def _():
+    os.environ["OCL_SPARSE_PCT"] = "100"      # k_sga_sparse whenever the sample selects < 100 %
+    try:
+        p = [(sw["p"], {"hi": 19_999})]
+        assert "CTA table" in check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=300)
+        assert "4 private slots" in check_sga(p, [sw["key"] % 3], [sw["v"]], C5AGGS, expected_groups=4)
+        assert "k_sga_bulk<Sig Q1 int64>" in check_sga([(li["shipdate"], {"hi": 8200})], Q1K, Q1V, Q1_AGGS,
+                                                       expected_groups=4)
+    finally:
+        del os.environ["OCL_SPARSE_PCT"]
+
+
 @case("sorted_radix_tier6")
 def _():
     lo = datagen.lineitem_host(50_000, datagen.BASE_SEED + 3)
