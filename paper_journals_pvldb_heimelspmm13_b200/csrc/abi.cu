@@ -471,7 +471,8 @@ ocl_status run_fused(ocl_ctx* ctx, const ocl_sga_args* a, Planned& P, void* ws, 
   if (ws_bytes < need || (!ws && need)) return fail(OCL_ERR_CAPACITY, "workspace %zu B < required %zu B", ws_bytes, need);
   P.plan.table = (uint8_t*)ws;
   *emit_ws = (uint8_t*)ws + P.table_bytes;
-  OCL_CUDA(cudaMemsetAsync(ws, 0, P.table_bytes, s), "table init");
+  if (P.pbits < 0 || P.plan.n == 0)      // the partitioned tier zeroes (only what it uses) itself
+    OCL_CUDA(cudaMemsetAsync(ws, 0, P.table_bytes, s), "table init");
   if (a->dev_status) OCL_CUDA(cudaMemsetAsync(a->dev_status, 0, sizeof(int32_t), s), "status init");
   if (P.plan.n > 0) {
     if (ctx->prof_begin) OCL_CUDA(cudaEventRecord(ctx->prof_begin, s), "profile event");

@@ -13,21 +13,27 @@
 // hash to P = 2^pbits partitions small enough for a shared-memory table:
 //
 //   pass 1a  k_part_count    fused select + key + values, per row-block histogram of
-//                            partition ids (shared-memory counters)
-//   scan     k_scan_*        exclusive scan of the partition counts
-//   pass 1b  k_part_scatter  the same rows again: each qualifying row becomes a
-//                            record {key, int32 values} at its partition's global
-//                            cursor (one atomic per row, or per warp for a hot one)
+//                            partition ids (shared-memory counters); per row block the
+//                            level-1 counts (top b1 = 7 hash bits)
+//   scan     k_scan_*        exclusive scans: partition starts, per-block level-1 ranges
+//   pass 1b  k_part_scatter_l1  the same rows again: each qualifying row becomes a record
+//                            {key, int32 values} in its row block's own range of its
+//                            level-1 partition (block-local cursors, no global claims),
+//                            staged per tile in shared memory and written as runs;
+//            k_part_scatter2 level-1 records -> final partitions, per tile one global
+//                            claim per partition met (direct-indexed tile map).  With
+//                            <= 2^7 partitions one tiled level (k_part_scatter).
 //   pass 2   k_part_agg      work items of <= kPartItem records of one partition; a
 //                            CTA aggregates an item in a shared-memory hash table
-//                            (32-bit atomics, the CTA-table layout of the fused
-//                            kernel) and merges every entry once into the HBM table
-//                            (plain read-modify-write when the partition is one item)
+//                            (32-bit atomics, field-major) and emits its groups straight
+//                            from shared memory (or merges them into the HBM table)
 //
 // The HBM table's start slot is the top bits of the key hash (common.cuh), so a
-// partition's keys occupy one contiguous slot range: pass-2 merges stay L2-local.
-// Rows the fast path cannot take (values outside int32, the key ~0) and records
-// whose partition overflows the shared table update the HBM table directly (exact).
+// partition's keys occupy one contiguous slot range (its region).  The table is zeroed
+// lazily: only regions that receive entries (exact-path rows, split or overflowing
+// partitions) are cleared.  Rows the fast path cannot take (values outside int32, the
+// key ~0) and records whose partition overflows the shared table update the HBM table
+// directly (exact).
 #include <string.h>
 
 #include "launch.cuh"
@@ -55,11 +61,17 @@ struct PartArgs {
   uint32_t* counts;     // [P] histogram of partition ids
   uint32_t* offs;       // [P] exclusive scan of counts: partition starts
   uint32_t* cur;        // [P] global write cursors of pass 1b (start = offs)
+  uint32_t* curp;       // [P << curp_shift] the same, one per 2^curp_shift words (one-level scatter:
+  int32_t curp_shift;   //   a cursor per L2 sector / line, so claims on different partitions do not queue)
   uint32_t* sums;       // scan chunk sums
   int64_t* m_dev;       // number of records
   uint8_t* recs;        // records: {key u64, int32 value x NV}, rec_bytes each, grouped by partition
   uint8_t* tmp;         // level-1 records (two-level scatter), grouped by the top b1 hash bits
   uint32_t* cur1;       // [2^b1] level-1 cursors
+  uint32_t* cnt1;       // [2^b1][nblk] level-1 counts per row block (count pass), then their
+                        // exclusive scan: each block's own range in every level-1 partition
+  uint32_t* sums1;      // scan chunk sums of cnt1
+  int32_t b1;           // level-1 bits (two-level scatter)
   uint32_t* icnt;       // [P] pass-2 work items per partition
   uint32_t* ioff;       // [P] exclusive scan of icnt
   uint32_t* isums;      // scan chunk sums of icnt
@@ -71,6 +83,11 @@ struct PartArgs {
   // their output rows (final or partial) straight from there; the others mark dirty[q] and
   // are emitted from their HBM slot range afterwards — no pass over the whole table.
   int32_t direct_emit;
+  // lazy = 1: the caller did not zero the HBM table; k_part_zero_regions clears the regions
+  // known to be used before pass 1b, a partition whose shared table overflows clears its own
+  // region and re-aggregates its item there (requires direct_emit).
+  int32_t lazy;
+  int32_t mm_check;     // pass 2: MIN / MAX read-before-atomic
   int32_t npo;                     // final outputs, resolved on the host (kind, CTA-entry fields, pointer)
   struct { int32_t kind, f0, f1, pad; void* out; } po[kMaxAggs];
   uint32_t* dirty;                 // [P]
@@ -182,6 +199,8 @@ __global__ void __launch_bounds__(kPartThreads) k_part_count(const __grid_consta
       const uint32_t part = ok[k] ? part_of((uint64_t)x[k].key, a.pbits) : 0xFFFFFFFFu;
       const uint32_t p0 = __shfl_sync(0xffffffffu, part, 0);
       const unsigned same = __ballot_sync(0xffffffffu, ok[k] && part == p0);
+      if (x[k].q && !ok[k] && (uint64_t)x[k].key != ~0ULL)   // exact-path row: its region is used
+        a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;
       if (ok[k] && part != p0) atomicAdd(&hist[part], 1u);
       if (lane == 0 && same) atomicAdd(&hist[p0], (uint32_t)__popc(same));
     }
@@ -189,6 +208,14 @@ __global__ void __launch_bounds__(kPartThreads) k_part_count(const __grid_consta
   __syncthreads();
   for (int i = threadIdx.x; i < P; i += blockDim.x)
     if (hist[i]) atomicAdd(&a.counts[i], hist[i]);
+  if (a.cnt1) {                            // two-level scatter: this block's level-1 counts
+    const int P1 = 1 << a.b1, w = 1 << (a.pbits - a.b1);
+    for (int t = threadIdx.x; t < P1; t += blockDim.x) {
+      uint32_t c = 0;
+      for (int i = 0; i < w; ++i) c += hist[t * w + i];
+      a.cnt1[(size_t)t * a.nblk + blockIdx.x] = c;
+    }
+  }
 }
 
 // ------------------------------------------------------------------ pass 1b: scatter
@@ -289,6 +316,40 @@ __device__ __forceinline__ void tile_map_claim(TileMap& m, uint32_t* cur, uint32
   if (t == 0) m.total = run0;
 }
 
+// Direct-indexed variant (slot i = partition qb + i, i < width): the same claim over every
+// slot of the range instead of the used list.
+constexpr uint32_t kDirectMap = 1024;
+__device__ __forceinline__ void tile_dmap_claim(TileMap& m, uint32_t width, uint32_t qb, uint32_t* cur,
+                                                uint32_t* wsum) {
+  const int t = threadIdx.x, lane = t & 31, w = t >> 5;
+  uint32_t run0 = 0;
+  for (uint32_t b0 = 0; b0 < width; b0 += kPartThreads) {
+    const uint32_t i = b0 + t;
+    const uint32_t c = i < width ? m.cnt[i] : 0u;
+    uint32_t incl = c;
+#pragma unroll
+    for (int o = 1; o < 32; o <<= 1) {
+      const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+      if (lane >= o) incl += y;
+    }
+    if (lane == 31) wsum[w] = incl;
+    __syncthreads();
+    uint32_t off = 0, tot = 0;
+#pragma unroll
+    for (int k = 0; k < kPartThreads / 32; ++k) {
+      off += k < w ? wsum[k] : 0u;
+      tot += wsum[k];
+    }
+    if (i < width) {
+      m.off[i] = run0 + off + incl - c;
+      m.cnt[i] = c ? atomicAdd(&cur[qb + i], c) : 0u;
+    }
+    run0 += tot;
+    __syncthreads();
+  }
+  if (t == 0) m.total = run0;
+}
+
 // Stage item (slot, rank) in the tile's partition-grouped order.
 __device__ __forceinline__ void tile_stage(TileMap& m, uint32_t slot, uint32_t rank, uint4 rec) {
   const uint32_t i = m.off[slot] + rank;
@@ -335,7 +396,7 @@ __device__ __forceinline__ void load_rec(const uint8_t* rec, uint64_t& key, int3
 
 // Level 1: rows -> records grouped by the top `pb` hash bits (cursors `cur`, output `out`).
 template <class Sh, int NV>
-__global__ void __launch_bounds__(kPartThreads) k_part_scatter(const __grid_constant__ Plan p, PartArgs a, int pb,
+__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter(const __grid_constant__ Plan p, PartArgs a, int pb,
                                                                uint32_t* cur, uint8_t* out) {
   extern __shared__ __align__(16) uint8_t dsm[];
   TileMap& map = *(TileMap*)dsm;
@@ -393,11 +454,282 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter(const __grid_cons
   }
 }
 
+// One level, no tiles: every qualifying row claims its record position with one returning
+// atomic on its partition's cursor (lanes sharing lane 0's partition — hot keys — take one
+// atomic of lane 0) and stores its 16-byte record there.  No barriers or shared-memory
+// maps: the claims of kPartILP rows are in flight together, and the next rows' loads are
+// issued before this group's claims return.  The P cursors keep one partially written
+// line per partition open in L2 (P x 128 B = 2 MB at 2^14 partitions), so the scattered
+// 16-byte stores still leave L2 as whole sectors.
+// PF: the next rows' loads are issued before this group's claims (1 CTA / SM); otherwise
+// RG groups of kPartILP rows per thread are loaded, then all their claims issued (2 CTAs / SM).
+template <class Sh, int NV, bool PF, int RG>
+__global__ void __launch_bounds__(kPartThreads, PF ? 1 : 2) k_part_scatter_direct(const __grid_constant__ Plan p, PartArgs a) {
+  constexpr int R = kPartILP * RG;
+  const int64_t r0 = blockIdx.x * a.rows_per_blk;
+  const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = lanemask_lt();
+  const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
+  Row<Sh, NV, false> nx[PF ? kPartILP : 1];
+  bool nok[PF ? kPartILP : 1];
+  if constexpr (PF)
+    if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
+  for (int64_t base0 = r0; base0 < r1; base0 += R * blockDim.x) {
+    Row<Sh, NV, false> x[R];
+    bool ok[R];
+    const int64_t wbase0 = base0 + woff;
+    if constexpr (PF) {
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k) {
+        x[k] = nx[k];
+        ok[k] = nok[k];
+      }
+      if (base0 + kPartILP * blockDim.x < r1) part_rows<Sh, NV>(p, wbase0 + kPartILP * blockDim.x, r1, lane, nx, nok);
+    } else {
+#pragma unroll
+      for (int g = 0; g < RG; ++g) {
+        Row<Sh, NV, false> y[kPartILP];
+        bool yk[kPartILP];
+        part_rows<Sh, NV>(p, wbase0 + (int64_t)g * kPartILP * blockDim.x, r1, lane, y, yk);
+#pragma unroll
+        for (int k = 0; k < kPartILP; ++k) {
+          x[g * kPartILP + k] = y[k];
+          ok[g * kPartILP + k] = yk[k];
+        }
+      }
+    }
+    uint32_t part[R], ret[R];
+    unsigned same[R];
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      part[k] = ok[k] ? part_of((uint64_t)x[k].key, a.pbits) : 0xFFFFFFFFu;
+      const uint32_t p0 = __shfl_sync(0xffffffffu, part[k], 0);
+      same[k] = __ballot_sync(0xffffffffu, ok[k] && part[k] == p0);
+      ret[k] = 0;
+      if (ok[k] && (lane == 0 || part[k] != p0))
+        ret[k] = atomicAdd(&a.curp[(size_t)part[k] << a.curp_shift], lane == 0 ? (uint32_t)__popc(same[k]) : 1u);
+    }
+#pragma unroll
+    for (int k = 0; k < R; ++k) {
+      const uint32_t b0 = __shfl_sync(0xffffffffu, ret[k], 0);
+      if (x[k].q && !ok[k]) {               // exact per-row path straight into the HBM table
+        uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
+        if (e) update_entry_slow(p, e, part_row(wbase0 + (int64_t)(k / kPartILP) * kPartILP * blockDim.x, lane, k % kPartILP));
+        if ((uint64_t)x[k].key != ~0ULL) a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;
+      }
+      if (!ok[k]) continue;
+      const uint32_t pos = (same[k] >> lane) & 1u ? b0 + (uint32_t)__popc(same[k] & lt) : ret[k];
+      int32_t v[NV > 0 ? NV : 1];
+#pragma unroll
+      for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
+      if constexpr (NV <= 2) *(uint4*)(a.recs + (size_t)pos * 16) = pack_rec16<NV>((uint64_t)x[k].key, v);
+      else store_rec<NV>(a.recs + (size_t)pos * a.rec_bytes, (uint64_t)x[k].key, v);
+    }
+  }
+}
+
+// The same scatter as a three-stage software pipeline over tiles of kPartILP rows per
+// thread: iteration i issues the loads of tile i + 1, the claims of tile i (whose rows
+// arrived during iteration i - 1) and the record stores of tile i - 1 (whose claims were
+// issued in iteration i - 1).  Every wait then covers one load and one claim latency: the
+// one-stage kernel above was latency-bound (ncu: long-scoreboard stalls on the key loads
+// and on the claim results, L2 at 37 % of its throughput, one CTA of 16 warps per SM).
+// Records of NV <= 2 values only (16 bytes).
+// One pipeline stage: tile `base` (rows x, arrived) claims into set C; set P (the previous
+// tile's records and claims) is stored; the next tile's loads were issued by the caller.
+// C and P alternate between two register sets (the loop is unrolled by two), so no claim
+// result is moved between registers before it is used: a move would wait for it.
+struct PipeSet {
+  uint4 rec[kPartILP];
+  uint32_t ret[kPartILP];
+  unsigned same[kPartILP];
+  bool ok[kPartILP];
+};
+
+template <class Sh, int NV>
+__device__ __forceinline__ void pipe_stage(const Plan& p, const PartArgs& a, int64_t wbase, bool have,
+                                           const Row<Sh, NV, false> (&x)[kPartILP], const bool (&xok)[kPartILP],
+                                           PipeSet& C, const PipeSet& P, int lane, uint32_t lt) {
+#pragma unroll
+  for (int k = 0; k < kPartILP; ++k) {
+    const bool ok = have && xok[k];
+    const uint32_t part = ok ? part_of((uint64_t)x[k].key, a.pbits) : 0xFFFFFFFFu;
+    const uint32_t p0 = __shfl_sync(0xffffffffu, part, 0);
+    C.same[k] = __ballot_sync(0xffffffffu, ok && part == p0);
+    C.ret[k] = 0;
+    if (ok && (lane == 0 || part != p0))
+      C.ret[k] = atomicAdd(&a.curp[(size_t)part << a.curp_shift], lane == 0 ? (uint32_t)__popc(C.same[k]) : 1u);
+    C.ok[k] = ok;
+    if (have && x[k].q && !ok) {           // exact per-row path straight into the HBM table
+      uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
+      if (e) update_entry_slow(p, e, part_row(wbase, lane, k));
+      if ((uint64_t)x[k].key != ~0ULL) a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;
+    }
+    int32_t v[NV > 0 ? NV : 1];
+#pragma unroll
+    for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
+    C.rec[k] = pack_rec16<NV>((uint64_t)x[k].key, v);
+  }
+#pragma unroll
+  for (int k = 0; k < kPartILP; ++k) {     // stores of the previous tile
+    const uint32_t b0 = __shfl_sync(0xffffffffu, P.ret[k], 0);
+    if (P.ok[k]) {
+      const uint32_t pos = (P.same[k] >> lane) & 1u ? b0 + (uint32_t)__popc(P.same[k] & lt) : P.ret[k];
+      *(uint4*)(a.recs + (size_t)pos * 16) = P.rec[k];
+    }
+  }
+}
+
+// The one-level scatter as a three-stage software pipeline over tiles of kPartILP rows per
+// thread: a stage issues the loads of tile i + 1, the claims of tile i (whose rows arrived
+// during stage i - 1) and the record stores of tile i - 1 (whose claims were issued in
+// stage i - 1).  Every wait then covers one load and one claim latency: the one-stage kernel
+// above is latency-bound (ncu: long-scoreboard stalls on the key loads and on the claim
+// results, L2 at 37 % of its throughput, one CTA of 16 warps per SM).  16-byte records.
+template <class Sh, int NV>
+__global__ void __launch_bounds__(kPartThreads, 1) k_part_scatter_pipe(const __grid_constant__ Plan p, PartArgs a) {
+  static_assert(NV <= 2, "16-byte records");
+  const int64_t r0 = blockIdx.x * a.rows_per_blk;
+  const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
+  const int lane = threadIdx.x & 31;
+  const uint32_t lt = lanemask_lt();
+  const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
+  const int64_t step = kPartILP * blockDim.x;
+  Row<Sh, NV, false> xa[kPartILP], xb[kPartILP];
+  bool oka[kPartILP], okb[kPartILP];
+  PipeSet A, B;
+#pragma unroll
+  for (int k = 0; k < kPartILP; ++k) B.ok[k] = false;
+  if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, xa, oka);
+  // stage order per pair: (tile in xa -> A, stores B), (tile in xb -> B, stores A)
+  for (int64_t base = r0; base < r1; base += 2 * step) {
+    if (base + step < r1) part_rows<Sh, NV>(p, base + step + woff, r1, lane, xb, okb);
+    pipe_stage<Sh, NV>(p, a, base + woff, true, xa, oka, A, B, lane, lt);
+    const bool h1 = base + step < r1;
+    if (base + 2 * step < r1) part_rows<Sh, NV>(p, base + 2 * step + woff, r1, lane, xa, oka);
+    pipe_stage<Sh, NV>(p, a, base + step + woff, h1, xb, okb, B, A, lane, lt);
+  }
+  // drain: the last stage claimed into B (a pair always ends with B)
+#pragma unroll
+  for (int k = 0; k < kPartILP; ++k) {
+    const uint32_t b0 = __shfl_sync(0xffffffffu, B.ret[k], 0);
+    if (B.ok[k]) {
+      const uint32_t pos = (B.same[k] >> lane) & 1u ? b0 + (uint32_t)__popc(B.same[k] & lt) : B.ret[k];
+      *(uint4*)(a.recs + (size_t)pos * 16) = B.rec[k];
+    }
+  }
+}
+
+__global__ void k_part_cur_pad(const uint32_t* offs, uint32_t* curp, int shift, int64_t L) {
+  const int64_t i = blockIdx.x * (int64_t)blockDim.x + threadIdx.x;
+  if (i < L) curp[i << shift] = offs[i];
+}
+
+// Lazily zeroed HBM table (PartArgs::lazy): only the regions that will hold entries are
+// cleared — partitions with exact-path rows (slowflag, set by the count pass) and
+// partitions split over several pass-2 work items.  One CTA per partition.
+__global__ void k_part_zero_regions(const __grid_constant__ Plan p, PartArgs a) {
+  const int64_t q = blockIdx.x;
+  const int64_t m = *a.m_dev;
+  const int64_t n = (q + 1 >= (1LL << a.pbits) ? m : (int64_t)a.offs[q + 1]) - (int64_t)a.offs[q];
+  if (!a.slowflag[q] && n <= kPartItem) return;             // CTA-uniform
+  uint4* r = (uint4*)(p.table + ((size_t)q << kPartCapBits) * p.stride);
+  const int nq = (int)(((size_t)p.stride << kPartCapBits) / 16);
+  for (int i = threadIdx.x; i < nq; i += blockDim.x) r[i] = make_uint4(0, 0, 0, 0);
+}
+
+// Level 1 with per-block ranges: rows -> records grouped by the top b1 hash bits (2^b1 <=
+// 256 partitions).  The count pass left each row block's level-1 counts and their scan
+// (a.cnt1: block c's range in level-1 partition t starts at cnt1[t][c]), so the block
+// advances its own cursors in shared memory: no global claims, and a block keeps only
+// 2^b1 partially written lines open in L2.  Per tile: ranks by shared atomics on the
+// 2^b1 counters, one scan, records staged in partition order and written as runs.
+template <class Sh, int NV>
+__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a) {
+  extern __shared__ __align__(16) uint8_t dsm[];
+  TileMap& m = *(TileMap*)dsm;            // cnt / off / key (= block cursor) used for 2^b1 slots
+  __shared__ uint32_t wsum[32];
+  const int P1 = 1 << a.b1;
+  const int64_t r0 = blockIdx.x * a.rows_per_blk;
+  const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
+  const int lane = threadIdx.x & 31, t = threadIdx.x, w = t >> 5;
+  for (int i = t; i < P1; i += blockDim.x) {
+    m.cnt[i] = 0;
+    m.key[i] = a.cnt1[(size_t)i * a.nblk + blockIdx.x];
+  }
+  Row<Sh, NV, false> nx[kPartILP];
+  bool nok[kPartILP];
+  const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
+  if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
+  __syncthreads();
+  for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
+    Row<Sh, NV, false> x[kPartILP];
+    bool ok[kPartILP];
+    uint32_t q[kPartILP], rank[kPartILP];
+    const int64_t wbase = base + woff;
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      x[k] = nx[k];
+      ok[k] = nok[k];
+    }
+    if (base + kPartILP * blockDim.x < r1) part_rows<Sh, NV>(p, wbase + kPartILP * blockDim.x, r1, lane, nx, nok);
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      if (x[k].q && !ok[k]) {               // exact per-row path straight into the HBM table
+        uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
+        if (e) update_entry_slow(p, e, part_row(wbase, lane, k));
+        if ((uint64_t)x[k].key != ~0ULL) a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;
+      }
+      q[k] = ok[k] ? part_of((uint64_t)x[k].key, a.b1) : 0u;
+      if (ok[k]) rank[k] = atomicAdd(&m.cnt[q[k]], 1u);
+    }
+    __syncthreads();
+    // offsets in the staging area (exclusive scan of the <= 256 counts) and global bases
+    {
+      const uint32_t c = t < P1 ? m.cnt[t] : 0u;
+      uint32_t incl = c;
+#pragma unroll
+      for (int o = 1; o < 32; o <<= 1) {
+        const uint32_t y = __shfl_up_sync(0xffffffffu, incl, o);
+        if (lane >= o) incl += y;
+      }
+      if (lane == 31 && w < 8) wsum[w] = incl;
+      __syncthreads();
+      if (t < P1) {
+        uint32_t off = 0;
+        for (int k = 0; k < w; ++k) off += wsum[k];
+        m.off[t] = off + incl - c;
+        const uint32_t g = m.key[t];
+        m.key[t] = g + c;                    // block cursor
+        m.cnt[t] = g;                        // this tile's global base
+        if (t == P1 - 1) m.total = off + incl;
+      }
+    }
+    __syncthreads();
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k) {
+      if (!ok[k]) continue;
+      int32_t v[NV > 0 ? NV : 1];
+#pragma unroll
+      for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
+      if constexpr (NV <= 2) tile_stage(m, q[k], rank[k], pack_rec16<NV>((uint64_t)x[k].key, v));
+      else store_rec<NV>(a.tmp + (size_t)(m.cnt[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
+    }
+    __syncthreads();
+    if constexpr (NV <= 2) tile_flush(m, m.total, a.tmp, a.rec_bytes);
+    __syncthreads();
+    for (int i = t; i < P1; i += blockDim.x) m.cnt[i] = 0;
+    // (the next tile's atomics on m.cnt come after the next barrier-free stretch: order them)
+    __syncthreads();
+  }
+}
+
 // Level 2: records grouped by their top b1 hash bits -> records grouped by all pbits.
 // A tile of consecutive level-1 records spans one or two level-1 partitions, so it
 // meets at most ~2^(pbits-b1) final partitions: the tile claims aggregate again.
 template <int NV>
-__global__ void __launch_bounds__(kPartThreads) k_part_scatter2(PartArgs a) {
+__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
   extern __shared__ __align__(16) uint8_t dsm[];
   TileMap& map = *(TileMap*)dsm;
   __shared__ uint32_t wsum[32];
@@ -431,12 +763,30 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter2(PartArgs a) {
       for (int i = 0; i < NV; ++i) v[k][i] = nv[k][i];
     }
     if (base + TILE < j1) fetch(base + TILE);
+    // the tile's final partitions lie in [qb, qb + width): its first and last record's
+    // level-1 partitions bound them (level-1 records are in level-1 order)
+    const int sh = a.pbits - a.b1;
+    const uint32_t q1f = part_of(*(const uint64_t*)(a.tmp + (size_t)base * a.rec_bytes), a.b1);
+    const uint32_t q1l = part_of(*(const uint64_t*)(a.tmp + (size_t)(min(base + TILE, j1) - 1) * a.rec_bytes), a.b1);
+    const uint32_t qb = q1f << sh, width = (q1l - q1f + 1) << sh;
+    const bool dmap = a.b1 > 0 && width <= kDirectMap;       // CTA-uniform
     __syncthreads();
+    if (dmap) {                           // direct-indexed map: no hashing, no key slots
 #pragma unroll
-    for (int k = 0; k < kPartILP; ++k)
-      if (ok[k]) tile_map_add(map, part_of(key[k], a.pbits), slot[k], rank[k]);
-    __syncthreads();
-    tile_map_claim(map, a.cur, wsum);
+      for (int k = 0; k < kPartILP; ++k)
+        if (ok[k]) {
+          slot[k] = part_of(key[k], a.pbits) - qb;
+          rank[k] = atomicAdd(&map.cnt[slot[k]], 1u);
+        }
+      __syncthreads();
+      tile_dmap_claim(map, width, qb, a.cur, wsum);
+    } else {
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k)
+        if (ok[k]) tile_map_add(map, part_of(key[k], a.pbits), slot[k], rank[k]);
+      __syncthreads();
+      tile_map_claim(map, a.cur, wsum);
+    }
     __syncthreads();
 #pragma unroll
     for (int k = 0; k < kPartILP; ++k) {
@@ -449,6 +799,8 @@ __global__ void __launch_bounds__(kPartThreads) k_part_scatter2(PartArgs a) {
       tile_flush(map, map.total, a.recs, a.rec_bytes);
       __syncthreads();
     }
+    if (dmap)                             // (ordered before the next tile's adds by the reset barrier)
+      for (uint32_t i = threadIdx.x; i < width; i += blockDim.x) map.cnt[i] = 0;
   }
 }
 
@@ -597,9 +949,16 @@ __device__ __forceinline__ void part_cos(const Plan& p, int i, int& lo, int& mn,
   }
 }
 
+// MIN / MAX field update; mmc: read first and skip the atomic when the value cannot improve
+// (the field only grows, so a stale read can only cause an unneeded atomic).
+__device__ __forceinline__ void part_max(uint32_t* f, uint32_t x, bool mmc) {
+  if (!mmc || *(volatile uint32_t*)f < x) atomicMax(f, x);
+}
+
 // One record into slot `slot`.
 template <int NV, bool FIX>
-__device__ __forceinline__ void part_add(const Plan& p, uint8_t* tab, int slot, const int32_t (&v)[NV > 0 ? NV : 1]) {
+__device__ __forceinline__ void part_add(const Plan& p, uint8_t* tab, int slot, const int32_t (&v)[NV > 0 ? NV : 1],
+                                         bool mmc) {
   atomicAdd(pf32(tab, slot, 8), 1u);
 #pragma unroll
   for (int i = 0; i < NV; ++i) {
@@ -607,8 +966,8 @@ __device__ __forceinline__ void part_add(const Plan& p, uint8_t* tab, int slot, 
     int lo, mn, mx;
     part_cos<FIX>(p, i, lo, mn, mx);
     if (lo >= 0) part_add_sum(tab, slot, lo, (uint64_t)((uint32_t)v[i] ^ 0x80000000u));
-    if (mn >= 0) atomicMax(pf32(tab, slot, mn), enc32_min(v[i]));
-    if (mx >= 0) atomicMax(pf32(tab, slot, mx), enc32_max(v[i]));
+    if (mn >= 0) part_max(pf32(tab, slot, mn), enc32_min(v[i]), mmc);
+    if (mx >= 0) part_max(pf32(tab, slot, mx), enc32_max(v[i]), mmc);
   }
 }
 
@@ -776,8 +1135,13 @@ __device__ __forceinline__ void part_emit_row(const Plan& p, const PartArgs& a, 
   }
 }
 
+#ifndef OCL_AGG_BLOCKS
+#define OCL_AGG_BLOCKS 3
+#endif
+constexpr int kAggBlocks = OCL_AGG_BLOCKS;     // CTAs per SM of pass 2 (shared table 64 KB each)
+
 template <int NV, bool FIX>
-__global__ void __launch_bounds__(kPartThreads, 2) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
+__global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
                                                               const __grid_constant__ EmitArgs ea) {
   extern __shared__ __align__(16) uint8_t tab[];
   __shared__ int overflowed;
@@ -832,16 +1196,31 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_agg(const __grid_const
         if (!valid[k]) continue;
         const int ts = part_find(tab, key[k], direct, a.pbits);
         if (ts >= 0) {
-          part_add<NV, FIX>(p, tab, ts, v[k]);
+          part_add<NV, FIX>(p, tab, ts, v[k], a.mm_check != 0);
         } else {
           overflowed = 1;
+          if (a.lazy && direct) continue;                      // region not zeroed yet: redone below
           uint8_t* ge = table_find_or_insert(p.table, p.mask, p.stride, key[k], p.status);
           if (ge) update_entry_rec(p, ge, v[k], p.nvals);
         }
       }
     }
     __syncthreads();
-    if (direct && !overflowed && a.direct_emit) {               // the rows straight from shared memory
+    if (a.lazy && direct && overflowed) {
+      // shared table overflowed in a partition whose HBM region was left dirty: this CTA is
+      // the only one touching the region — clear it and aggregate the whole item there
+      uint4* r = (uint4*)(p.table + ((size_t)lo << kPartCapBits) * p.stride);
+      const int nq = (int)(((size_t)p.stride << kPartCapBits) / 16);
+      for (int i = threadIdx.x; i < nq; i += blockDim.x) r[i] = make_uint4(0, 0, 0, 0);
+      __syncthreads();
+      for (int64_t j = s + threadIdx.x; j < seg_end; j += blockDim.x) {
+        uint64_t key;
+        int32_t v[NV > 0 ? NV : 1];
+        load_rec<NV>(a.recs + (size_t)j * a.rec_bytes, key, v);
+        uint8_t* ge = table_find_or_insert(p.table, p.mask, p.stride, key, p.status);
+        if (ge) update_entry_rec(p, ge, v, p.nvals);
+      }
+    } else if (direct && !overflowed && a.direct_emit) {               // the rows straight from shared memory
       constexpr int PER = kPartCap / kPartThreads;
       uint32_t occ = 0;
 #pragma unroll
@@ -913,6 +1292,17 @@ using PShK64 = StaticShape<0, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF
 using PShP32K64 = StaticShape<4, false, 8, 0, 1, false, vop(0, VF_SUM | VF_MIN | VF_MAX, 0)>;
 
 static int part_rec_bytes(int nv) { return nv <= 2 ? 16 : 32; }
+
+// Pass 1b: 5 = two levels above 2^kPartLevelBits partitions, level 1 into per-block ranges
+// (k_part_scatter_l1), level 2 by tiles with direct-indexed maps (default; one tiled level
+// below); 0 = one-level scatter with per-row claims, three-stage pipeline (16-byte
+// records, else as 4); 4 = one-level, next rows prefetched; 2 / 3 = one-level without the
+// prefetch at two CTAs per SM, 4 / 8 rows per thread; 1 = tiled scatter, two levels above
+// 2^kPartLevelBits partitions (OCL_PSCAT=1; the round-1/2 design, kept for A/B).
+static int part_scatter_mode() {
+  const char* e = getenv("OCL_PSCAT");
+  return e ? atoi(e) : 5;
+}
 static size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 
 int part_bits_for(int64_t expected_groups) {
@@ -935,11 +1325,12 @@ bool part_eligible(const Plan& p) {
 }
 
 size_t part_ws_bytes(const Plan& p, int pbits, int sms) {
-  (void)sms;
   const int64_t L = 1LL << pbits;
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   const bool two = pbits > kPartLevelBits;
-  return align_up((size_t)L * 4, 256) * 7 + align_up((size_t)nchunks * 4, 256) * 2 + 768 +
+  const size_t n1 = ((size_t)1 << kPartLevelBits) * (size_t)sms * 4;   // level-1 counts per row block (nblk <= 4 sms)
+  return align_up((size_t)L * 4, 256) * 7 + align_up((size_t)L * 128, 256) + align_up((size_t)nchunks * 4, 256) * 2 + 768 +
+         align_up(n1 * 4, 256) + align_up((n1 / kScanChunk + 1) * 4, 256) +
          align_up((size_t)p.n * part_rec_bytes(p.nvals), 256) * (two ? 2 : 1) + (two ? align_up(4u << kPartLevelBits, 256) : 0);
 }
 
@@ -964,17 +1355,41 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
     if ((e = cudaMemsetAsync(a.dirty, 0, (size_t)L * 4, s))) return e;
     if ((e = cudaMemsetAsync(a.out_ctr, 0, 8, s))) return e;
   }
+  a.b1 = std::min(a.pbits, kPartLevelBits);
+  if (part_scatter_mode() != 5 || a.pbits <= kPartLevelBits) a.cnt1 = nullptr;
   count_launch(5);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
   k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
   k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums, nchunks, a.m_dev);
   k_scan_add<<<(int)((L + 255) / 256), 256, 0, s>>>(a.offs, a.cur, a.sums, L);
-  const int b1 = std::min(a.pbits, kPartLevelBits), b2 = a.pbits - b1;
+  if (a.lazy) {
+    count_launch();
+    k_part_zero_regions<<<(int)L, 256, 0, s>>>(p, a);
+  }
+  const int b1 = a.b1, b2 = a.pbits - b1;
   const size_t msm = sizeof(TileMap);
   auto ks2 = k_part_scatter2<NV>;
+  auto kl1 = k_part_scatter_l1<Sh, NV>;
   if ((e = cudaFuncSetAttribute(ks, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
   if ((e = cudaFuncSetAttribute(ks2, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
-  if (b2 == 0) {
+  if ((e = cudaFuncSetAttribute(kl1, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
+  const int smode = part_scatter_mode();
+  if (a.cnt1) {                           // two levels, level 1 into per-block ranges
+    const int64_t n1 = ((int64_t)1 << b1) * a.nblk, nc1 = (n1 + kScanChunk - 1) / kScanChunk;
+    count_launch(5);
+    k_scan_chunks<<<(int)nc1, kScanThreads, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
+    k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums1, nc1, a.nitems_dev);     // (total unused; rewritten below)
+    k_scan_add<<<(int)((n1 + 255) / 256), 256, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
+    kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a);
+    ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
+  } else if (smode != 1 && smode != 5) {
+    count_launch(2);
+    k_part_cur_pad<<<(int)((L + 255) / 256), 256, 0, s>>>(a.offs, a.curp, a.curp_shift, L);
+    if (smode == 0 && NV <= 2) k_part_scatter_pipe<Sh, NV <= 2 ? NV : 2><<<a.nblk, kPartThreads, 0, s>>>(p, a);
+    else if (smode == 0 || smode == 4) k_part_scatter_direct<Sh, NV, true, 1><<<a.nblk, kPartThreads, 0, s>>>(p, a);
+    else if (smode == 2) k_part_scatter_direct<Sh, NV, false, 1><<<a.nblk, kPartThreads, 0, s>>>(p, a);
+    else k_part_scatter_direct<Sh, NV, false, 2><<<a.nblk, kPartThreads, 0, s>>>(p, a);
+  } else if (b2 == 0) {
     ks<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.pbits, a.cur, a.recs);
   } else {
     count_launch(3);
@@ -1001,7 +1416,8 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   return cudaGetLastError();
 }
 
-// Run the partitioned tier for plan p (p.table zeroed by the caller).  *kind reports
+// Run the partitioned tier for plan p (p.table NOT zeroed by the caller: done here, fully or
+// lazily; p.n > 0).  *kind reports
 // the shape (30 dynamic, 31 key i64, 32 pred i32 + key i64).
 cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cudaStream_t s, int* kind,
                                const EmitArgs* ea, int64_t* count_out, int64_t out_capacity, bool* emitted) {
@@ -1048,9 +1464,23 @@ cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cuda
   }
   a.dirty = (uint32_t*)w;
   w += align_up((size_t)L * 4, 256);
+  a.curp = (uint32_t*)w;
+  w += align_up((size_t)L * 128, 256);
+  {
+    const size_t n1 = ((size_t)1 << kPartLevelBits) * (size_t)sms * 4;
+    a.cnt1 = (uint32_t*)w;
+    w += align_up(n1 * 4, 256);
+    a.sums1 = (uint32_t*)w;
+    w += align_up((n1 / kScanChunk + 1) * 4, 256);
+  }
+  a.curp_shift = 0;                                     // packed (padding to a sector or line measured slower)
+  if (const char* cp = getenv("OCL_CURPAD")) a.curp_shift = std::min(5, std::max(0, atoi(cp)));
   a.out_ctr = (unsigned long long*)w;
   a.count_out = count_out;
   a.direct_emit = (ea && count_out && a.direct_ok && p.stride <= 256) ? 1 : 0;
+  a.lazy = 0;
+  a.mm_check = 0;                                       // C3 uniform: 3.09 (on) -> 3.02 ms (off)
+  if (const char* mc = getenv("OCL_MM_CHECK")) a.mm_check = atoi(mc) != 0;
   EmitArgs none;
   memset(&none, 0, sizeof(none));
   const EmitArgs& e = ea ? *ea : none;
@@ -1082,6 +1512,16 @@ cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cuda
     }
   }
   if (emitted) *emitted = a.direct_emit != 0;
+  // The HBM table (cap + 1 entries; the caller leaves it unzeroed): with direct emission only
+  // the regions that receive entries are cleared on the device (k_part_zero_regions, the
+  // overflow branch of k_part_agg) and the side entry here; otherwise all of it.
+  a.lazy = a.direct_emit && getenv("OCL_PART_EAGER") == nullptr ? 1 : 0;
+  {
+    const size_t tb = (size_t)(p.mask + 2) * p.stride;
+    cudaError_t ze = a.lazy ? cudaMemsetAsync(p.table + (size_t)(p.mask + 1) * p.stride, 0, p.stride, s)
+                            : cudaMemsetAsync(p.table, 0, tb, s);
+    if (ze) return ze;
+  }
   if (p.vec_ok && p.nkeys == 1 && p.npreds == 0 && values_match<PShK64>(p) && p.keys[0].col.width == 8) {
     *kind = 31;
     return part_run<PShK64, 1>(p, a, sms, s, e, out_capacity);

@@ -192,12 +192,13 @@ def ran_kernel():
 
 
 def _check_sga(preds, keys, vals, aggs, expected_groups=4, tier=0, order_by_key=False, bitmap=False, rtol=1e-9,
-               kernel=None):
+               kernel=None, out_capacity=None):
     """Fused call vs oracle.sga; kernel (substring) asserts which fused kernel ran, so a dispatch change
     cannot silently move a test away from the kernel it is meant to cover."""
     k, outs, bm = ocl.select_group_aggregate([(dev(c), s) for c, s in preds], [dev(c) for c in keys],
                                              [dev(c) for c in vals], aggs, expected_groups=expected_groups,
-                                             tier=tier, order_by_key=order_by_key, bitmap=bitmap)
+                                             tier=tier, order_by_key=order_by_key, bitmap=bitmap,
+                                             out_capacity=out_capacity)
     if kernel is not None:
         assert kernel in ran_kernel(), (kernel, ran_kernel())
     rk, routs = oracle.sga(preds, keys, vals, aggs, order_by_key=order_by_key)
@@ -362,6 +363,23 @@ def test_fused_partitioned_edges(n):
     k32 = (x % 5).astype(np.int32)
     _check_sga([], [(key & 0x7FFFFFFF).astype(np.int32), k32], [x], [{"op": "count"}, {"op": "sum", "a": 0}], expected_groups=max(8, n // 2), tier=5)
     _check_sga([(x, {"lo": 5000})], [key], [x], [{"op": "count"}], expected_groups=n + 8, tier=5)   # empty
+
+
+@pytest.mark.parametrize("n,scatter", [(1 << 20, None), (1 << 20, "0"), (1 << 20, "1"), (1 << 20, "2"), (1 << 20, "3"), (1 << 23, None), (1 << 23, "1")])
+def test_fused_partitioned_near_full(n, scatter, monkeypatch):
+    """Tier 5 with ~1.8x the expected groups: 128 partitions of ~1840 keys in 2048-slot shared tables, so
+    probe sequences pass the shared table's limit and partitions overflow into their HBM region.  At 2^20
+    rows every partition is one work item (the lazily zeroed region is cleared by the overflowing CTA);
+    at 2^23 partitions are split over work items (regions cleared before pass 1b).  Every pass-1b
+    scatter mode (OCL_PSCAT: 0 one-level per-row claims, 1 tiled, 2 / 3 one-level without prefetch, 4 / 8 rows)."""
+    if scatter is not None:
+        monkeypatch.setenv("OCL_PSCAT", scatter)
+    rng = np.random.default_rng(n + 17)
+    E = 1 << 17
+    key = rng.integers(0, int(1.8 * E), n).astype(np.int64) * 7919
+    x = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    _check_sga([], [key], [x], aggs, expected_groups=E, tier=5, out_capacity=4 * E, kernel="hash-partitioned")
 
 
 def test_fused_capacity_retry():

@@ -109,6 +109,17 @@ def _():
     check_sga(p, [sw["key"]], [sw["v"]], C5AGGS, expected_groups=2000, tier=5)   # hash-partitioned
 
 
+@case("partitioned_two_level")
+def _():
+    # 256 partitions: level-1 scatter into per-block ranges, level-2 direct-map tiles; ~1.8x the
+    # expected groups, so shared tables overflow into lazily zeroed HBM regions
+    rng = np.random.default_rng(29)
+    n, E = 1 << 20, 1 << 18
+    key = rng.integers(0, int(1.8 * E), n).astype(np.int64) * 7919
+    x = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    assert "partitioned" in check_sga([], [key], [x], C5AGGS, expected_groups=E, tier=5, out_capacity=4 * E)
+
+
 @case("fused_select_compact_gather")
 def _():
     os.environ["OCL_SPARSE_PCT"] = "100"      # k_sga_sparse whenever the sample selects < 100 %
