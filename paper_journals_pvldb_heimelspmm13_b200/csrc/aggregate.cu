@@ -25,6 +25,9 @@
 namespace ocl {
 
 constexpr size_t kAggSmemBudget = 160 * 1024;
+#ifndef OCL_GAGG_R
+#define OCL_GAGG_R 8
+#endif
 
 // Static shapes: the NC distinct value columns of row r were gathered into c[] by the
 // caller (all loads of a thread's R rows are issued before any update).
@@ -84,7 +87,10 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
   // R rows per thread per round: every gid/oid/value load of the R rows is in flight
   // before the first update (the value loads depend on the oid loads: memory-level
   // parallelism, not bandwidth, bounds a one-row-at-a-time gather).
-  constexpr int R = Sh::kStatic ? 8 : 1;      // 8: 7.17 -> 6.49 ms on the Q1 set at 600M rows (16: 9.9)
+  // 8: 7.17 -> 6.49 ms on the Q1 set at 600M rows (16: 9.9).  Also measured (round 2, same box,
+  // 6.48 ms base): R = 4 at 3 CTAs/SM 7.25, R = 4 / 2 at 4 CTAs/SM 8.28 / 8.84, R = 6 at 3 CTAs/SM
+  // 8.14 (spills)
+  constexpr int R = Sh::kStatic ? OCL_GAGG_R : 1;
   constexpr int NCc = Sh::kStatic ? Sh::NC : 1;
   constexpr int64_t kFlushRounds = 256 / R;                   // 2^16 rows per CTA between CTA-tier flushes
   const int64_t per_round = (int64_t)gridDim.x * T * R;
@@ -103,16 +109,21 @@ __global__ void __launch_bounds__(kFusedThreads) k_group_aggregate(const __grid_
     for (int k = 0; k < R; ++k) {
       const int64_t j = base + (int64_t)k * T;
       gk[k] = j < m ? __ldg(p.gids + j) : -1;
-      if (gk[k] >= G) gk[k] = -1;
-      rk[k] = gk[k] >= 0 ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : 0;
+      rk[k] = j < m ? (p.oids ? (int64_t)__ldg(p.oids + j) : j) : -1;
     }
+    // the oid and value loads do not wait for the gid (row j < m has a valid oid): two
+    // dependent round trips (gid || oid -> values) instead of three (gid -> oid -> values):
+    // Q1 set at 600M rows 6.48 -> 5.14 ms
     if constexpr (Sh::kStatic) {
 #pragma unroll
       for (int k = 0; k < R; ++k)
 #pragma unroll
         for (int i = 0; i < NCc; ++i)
-          c[k][i] = gk[k] >= 0 ? (uint64_t)__ldg((const long long*)p.vcols[i].ptr + rk[k]) : 0;
+          c[k][i] = rk[k] >= 0 ? (uint64_t)__ldg((const long long*)p.vcols[i].ptr + rk[k]) : 0;
     }
+#pragma unroll
+    for (int k = 0; k < R; ++k)
+      if (gk[k] >= G) gk[k] = -1;
 #pragma unroll
     for (int k = 0; k < R; ++k) {
       const int32_t g = gk[k];

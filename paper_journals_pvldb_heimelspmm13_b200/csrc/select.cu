@@ -64,41 +64,66 @@ __device__ __forceinline__ bool row_pred_scalar(const SelParams& p, int64_t r) {
   return ok != (bool)p.anti;
 }
 
+// One 1024-row tile whose 16-byte chunks v[] are loaded: lane `lane` gets word `lane`.
 template <int W>
-__global__ void __launch_bounds__(256) k_select_bitmap(const __grid_constant__ SelParams p) {
+__device__ __forceinline__ uint32_t tile_word(const SelParams& p, const uint4 (&v)[2 * W], int lane) {
   constexpr int R = 16 / W;          // rows per 16-byte chunk
   constexpr int K = 32 / R;          // lanes per output word
   constexpr int U = 2 * W;           // chunks per lane per 1024-row tile
+  uint32_t mine = 0;
+#pragma unroll
+  for (int u = 0; u < U; ++u) {
+    uint32_t w = chunk_bits<W>(p, v[u]) << ((lane % K) * R);
+#pragma unroll
+    for (int o = 1; o < K; o <<= 1) w |= __shfl_xor_sync(0xffffffffu, w, o);
+    uint32_t val = __shfl_sync(0xffffffffu, w, (lane % R) * K);
+    if (lane / R == u) mine = val;
+  }
+  return mine;
+}
+
+// M consecutive 1024-row tiles per warp iteration, all their loads in flight first (M = 4
+// for 1-byte columns: 2 chunks per lane per tile alone left too few bytes in flight).
+template <int W, int M>
+__global__ void __launch_bounds__(256) k_select_bitmap(const __grid_constant__ SelParams p) {
+  constexpr int U = 2 * W;
   const int lane = threadIdx.x & 31;
   const int64_t warp = (blockIdx.x * (int64_t)blockDim.x + threadIdx.x) >> 5;
   const int64_t nwarps = ((int64_t)gridDim.x * blockDim.x) >> 5;
   const int64_t tiles = (p.n + 1023) >> 10;
   const int64_t words = (p.n + 31) >> 5;
-  for (int64_t t = warp; t < tiles; t += nwarps) {
-    const int64_t row0 = t << 10;
-    uint32_t mine = 0;
-    if (p.vec_ok && row0 + 1024 <= p.n) {
-      const uint4* src = (const uint4*)((const uint8_t*)p.col + row0 * W);
-      uint4 v[U];
+  for (int64_t t0 = warp * M; t0 < tiles; t0 += nwarps * M) {
+    if (p.vec_ok && ((t0 + M) << 10) <= p.n) {
+      uint4 v[M][U];
 #pragma unroll
-      for (int u = 0; u < U; ++u) v[u] = __ldcs(src + lane + 32 * u);   // streaming: read once
+      for (int i = 0; i < M; ++i) {
+        const uint4* src = (const uint4*)((const uint8_t*)p.col + ((t0 + i) << 10) * W);
 #pragma unroll
-      for (int u = 0; u < U; ++u) {
-        uint32_t w = chunk_bits<W>(p, v[u]) << ((lane % K) * R);
-#pragma unroll
-        for (int o = 1; o < K; o <<= 1) w |= __shfl_xor_sync(0xffffffffu, w, o);
-        uint32_t val = __shfl_sync(0xffffffffu, w, (lane % R) * K);
-        if (lane / R == u) mine = val;
+        for (int u = 0; u < U; ++u) v[i][u] = __ldcs(src + lane + 32 * u);   // streaming: read once
       }
-    } else {
-      // ragged tail or unaligned column: lane j evaluates the 32 rows of word j
-      for (int bit = 0; bit < 32; ++bit) {
-        int64_t r = row0 + 32 * lane + bit;
-        if (r < p.n && row_pred_scalar(p, r)) mine |= 1u << bit;
-      }
+#pragma unroll
+      for (int i = 0; i < M; ++i) p.out[((t0 + i) << 5) + lane] = tile_word<W>(p, v[i], lane);
+      continue;
     }
-    int64_t wi = (t << 5) + lane;
-    if (wi < words) p.out[wi] = mine;
+    for (int64_t t = t0; t < t0 + M && t < tiles; ++t) {
+      const int64_t row0 = t << 10;
+      uint32_t mine = 0;
+      if (p.vec_ok && row0 + 1024 <= p.n) {
+        const uint4* src = (const uint4*)((const uint8_t*)p.col + row0 * W);
+        uint4 v[U];
+#pragma unroll
+        for (int u = 0; u < U; ++u) v[u] = __ldcs(src + lane + 32 * u);
+        mine = tile_word<W>(p, v, lane);
+      } else {
+        // ragged tail or unaligned column: lane j evaluates the 32 rows of word j
+        for (int bit = 0; bit < 32; ++bit) {
+          int64_t r = row0 + 32 * lane + bit;
+          if (r < p.n && row_pred_scalar(p, r)) mine |= 1u << bit;
+        }
+      }
+      int64_t wi = (t << 5) + lane;
+      if (wi < words) p.out[wi] = mine;
+    }
   }
 }
 
@@ -168,12 +193,14 @@ cudaError_t launch_select_bitmap(const SelParams& p0, int grid, cudaStream_t s) 
     }
   }
   int64_t tiles = (p.n + 1023) >> 10;
-  int64_t g = (tiles + 7) / 8;             // 8 warps per block
+  const int W = dtype_width(p.dtype);
+  const int M = W == 1 ? 4 : 1;            // tiles per warp iteration
+  int64_t g = ((tiles + M - 1) / M + 7) / 8;   // 8 warps per block
   if (g > grid) g = grid;
-  switch (dtype_width(p.dtype)) {
-    case 1: { count_launch(); k_select_bitmap<1><<<(int)g, 256, 0, s>>>(p); break; }
-    case 4: { count_launch(); k_select_bitmap<4><<<(int)g, 256, 0, s>>>(p); break; }
-    default: { count_launch(); k_select_bitmap<8><<<(int)g, 256, 0, s>>>(p); break; }
+  switch (W) {
+    case 1: { count_launch(); k_select_bitmap<1, 4><<<(int)g, 256, 0, s>>>(p); break; }
+    case 4: { count_launch(); k_select_bitmap<4, 1><<<(int)g, 256, 0, s>>>(p); break; }
+    default: { count_launch(); k_select_bitmap<8, 1><<<(int)g, 256, 0, s>>>(p); break; }
   }
   return cudaGetLastError();
 }

@@ -6,6 +6,8 @@
 // the per-work-group aggregation "a single thread is scheduled per group to
 // compute the final aggregate" (L567-568 §4.1.7).  Here one thread per table
 // slot decodes the states (AVG = SUM / COUNT) and writes the dense output row.
+#include <type_traits>
+#include <stdlib.h>
 #include "launch.cuh"
 #include "rowops.cuh"
 
@@ -228,11 +230,11 @@ __device__ __forceinline__ uint64_t* table_claim(uint8_t* table, uint64_t mask, 
   return nullptr;
 }
 
-template <int W0, int W1>
+template <int W0, int W1, int R>
 __global__ void __launch_bounds__(256) k_group_build(const __grid_constant__ Plan p, int32_t* gid_out,
                                                      int64_t max_rows, int64_t* ngroups, int64_t* keys_out,
                                                      int64_t out_capacity) {
-  constexpr int R = 4;                     // rows per thread per iteration (independent gathers in flight)
+  // R rows per thread per iteration: every oid load, then every (dependent) key gather, in flight
   __shared__ unsigned long long ck[kGroupCache];
   __shared__ int32_t cs[kGroupCache];
   for (int i = threadIdx.x; i < kGroupCache; i += blockDim.x) {
@@ -411,13 +413,22 @@ cudaError_t launch_group_build(const Plan& p, int32_t* gid_out, int64_t max_rows
   if (max_rows == 0) return cudaSuccess;
   int64_t g = (max_rows + 1023) / 1024;
   if (g > grid) g = grid;
-  auto fn = k_group_build<0, 0>;
-  const int w0 = p.keys[0].col.width, w1 = p.nkeys > 1 ? p.keys[1].col.width : 0;
-  if (p.nkeys == 2 && w0 == 1 && w1 == 1) fn = k_group_build<1, 1>;
-  else if (p.nkeys == 2 && w0 == 4 && w1 == 4) fn = k_group_build<4, 4>;
-  else if (p.nkeys == 1 && w0 == 1) fn = k_group_build<1, 0>;
-  else if (p.nkeys == 1 && w0 == 4) fn = k_group_build<4, 0>;
-  else if (p.nkeys == 1 && w0 == 8) fn = k_group_build<8, 0>;
+  const char* er = getenv("OCL_GB_R");
+  const int rr = er ? atoi(er) : 4;
+  auto pick = [&](auto r) {
+    constexpr int R = decltype(r)::value;
+    auto fn = k_group_build<0, 0, R>;
+    const int w0 = p.keys[0].col.width, w1 = p.nkeys > 1 ? p.keys[1].col.width : 0;
+    if (p.nkeys == 2 && w0 == 1 && w1 == 1) fn = k_group_build<1, 1, R>;
+    else if (p.nkeys == 2 && w0 == 4 && w1 == 4) fn = k_group_build<4, 4, R>;
+    else if (p.nkeys == 1 && w0 == 1) fn = k_group_build<1, 0, R>;
+    else if (p.nkeys == 1 && w0 == 4) fn = k_group_build<4, 0, R>;
+    else if (p.nkeys == 1 && w0 == 8) fn = k_group_build<8, 0, R>;
+    return fn;
+  };
+  auto fn = rr >= 16 ? pick(std::integral_constant<int, 16>{})
+            : rr >= 8 ? pick(std::integral_constant<int, 8>{})
+            : rr <= 2 ? pick(std::integral_constant<int, 2>{}) : pick(std::integral_constant<int, 4>{});
   count_launch();
   fn<<<(int)g, 256, 0, s>>>(p, gid_out, max_rows, ngroups, keys_out, out_capacity);
   return cudaGetLastError();
