@@ -93,7 +93,11 @@ def workload_columns(wl, cols):
                 aggs, 4 + 1 + 1 + 4 * 8)
     aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
     if wl["kind"] == "sweep":
-        return [(cols["p"], {"hi": wl["threshold"] - 1})], [cols["key"]], [cols["v"]], aggs, 20
+        # the predicate column always, then key and value sectors of 32-byte lines
+        # holding a qualifying row: 4 + 16 (1 - (1 - sel)^4) B/row (20 B at 100 %)
+        sel = wl["threshold"] / 10**6
+        return [(cols["p"], {"hi": wl["threshold"] - 1})], [cols["key"]], [cols["v"]], aggs, \
+            4 + 16 * (1 - (1 - sel) ** 4)
     return [], [cols["orderkey"]], [cols["quantity"]], aggs, 16
 
 

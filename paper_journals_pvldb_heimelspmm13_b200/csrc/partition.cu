@@ -1139,6 +1139,10 @@ __device__ __forceinline__ void part_emit_row(const Plan& p, const PartArgs& a, 
 #define OCL_AGG_BLOCKS 3
 #endif
 constexpr int kAggBlocks = OCL_AGG_BLOCKS;     // CTAs per SM of pass 2 (shared table 64 KB each)
+#ifndef OCL_AGG_ILP
+#define OCL_AGG_ILP 4
+#endif
+constexpr int kAggILP = OCL_AGG_ILP;           // records per thread in flight in pass 2
 
 template <int NV, bool FIX>
 __global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __grid_constant__ Plan p, PartArgs a,
@@ -1170,12 +1174,12 @@ __global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __g
     for (int i = threadIdx.x; i < kPartCap * cs / 16; i += blockDim.x) ((uint4*)tab)[i] = make_uint4(0, 0, 0, 0);
     if (threadIdx.x == 0) overflowed = 0;
     __syncthreads();
-    for (int64_t base = s; base < seg_end; base += kPartILP * blockDim.x) {
-      uint64_t key[kPartILP];
-      int32_t v[kPartILP][NV > 0 ? NV : 1];
-      bool valid[kPartILP];
+    for (int64_t base = s; base < seg_end; base += kAggILP * blockDim.x) {
+      uint64_t key[kAggILP];
+      int32_t v[kAggILP][NV > 0 ? NV : 1];
+      bool valid[kAggILP];
 #pragma unroll
-      for (int k = 0; k < kPartILP; ++k) {   // loads of kPartILP records first
+      for (int k = 0; k < kAggILP; ++k) {   // loads of kAggILP records first
         const int64_t j = base + k * blockDim.x + threadIdx.x;
         valid[k] = j < seg_end;
         key[k] = 0;
@@ -1184,7 +1188,7 @@ __global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __g
         if (valid[k]) load_rec<NV>(a.recs + (size_t)j * a.rec_bytes, key[k], v[k]);
       }
 #pragma unroll
-      for (int k = 0; k < kPartILP; ++k) {
+      for (int k = 0; k < kAggILP; ++k) {
         const uint64_t k0 = __shfl_sync(0xffffffffu, key[k], 0);
         if (__all_sync(0xffffffffu, valid[k] && key[k] == k0)) {    // heavy hitter: one update per warp
           const int ts = __shfl_sync(0xffffffffu, lane == 0 ? part_find(tab, k0, direct, a.pbits) : -1, 0);
