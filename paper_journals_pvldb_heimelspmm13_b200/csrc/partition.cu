@@ -646,7 +646,8 @@ __global__ void k_part_zero_regions(const __grid_constant__ Plan p, PartArgs a) 
 // 2^b1 partially written lines open in L2.  Per tile: ranks by shared atomics on the
 // 2^b1 counters, one scan, records staged in partition order and written as runs.
 template <class Sh, int NV>
-__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a) {
+__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a,
+                                                                     uint8_t* out) {
   extern __shared__ __align__(16) uint8_t dsm[];
   TileMap& m = *(TileMap*)dsm;            // cnt / off / key (= block cursor) used for 2^b1 slots
   __shared__ uint32_t wsum[32];
@@ -714,10 +715,10 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __gri
 #pragma unroll
       for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
       if constexpr (NV <= 2) tile_stage(m, q[k], rank[k], pack_rec16<NV>((uint64_t)x[k].key, v));
-      else store_rec<NV>(a.tmp + (size_t)(m.cnt[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
+      else store_rec<NV>(out + (size_t)(m.cnt[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
     }
     __syncthreads();
-    if constexpr (NV <= 2) tile_flush(m, m.total, a.tmp, a.rec_bytes);
+    if constexpr (NV <= 2) tile_flush(m, m.total, out, a.rec_bytes);
     __syncthreads();
     for (int i = t; i < P1; i += blockDim.x) m.cnt[i] = 0;
     // (the next tile's atomics on m.cnt come after the next barrier-free stretch: order them)
@@ -1414,7 +1415,7 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
     if ((e = cudaMemsetAsync(a.out_ctr, 0, 8, s))) return e;
   }
   a.b1 = std::min(a.pbits, kPartLevelBits);
-  if (part_scatter_mode() != 5 || a.pbits <= kPartLevelBits) a.cnt1 = nullptr;
+  if (part_scatter_mode() != 5) a.cnt1 = nullptr;
   count_launch(5);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
   k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
@@ -1434,12 +1435,17 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   const int smode = part_scatter_mode();
   if (a.cnt1) {                           // two levels, level 1 into per-block ranges
     const int64_t n1 = ((int64_t)1 << b1) * a.nblk, nc1 = (n1 + kScanChunk - 1) / kScanChunk;
-    count_launch(5);
+    count_launch(4);
     k_scan_chunks<<<(int)nc1, kScanThreads, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
     k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums1, nc1, a.nitems_dev);     // (total unused; rewritten below)
     k_scan_add<<<(int)((n1 + 255) / 256), 256, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
-    kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a);
-    ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
+    if (b2 == 0) {                        // one level: the per-block ranges are the final partitions
+      kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.recs);
+    } else {
+      count_launch();
+      kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.tmp);
+      ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
+    }
   } else if (smode != 1 && smode != 5) {
     count_launch(2);
     k_part_cur_pad<<<(int)((L + 255) / 256), 256, 0, s>>>(a.offs, a.curp, a.curp_shift, L);
