@@ -1060,11 +1060,11 @@ __device__ __forceinline__ void part_flush_slot_excl(const Plan& p, const uint8_
   }
 }
 
-// Shared-table find-or-insert for pass 2 -> slot, or -1 (probe limit).  In direct mode the
-// start slot and the linear probing (wrapping inside the table) mirror the key's slot range
-// in the HBM table — the table's start slot is the top log2(cap) hash bits and a partition's
-// range has exactly kPartCap slots — so the entries can be stored to the HBM table position
-// by position, without probing it.
+// Shared-table find-or-insert for pass 2 -> slot, or -1 (probe limit).  Triangular
+// (quadratic) probing from the home slot: linear probing's clusters made the warp-wide
+// longest probe sequence the cost of every lookup at load 1/2 (ncu on C5 with 2^16 groups:
+// ~half of pass 2's instructions in the probe loop).  The shared table's layout is private to
+// the CTA (entries reach HBM through table_find_or_insert or as output rows).
 constexpr int kPartProbes = 64;
 
 __device__ __forceinline__ int part_find(uint8_t* tab, uint64_t key, bool direct, int pbits) {
@@ -1079,16 +1079,16 @@ __device__ __forceinline__ int part_find(uint8_t* tab, uint64_t key, bool direct
       const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
       if (prev == 0 || prev == sk) return (int)i;
     }
-    i = (i + 1) & (kPartCap - 1);
+    i = (i + probe + 1) & (kPartCap - 1);   // triangular (quadratic) probing
   }
   return -1;
 }
 
-// Claim path of part_find_warp, out of line: linear probing with CAS from slot i (the first
-// empty slot this lane saw), up to kPartProbes more slots.
-static __device__ __noinline__ int part_claim_slow(uint8_t* tab, uint64_t key, uint32_t i) {
+// Claim path of part_find_warp, out of line: the same probe sequence with CAS from slot i
+// (the first empty slot this lane saw, reached after `np` steps).
+static __device__ __noinline__ int part_claim_slow(uint8_t* tab, uint64_t key, uint32_t i, int np) {
   const uint64_t sk = ~key;
-  for (int probe = 0; probe < kPartProbes; ++probe) {
+  for (int probe = np; probe < kPartProbes; ++probe) {
     uint64_t* kp = pkey(tab, (int)i);
     const uint64_t cur = *(volatile uint64_t*)kp;
     if (cur == sk) return (int)i;
@@ -1096,7 +1096,7 @@ static __device__ __noinline__ int part_claim_slow(uint8_t* tab, uint64_t key, u
       const uint64_t prev = atomicCAS((unsigned long long*)kp, 0ULL, (unsigned long long)sk);
       if (prev == 0 || prev == sk) return (int)i;
     }
-    i = (i + 1) & (kPartCap - 1);
+    i = (i + probe + 1) & (kPartCap - 1);
   }
   return -1;
 }
@@ -1116,10 +1116,11 @@ __device__ __forceinline__ int part_find_warp(uint8_t* tab, uint64_t key, bool a
   if (__any_sync(0xffffffffu, act && ts < 0)) {
     bool pend = act && ts < 0 && c != 0;
     bool claim = act && ts < 0 && c == 0;
-    int np = 0;
+    int np = 0;                           // probe steps taken (slot i = home + np (np + 1) / 2)
     while (__any_sync(0xffffffffu, pend)) {
       if (pend) {
-        i = (i + 1) & (kPartCap - 1);
+        i = (i + np + 1) & (kPartCap - 1);
+        ++np;
         c = *(volatile uint64_t*)pkey(tab, (int)i);
         if (c == sk) {
           ts = (int)i;
@@ -1127,18 +1128,18 @@ __device__ __forceinline__ int part_find_warp(uint8_t* tab, uint64_t key, bool a
         } else if (c == 0) {
           claim = true;
           pend = false;
-        } else if (++np >= kPartProbes) {
+        } else if (np >= kPartProbes) {
           pend = false;                   // probe limit: overflow
         }
       }
     }
     if (__any_sync(0xffffffffu, claim))
-      if (claim) ts = part_claim_slow(tab, key, i);
+      if (claim) ts = part_claim_slow(tab, key, i, np);
   }
   return ts;
 }
 
-// Direct merge: shared slot -> HBM slot region + slot (the region holds no entries yet).
+// A shared slot as a table-format entry at e (partial output rows).
 __device__ __forceinline__ void part_store_slot(const Plan& p, const uint8_t* tab, int slot, uint8_t* e) {
   const uint64_t sk = *pkey((uint8_t*)tab, slot);
   const uint32_t cnt = *pf32(tab, slot, 8);
@@ -1225,7 +1226,8 @@ __global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __g
     const int64_t s = q0 + (item - (int64_t)a.ioff[lo]) * kPartItem;
     const int64_t seg_end = min(q1, s + kPartItem);
     const bool exclusive = q1 - q0 <= kPartItem;
-    const bool direct = a.direct_ok && exclusive && a.slowflag[lo] == 0;
+    // direct: rows emitted straight from shared memory (one-item partition, no exact-path rows)
+    const bool direct = a.direct_ok && a.direct_emit && exclusive && a.slowflag[lo] == 0;
     for (int i = threadIdx.x; i < kPartCap * cs / 16; i += blockDim.x) ((uint4*)tab)[i] = make_uint4(0, 0, 0, 0);
     if (threadIdx.x == 0) overflowed = 0;
     __syncthreads();
@@ -1300,9 +1302,6 @@ __global__ void __launch_bounds__(kPartThreads, kAggBlocks) k_part_agg(const __g
       __syncthreads();
       for (uint32_t i = threadIdx.x; i < tot; i += kPartThreads)
         part_emit_row(p, a, ea, tab, slot_list[i], (int64_t)base_s + i);
-    } else if (direct && !overflowed) {
-      uint8_t* region = p.table + ((size_t)lo << kPartCapBits) * p.stride;
-      for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) part_store_slot(p, tab, i, region + (size_t)i * p.stride);
     } else if (exclusive) {
       for (int i = threadIdx.x; i < kPartCap; i += blockDim.x) part_flush_slot_excl(p, tab, i);
     } else {
