@@ -650,6 +650,7 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __gri
                                                                      uint8_t* out) {
   extern __shared__ __align__(16) uint8_t dsm[];
   TileMap& m = *(TileMap*)dsm;            // cnt / off / key (= block cursor) used for 2^b1 slots
+  uint32_t* gb = (uint32_t*)m.used;       // this tile's global base per slot (the used list is idle here)
   __shared__ uint32_t wsum[32];
   const int P1 = 1 << a.b1;
   const int64_t r0 = blockIdx.x * a.rows_per_blk;
@@ -703,7 +704,9 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __gri
         m.off[t] = off + incl - c;
         const uint32_t g = m.key[t];
         m.key[t] = g + c;                    // block cursor
-        m.cnt[t] = g;                        // this tile's global base
+        gb[t] = g;                           // this tile's global base
+        m.cnt[t] = 0;                        // ranks taken: ready for the next tile (its atomics
+                                             // follow two more barriers)
         if (t == P1 - 1) m.total = off + incl;
       }
     }
@@ -715,14 +718,15 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __gri
 #pragma unroll
       for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
       if constexpr (NV <= 2) tile_stage(m, q[k], rank[k], pack_rec16<NV>((uint64_t)x[k].key, v));
-      else store_rec<NV>(out + (size_t)(m.cnt[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
+      else store_rec<NV>(out + (size_t)(gb[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
     }
     __syncthreads();
-    if constexpr (NV <= 2) tile_flush(m, m.total, out, a.rec_bytes);
-    __syncthreads();
-    for (int i = t; i < P1; i += blockDim.x) m.cnt[i] = 0;
-    // (the next tile's atomics on m.cnt come after the next barrier-free stretch: order them)
-    __syncthreads();
+    if constexpr (NV <= 2)
+      for (uint32_t i = t; i < m.total; i += blockDim.x) {
+        const uint32_t sl = m.sslot[i];
+        *(uint4*)(out + (size_t)(gb[sl] + (i - m.off[sl])) * 16) = m.stage[i];
+      }
+    __syncthreads();                      // stage / gb / off are rewritten by the next tile
   }
 }
 
