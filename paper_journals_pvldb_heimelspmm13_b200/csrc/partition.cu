@@ -317,10 +317,11 @@ __device__ __forceinline__ void tile_map_claim(TileMap& m, uint32_t* cur, uint32
 }
 
 // Direct-indexed variant (slot i = partition qb + i, i < width): the same claim over every
-// slot of the range instead of the used list.
+// slot of the range instead of the used list; bases go to gb[] and the counters are left
+// zeroed (no reset pass after the flush).
 constexpr uint32_t kDirectMap = 1024;
 __device__ __forceinline__ void tile_dmap_claim(TileMap& m, uint32_t width, uint32_t qb, uint32_t* cur,
-                                                uint32_t* wsum) {
+                                                uint32_t* wsum, uint32_t* gb) {
   const int t = threadIdx.x, lane = t & 31, w = t >> 5;
   uint32_t run0 = 0;
   for (uint32_t b0 = 0; b0 < width; b0 += kPartThreads) {
@@ -342,7 +343,8 @@ __device__ __forceinline__ void tile_dmap_claim(TileMap& m, uint32_t width, uint
     }
     if (i < width) {
       m.off[i] = run0 + off + incl - c;
-      m.cnt[i] = c ? atomicAdd(&cur[qb + i], c) : 0u;
+      gb[i] = c ? atomicAdd(&cur[qb + i], c) : 0u;   // global base of the slot's range
+      m.cnt[i] = 0;                                 // ranks taken: clean for the next tile
     }
     run0 += tot;
     __syncthreads();
@@ -738,6 +740,8 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
   extern __shared__ __align__(16) uint8_t dsm[];
   TileMap& map = *(TileMap*)dsm;
   __shared__ uint32_t wsum[32];
+  uint32_t* gb = map.off + kTileMap / 2;  // direct-map tiles: global bases (slots < kDirectMap)
+  static_assert(kDirectMap <= kTileMap / 2, "direct-map bases share the off array");
   const int64_t m = *a.m_dev;
   constexpr int TILE = kPartILP * kPartThreads;
   const int64_t per = ((m + gridDim.x - 1) / gridDim.x + TILE - 1) / TILE * TILE;
@@ -754,8 +758,12 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
   if (j0 < j1) fetch(j0);
   tile_map_init(map);
   __syncthreads();
+  bool hashed = false;                    // the previous tile used the hashed map (CTA-uniform)
   for (int64_t base = j0; base < j1; base += TILE) {
-    tile_map_reset(map);
+    if (hashed || NV > 2) {
+      tile_map_reset(map);
+      __syncthreads();
+    }
     uint64_t key[kPartILP];
     int32_t v[kPartILP][NV > 0 ? NV : 1];
     bool ok[kPartILP];
@@ -774,8 +782,8 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
     const uint32_t q1f = part_of(*(const uint64_t*)(a.tmp + (size_t)base * a.rec_bytes), a.b1);
     const uint32_t q1l = part_of(*(const uint64_t*)(a.tmp + (size_t)(min(base + TILE, j1) - 1) * a.rec_bytes), a.b1);
     const uint32_t qb = q1f << sh, width = (q1l - q1f + 1) << sh;
-    const bool dmap = a.b1 > 0 && width <= kDirectMap;       // CTA-uniform
-    __syncthreads();
+    const bool dmap = a.b1 > 0 && width <= kDirectMap && NV <= 2;   // CTA-uniform
+    hashed = !dmap;
     if (dmap) {                           // direct-indexed map: no hashing, no key slots
 #pragma unroll
       for (int k = 0; k < kPartILP; ++k)
@@ -784,14 +792,24 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
           rank[k] = atomicAdd(&map.cnt[slot[k]], 1u);
         }
       __syncthreads();
-      tile_dmap_claim(map, width, qb, a.cur, wsum);
-    } else {
+      tile_dmap_claim(map, width, qb, a.cur, wsum, gb);
+      __syncthreads();
 #pragma unroll
       for (int k = 0; k < kPartILP; ++k)
-        if (ok[k]) tile_map_add(map, part_of(key[k], a.pbits), slot[k], rank[k]);
+        if (ok[k]) tile_stage(map, slot[k], rank[k], pack_rec16<NV>(key[k], v[k]));
       __syncthreads();
-      tile_map_claim(map, a.cur, wsum);
+      for (uint32_t i = threadIdx.x; i < map.total; i += blockDim.x) {
+        const uint32_t sl = map.sslot[i];
+        *(uint4*)(a.recs + (size_t)(gb[sl] + (i - map.off[sl])) * 16) = map.stage[i];
+      }
+      __syncthreads();                    // stage / off / gb are rewritten by the next tile
+      continue;
     }
+#pragma unroll
+    for (int k = 0; k < kPartILP; ++k)
+      if (ok[k]) tile_map_add(map, part_of(key[k], a.pbits), slot[k], rank[k]);
+    __syncthreads();
+    tile_map_claim(map, a.cur, wsum);
     __syncthreads();
 #pragma unroll
     for (int k = 0; k < kPartILP; ++k) {
@@ -804,8 +822,6 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter2(PartArgs a) {
       tile_flush(map, map.total, a.recs, a.rec_bytes);
       __syncthreads();
     }
-    if (dmap)                             // (ordered before the next tile's adds by the reset barrier)
-      for (uint32_t i = threadIdx.x; i < width; i += blockDim.x) map.cnt[i] = 0;
   }
 }
 
