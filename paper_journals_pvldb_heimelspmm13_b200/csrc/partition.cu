@@ -1087,10 +1087,18 @@ __device__ __forceinline__ void part_flush_slot_excl(const Plan& p, const uint8_
 // the CTA (entries reach HBM through table_find_or_insert or as output rows).
 constexpr int kPartProbes = 64;
 
+// Home slot in the pass-2 shared table: multiplicative (Fibonacci) hashing — the partition
+// already fixed the key's top fmix64 bits, and the shared layout is private to the CTA, so
+// one 64-bit multiply replaces a second fmix64 per record.
+__device__ __forceinline__ uint32_t part_home(uint64_t key) {
+  return (uint32_t)((key * 0x9E3779B97F4A7C15ULL) >> (64 - kPartCapBits));
+}
+
 __device__ __forceinline__ int part_find(uint8_t* tab, uint64_t key, bool direct, int pbits) {
   const uint64_t sk = ~key;
-  const uint64_t h = fmix64(key);
-  uint32_t i = direct ? (uint32_t)((h << pbits) >> (64 - kPartCapBits)) : (uint32_t)h & (kPartCap - 1);
+  (void)direct;
+  (void)pbits;
+  uint32_t i = part_home(key);
   for (int probe = 0; probe < kPartProbes; ++probe) {
     uint64_t* kp = pkey(tab, (int)i);
     const uint64_t cur = *(volatile uint64_t*)kp;
@@ -1129,8 +1137,9 @@ static __device__ __noinline__ int part_claim_slow(uint8_t* tab, uint64_t key, u
 // sequence and its CAS branch structure.  Same slots, same probe limit as part_find.
 __device__ __forceinline__ int part_find_warp(uint8_t* tab, uint64_t key, bool act, bool direct, int pbits) {
   const uint64_t sk = ~key;
-  const uint64_t hsh = fmix64(key);
-  uint32_t i = direct ? (uint32_t)((hsh << pbits) >> (64 - kPartCapBits)) : (uint32_t)hsh & (kPartCap - 1);
+  (void)direct;
+  (void)pbits;
+  uint32_t i = part_home(key);
   uint64_t c = *(volatile uint64_t*)pkey(tab, (int)i);
   int ts = act && c == sk ? (int)i : -1;
   if (__any_sync(0xffffffffu, act && ts < 0)) {
