@@ -647,12 +647,25 @@ __global__ void k_part_zero_regions(const __grid_constant__ Plan p, PartArgs a) 
 // advances its own cursors in shared memory: no global claims, and a block keeps only
 // 2^b1 partially written lines open in L2.  Per tile: ranks by shared atomics on the
 // 2^b1 counters, one scan, records staged in partition order and written as runs.
-template <class Sh, int NV>
-__global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a,
-                                                                     uint8_t* out) {
+// The level-1 tile state of a T-thread block (~21 KB at T = 256: four blocks of 8 warps per
+// SM, so one block's barriers overlap the others' loads; at T = 512 two blocks fit).
+template <int T>
+struct L1Map {
+  uint4 stage[kPartILP * T];              // the tile's records, grouped by partition
+  uint32_t cnt[256];                      // ranks, then zero again
+  uint32_t off[256];                      // the slot's first index in the staging area
+  uint32_t key[256];                      // block cursor
+  uint32_t gb[256];                       // this tile's global base per slot
+  uint8_t sslot[kPartILP * T];            // slot of each staged record
+  uint32_t total;
+};
+
+template <class Sh, int NV, int T>
+__global__ void __launch_bounds__(T, T == 256 ? 4 : 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a,
+                                                                         uint8_t* out) {
   extern __shared__ __align__(16) uint8_t dsm[];
-  TileMap& m = *(TileMap*)dsm;            // cnt / off / key (= block cursor) used for 2^b1 slots
-  uint32_t* gb = (uint32_t*)m.used;       // this tile's global base per slot (the used list is idle here)
+  L1Map<T>& m = *(L1Map<T>*)dsm;
+  uint32_t* gb = m.gb;
   __shared__ uint32_t wsum[32];
   const int P1 = 1 << a.b1;
   const int64_t r0 = blockIdx.x * a.rows_per_blk;
@@ -719,7 +732,11 @@ __global__ void __launch_bounds__(kPartThreads, 2) k_part_scatter_l1(const __gri
       int32_t v[NV > 0 ? NV : 1];
 #pragma unroll
       for (int i = 0; i < NV; ++i) v[i] = (int32_t)x[k].vi[i];
-      if constexpr (NV <= 2) tile_stage(m, q[k], rank[k], pack_rec16<NV>((uint64_t)x[k].key, v));
+      if constexpr (NV <= 2) {
+        const uint32_t i = m.off[q[k]] + rank[k];
+        m.stage[i] = pack_rec16<NV>((uint64_t)x[k].key, v);
+        m.sslot[i] = (uint8_t)q[k];
+      }
       else store_rec<NV>(out + (size_t)(gb[q[k]] + rank[k]) * a.rec_bytes, (uint64_t)x[k].key, v);
     }
     __syncthreads();
@@ -1456,10 +1473,13 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   const int b1 = a.b1, b2 = a.pbits - b1;
   const size_t msm = sizeof(TileMap);
   auto ks2 = k_part_scatter2<NV>;
-  auto kl1 = k_part_scatter_l1<Sh, NV>;
+  const bool l1_512 = getenv("OCL_L1T") && atoi(getenv("OCL_L1T")) == 512;   // A/B: 512-thread level-1 blocks
+  auto kl1 = l1_512 ? k_part_scatter_l1<Sh, NV, 512> : k_part_scatter_l1<Sh, NV, 256>;
+  const int l1t = l1_512 ? 512 : 256;
+  const size_t l1sm = l1_512 ? sizeof(L1Map<512>) : sizeof(L1Map<256>);
   if ((e = cudaFuncSetAttribute(ks, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
   if ((e = cudaFuncSetAttribute(ks2, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
-  if ((e = cudaFuncSetAttribute(kl1, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
+  if ((e = cudaFuncSetAttribute(kl1, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)l1sm))) return e;
   const int smode = part_scatter_mode();
   if (a.cnt1) {                           // two levels, level 1 into per-block ranges
     const int64_t n1 = ((int64_t)1 << b1) * a.nblk, nc1 = (n1 + kScanChunk - 1) / kScanChunk;
@@ -1468,10 +1488,10 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
     k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums1, nc1, a.nitems_dev);     // (total unused; rewritten below)
     k_scan_add<<<(int)((n1 + 255) / 256), 256, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
     if (b2 == 0) {                        // one level: the per-block ranges are the final partitions
-      kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.recs);
+      kl1<<<a.nblk, l1t, l1sm, s>>>(p, a, a.recs);
     } else {
       count_launch();
-      kl1<<<a.nblk, kPartThreads, msm, s>>>(p, a, a.tmp);
+      kl1<<<a.nblk, l1t, l1sm, s>>>(p, a, a.tmp);
       ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
     }
   } else if (smode != 1 && smode != 5) {
