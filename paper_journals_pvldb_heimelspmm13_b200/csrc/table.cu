@@ -234,7 +234,9 @@ template <int W0, int W1, int R>
 __global__ void __launch_bounds__(256) k_group_build(const __grid_constant__ Plan p, int32_t* gid_out,
                                                      int64_t max_rows, int64_t* ngroups, int64_t* keys_out,
                                                      int64_t out_capacity) {
-  // R rows per thread per iteration: every oid load, then every (dependent) key gather, in flight
+  // R rows per thread per iteration: every oid load, then every (dependent) key gather, in flight.
+  // Measured on the 2 x u8 Q1 keys at 600M rows (2.05 ms at R = 4, 48 registers): R = 2 / 8 / 16
+  // 2.67 / 2.51 / 4.16 ms; 6 or 8 blocks per SM (40 / 32 registers) 2.11 / 2.21 ms
   __shared__ unsigned long long ck[kGroupCache];
   __shared__ int32_t cs[kGroupCache];
   for (int i = threadIdx.x; i < kGroupCache; i += blockDim.x) {
