@@ -72,6 +72,13 @@ struct PartArgs {
                         // exclusive scan: each block's own range in every level-1 partition
   uint32_t* sums1;      // scan chunk sums of cnt1
   int32_t b1;           // level-1 bits (two-level scatter)
+  // low selectivity (sparse_dev != NULL and *sparse_dev = 1, decided on the device from a
+  // sample): the count pass streams the predicate columns only, evaluates the other columns
+  // of qualifying rows and lists their row ids in its block's range of soids (nq[block] of
+  // them); the level-1 scatter reads those lists instead of the columns
+  int32_t* sparse_dev;
+  uint32_t* soids;      // [n] row ids, block b's list at [b * rows_per_blk, + nq[b])
+  uint32_t* nq;         // [nblk]
   uint32_t* icnt;       // [P] pass-2 work items per partition
   uint32_t* ioff;       // [P] exclusive scan of icnt
   uint32_t* isums;      // scan chunk sums of icnt
@@ -179,9 +186,37 @@ __device__ __forceinline__ void part_rows(const Plan& p, int64_t wbase, int64_t 
   for (int i = 0; i < 4; ++i) part_eval<Sh, NV>(p, part_row(wbase, lane, i), r1, x[i], ok[i]);
 }
 
+// Predicates only (row r < n): the first step of the sparse mode.
+template <class Sh>
+__device__ __forceinline__ bool row_qualifies(const Plan& p, int64_t r) {
+  bool q = true;
+#pragma unroll
+  for (int i = 0; i < kMaxPreds; ++i) {
+    if (i >= Sh::np(p)) break;
+    q = q && pred_ok<Sh>(p, i, ld1w(Sh::pw(p, i), p.preds[i].col.ptr, r));
+  }
+  return q;
+}
+
+// Sparse-mode decision: the predicates on 1024 rows spread over the input (one CTA).
+constexpr int kPartSparsePct = 8;     // below this many percent qualifying: sparse mode
+template <class Sh>
+__global__ void __launch_bounds__(1024) k_part_sample(const __grid_constant__ Plan p, int32_t* sparse_dev) {
+  __shared__ int cnt;
+  if (threadIdx.x == 0) cnt = 0;
+  __syncthreads();
+  const int64_t span = p.n / 1024;
+  if (span > 0 && row_qualifies<Sh>(p, (int64_t)threadIdx.x * span)) atomicAdd(&cnt, 1);
+  __syncthreads();
+  if (threadIdx.x == 0) *sparse_dev = (span > 0 && 100 * cnt < kPartSparsePct * 1024) ? 1 : 0;
+}
+
 // ------------------------------------------------------------------ pass 1a: histogram
-template <class Sh, int NV>
+template <class Sh, int NV, bool SPARSE>
 __global__ void __launch_bounds__(kPartThreads) k_part_count(const __grid_constant__ Plan p, PartArgs a) {
+  // SPARSE: the low-selectivity variant, launched next to the dense one; each returns at
+  // once unless the device-side sample chose its mode (grid-uniform)
+  if (a.sparse_dev && (*a.sparse_dev != 0) != SPARSE) return;
   extern __shared__ uint32_t hist[];
   const int P = 1 << a.pbits;
   const int lane = threadIdx.x & 31;
@@ -190,7 +225,51 @@ __global__ void __launch_bounds__(kPartThreads) k_part_count(const __grid_consta
   const int64_t r0 = blockIdx.x * a.rows_per_blk;
   const int64_t r1 = min(p.n, r0 + a.rows_per_blk);
   const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
-  for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
+  constexpr bool sparse = SPARSE;
+  if constexpr (SPARSE) {
+    // 256 rows per warp step, lane l row base + l + 32 i: coalesced predicate loads, then
+    // qualifying rows listed (warp-aggregated claim in the block's list) and evaluated
+    __shared__ uint32_t blk_n;
+    if (threadIdx.x == 0) blk_n = 0;
+    __syncthreads();
+    const uint32_t lt = lanemask_lt();
+    const int64_t nwarp = blockDim.x >> 5;
+    for (int64_t base = r0 + (int64_t)(threadIdx.x >> 5) * 256; base < r1; base += nwarp * 256) {
+      bool q[8];
+      unsigned bal[8];
+      uint32_t tot = 0;
+#pragma unroll
+      for (int i = 0; i < 8; ++i) {
+        const int64_t r = base + 32 * i + lane;
+        q[i] = r < r1 && row_qualifies<Sh>(p, r);
+      }
+#pragma unroll
+      for (int i = 0; i < 8; ++i) {
+        bal[i] = __ballot_sync(0xffffffffu, q[i]);
+        tot += __popc(bal[i]);
+      }
+      if (tot == 0) continue;
+      uint32_t wb = 0;
+      if (lane == 0) wb = atomicAdd(&blk_n, tot);
+      wb = __shfl_sync(0xffffffffu, wb, 0);
+#pragma unroll
+      for (int i = 0; i < 8; ++i) {
+        const int64_t r = base + 32 * i + lane;
+        if (q[i]) {
+          a.soids[r0 + wb + __popc(bal[i] & lt)] = (uint32_t)r;
+          Row<Sh, NV, false> x;
+          eval_one<Sh, NV, false>(p, r, x);
+          const bool ok = x.q && x.fast && !Sh::special(x.key);
+          if (ok) atomicAdd(&hist[part_of((uint64_t)x.key, a.pbits)], 1u);
+          else if (x.q && (uint64_t)x.key != ~0ULL) a.slowflag[part_of((uint64_t)x.key, a.pbits)] = 1u;
+        }
+        wb += __popc(bal[i]);
+      }
+    }
+    __syncthreads();
+    if (threadIdx.x == 0) a.nq[blockIdx.x] = blk_n;
+  }
+  for (int64_t base = r0; base < (sparse ? r0 : r1); base += kPartILP * blockDim.x) {
     Row<Sh, NV, false> x[kPartILP];
     bool ok[kPartILP];
     part_rows<Sh, NV>(p, base + woff, r1, lane, x, ok);
@@ -660,9 +739,10 @@ struct L1Map {
   uint32_t total;
 };
 
-template <class Sh, int NV, int T>
+template <class Sh, int NV, int T, bool SPARSE>
 __global__ void __launch_bounds__(T, T == 256 ? 4 : 2) k_part_scatter_l1(const __grid_constant__ Plan p, PartArgs a,
                                                                          uint8_t* out) {
+  if (a.sparse_dev && (*a.sparse_dev != 0) != SPARSE) return;     // the other variant runs (grid-uniform)
   extern __shared__ __align__(16) uint8_t dsm[];
   L1Map<T>& m = *(L1Map<T>*)dsm;
   uint32_t* gb = m.gb;
@@ -678,24 +758,42 @@ __global__ void __launch_bounds__(T, T == 256 ? 4 : 2) k_part_scatter_l1(const _
   Row<Sh, NV, false> nx[kPartILP];
   bool nok[kPartILP];
   const int64_t woff = (int64_t)(threadIdx.x >> 5) * 128;
-  if (r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
+  // sparse mode: the block's list of qualifying rows (count pass) is the row source
+  constexpr bool sparse = SPARSE;
+  const int64_t s1 = sparse ? r0 + (int64_t)a.nq[blockIdx.x] : r1;
+  if (!sparse && r0 < r1) part_rows<Sh, NV>(p, r0 + woff, r1, lane, nx, nok);
   __syncthreads();
-  for (int64_t base = r0; base < r1; base += kPartILP * blockDim.x) {
+  for (int64_t base = r0; base < s1; base += kPartILP * blockDim.x) {
     Row<Sh, NV, false> x[kPartILP];
     bool ok[kPartILP];
+    int64_t rid[kPartILP];
     uint32_t q[kPartILP], rank[kPartILP];
     const int64_t wbase = base + woff;
+    if constexpr (SPARSE) {
 #pragma unroll
-    for (int k = 0; k < kPartILP; ++k) {
-      x[k] = nx[k];
-      ok[k] = nok[k];
+      for (int k = 0; k < kPartILP; ++k) {
+        const int64_t j = base + (int64_t)k * blockDim.x + threadIdx.x;
+        rid[k] = j < s1 ? (int64_t)a.soids[j] : p.n;
+      }
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k) {
+        eval_one<Sh, NV, false>(p, rid[k], x[k]);       // (row n: x.q = false)
+        ok[k] = x[k].q && x[k].fast && !Sh::special(x[k].key);
+      }
+    } else {
+#pragma unroll
+      for (int k = 0; k < kPartILP; ++k) {
+        x[k] = nx[k];
+        ok[k] = nok[k];
+        rid[k] = part_row(wbase, lane, k);
+      }
+      if (base + kPartILP * blockDim.x < r1) part_rows<Sh, NV>(p, wbase + kPartILP * blockDim.x, r1, lane, nx, nok);
     }
-    if (base + kPartILP * blockDim.x < r1) part_rows<Sh, NV>(p, wbase + kPartILP * blockDim.x, r1, lane, nx, nok);
 #pragma unroll
     for (int k = 0; k < kPartILP; ++k) {
       if (x[k].q && !ok[k]) {               // exact per-row path straight into the HBM table
         uint8_t* e = table_find_or_insert(p.table, p.mask, p.stride, (uint64_t)x[k].key, p.status);
-        if (e) update_entry_slow(p, e, part_row(wbase, lane, k));
+        if (e) update_entry_slow(p, e, rid[k]);
         if ((uint64_t)x[k].key != ~0ULL) a.slowflag[part_of((uint64_t)x[k].key, a.pbits)] = 1u;
       }
       q[k] = ok[k] ? part_of((uint64_t)x[k].key, a.b1) : 0u;
@@ -1433,8 +1531,9 @@ size_t part_ws_bytes(const Plan& p, int pbits, int sms) {
   const int64_t nchunks = (L + kScanChunk - 1) / kScanChunk;
   const bool two = pbits > kPartLevelBits;
   const size_t n1 = ((size_t)1 << kPartLevelBits) * (size_t)sms * 4;   // level-1 counts per row block (nblk <= 4 sms)
+  const size_t sparse = p.npreds > 0 ? align_up((size_t)p.n * 4, 256) + align_up((size_t)sms * 16, 256) + 256 : 0;
   return align_up((size_t)L * 4, 256) * 7 + align_up((size_t)L * 128, 256) + align_up((size_t)nchunks * 4, 256) * 2 + 768 +
-         align_up(n1 * 4, 256) + align_up((n1 / kScanChunk + 1) * 4, 256) +
+         align_up(n1 * 4, 256) + align_up((n1 / kScanChunk + 1) * 4, 256) + sparse +
          align_up((size_t)p.n * part_rec_bytes(p.nvals), 256) * (two ? 2 : 1) + (two ? align_up(4u << kPartLevelBits, 256) : 0);
 }
 
@@ -1442,13 +1541,15 @@ template <class Sh, int NV>
 static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, const EmitArgs& ea,
                             int64_t out_capacity) {
   const size_t hsm = (size_t)4 << a.pbits;
-  auto kc = k_part_count<Sh, NV>;
+  auto kc = k_part_count<Sh, NV, false>;
+  auto kcs = k_part_count<Sh, NV, true>;
   auto ks = k_part_scatter<Sh, NV>;
   const bool fix = NV == 1 && p.nvals == 1 && p.vals[0].co_lo == 12 && p.vals[0].co_hi == 16 &&
                    p.vals[0].co_min == 20 && p.vals[0].co_max == 24;
   auto ka = fix ? k_part_agg<NV, NV == 1> : k_part_agg<NV, false>;
   cudaError_t e;
   if ((e = cudaFuncSetAttribute(kc, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)hsm))) return e;
+  if ((e = cudaFuncSetAttribute(kcs, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)hsm))) return e;
   const size_t tsm = (size_t)kPartCap * p.cta_stride;
   if ((e = cudaFuncSetAttribute(ka, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)tsm))) return e;
   const int64_t L = 1LL << a.pbits;
@@ -1461,8 +1562,17 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   }
   a.b1 = std::min(a.pbits, kPartLevelBits);
   if (part_scatter_mode() != 5) a.cnt1 = nullptr;
+  if (!a.cnt1 || (getenv("OCL_PART_SPARSE") && atoi(getenv("OCL_PART_SPARSE")) == 0)) a.sparse_dev = nullptr;
+  if (a.sparse_dev) {
+    count_launch();
+    k_part_sample<Sh><<<1, 1024, 0, s>>>(p, a.sparse_dev);
+  }
   count_launch(5);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
+  if (a.sparse_dev) {
+    count_launch();
+    kcs<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
+  }
   k_scan_chunks<<<(int)nchunks, kScanThreads, 0, s>>>(a.counts, a.offs, a.sums, L);
   k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums, nchunks, a.m_dev);
   k_scan_add<<<(int)((L + 255) / 256), 256, 0, s>>>(a.offs, a.cur, a.sums, L);
@@ -1474,12 +1584,14 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
   const size_t msm = sizeof(TileMap);
   auto ks2 = k_part_scatter2<NV>;
   const bool l1_512 = getenv("OCL_L1T") && atoi(getenv("OCL_L1T")) == 512;   // A/B: 512-thread level-1 blocks
-  auto kl1 = l1_512 ? k_part_scatter_l1<Sh, NV, 512> : k_part_scatter_l1<Sh, NV, 256>;
+  auto kl1 = l1_512 ? k_part_scatter_l1<Sh, NV, 512, false> : k_part_scatter_l1<Sh, NV, 256, false>;
+  auto kl1s = k_part_scatter_l1<Sh, NV, 256, true>;
   const int l1t = l1_512 ? 512 : 256;
   const size_t l1sm = l1_512 ? sizeof(L1Map<512>) : sizeof(L1Map<256>);
   if ((e = cudaFuncSetAttribute(ks, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
   if ((e = cudaFuncSetAttribute(ks2, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)msm))) return e;
   if ((e = cudaFuncSetAttribute(kl1, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)l1sm))) return e;
+  if ((e = cudaFuncSetAttribute(kl1s, cudaFuncAttributeMaxDynamicSharedMemorySize, (int)sizeof(L1Map<256>)))) return e;
   const int smode = part_scatter_mode();
   if (a.cnt1) {                           // two levels, level 1 into per-block ranges
     const int64_t n1 = ((int64_t)1 << b1) * a.nblk, nc1 = (n1 + kScanChunk - 1) / kScanChunk;
@@ -1487,11 +1599,14 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
     k_scan_chunks<<<(int)nc1, kScanThreads, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
     k_scan_sums<<<1, kScanThreads, 0, s>>>(a.sums1, nc1, a.nitems_dev);     // (total unused; rewritten below)
     k_scan_add<<<(int)((n1 + 255) / 256), 256, 0, s>>>(a.cnt1, a.cnt1, a.sums1, n1);
-    if (b2 == 0) {                        // one level: the per-block ranges are the final partitions
-      kl1<<<a.nblk, l1t, l1sm, s>>>(p, a, a.recs);
-    } else {
+    uint8_t* l1out = b2 == 0 ? a.recs : a.tmp;   // one level: the per-block ranges are the final partitions
+    kl1<<<a.nblk, l1t, l1sm, s>>>(p, a, l1out);
+    if (a.sparse_dev) {
       count_launch();
-      kl1<<<a.nblk, l1t, l1sm, s>>>(p, a, a.tmp);
+      kl1s<<<a.nblk, 256, sizeof(L1Map<256>), s>>>(p, a, l1out);
+    }
+    if (b2 != 0) {
+      count_launch();
       ks2<<<a.nblk, kPartThreads, msm, s>>>(a);
     }
   } else if (smode != 1 && smode != 5) {
@@ -1584,6 +1699,17 @@ cudaError_t launch_partitioned(const Plan& p, int pbits, void* ws, int sms, cuda
     w += align_up(n1 * 4, 256);
     a.sums1 = (uint32_t*)w;
     w += align_up((n1 / kScanChunk + 1) * 4, 256);
+  }
+  a.sparse_dev = nullptr;
+  a.soids = nullptr;
+  a.nq = nullptr;
+  if (p.npreds > 0) {
+    a.soids = (uint32_t*)w;
+    w += align_up((size_t)p.n * 4, 256);
+    a.nq = (uint32_t*)w;
+    w += align_up((size_t)sms * 16, 256);
+    a.sparse_dev = (int32_t*)w;
+    w += 256;
   }
   a.curp_shift = 0;                                     // packed (padding to a sector or line measured slower)
   if (const char* cp = getenv("OCL_CURPAD")) a.curp_shift = std::min(5, std::max(0, atoi(cp)));

@@ -382,6 +382,22 @@ def test_fused_partitioned_near_full(n, scatter, monkeypatch):
     _check_sga([], [key], [x], aggs, expected_groups=E, tier=5, out_capacity=4 * E, kernel="hash-partitioned")
 
 
+@pytest.mark.parametrize("G", [5000, 300000])
+def test_fused_partitioned_sparse(G):
+    """Tier 5 at ~2 % selectivity: the device-side sample picks the sparse mode (count pass lists the
+    qualifying rows per block, the level-1 scatter reads those lists); one level (G = 5000) and two
+    levels (G = 300000); qualifying rows include values outside int32 and the key ~0 (exact path)."""
+    n = 1 << 21
+    rng = np.random.default_rng(G)
+    pcol = rng.integers(0, 1000, n).astype(np.int32)
+    key = rng.integers(0, G, n).astype(np.int64) * 2654435761
+    key[::997] = -1
+    x = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    x[::1301] = 2**40 + 7
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0}]
+    _check_sga([(pcol, {"hi": 19})], [key], [x], aggs, expected_groups=G, tier=5, kernel="hash-partitioned")
+
+
 def test_fused_capacity_retry():
     n = 50000
     x = np.arange(n, dtype=np.int64)
