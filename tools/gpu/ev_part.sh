@@ -8,6 +8,8 @@ b c3 --workload c3 --no-e2e
 for g in 4096 65536 1048576 16777216; do b c5_g$g --workload c5 --c5-groups $g --no-e2e --no-cpu; done
 b c5_g256_sel1 --workload c5 --c5-groups 256 --c5-sel 0.01 --no-e2e --no-cpu
 b c5_g1024_sel1 --workload c5 --c5-groups 1024 --c5-sel 0.01 --no-e2e --no-cpu
+b c5_g65536_sel1 --workload c5 --c5-groups 65536 --c5-sel 0.01 --no-e2e --no-cpu
+b c5_g16777216_sel1 --workload c5 --c5-groups 16777216 --c5-sel 0.01 --no-e2e --no-cpu
 M=gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum,lts__t_sectors_op_atom.sum,lts__t_sectors_op_red.sum,l1tex__data_pipe_lsu_wavefronts_mem_shared_op_atom.sum
 l() { n=$1; shift; timeout 900 ncu --metrics $M --clock-control none --csv python bench.py --steps 2 --warmup 1 --no-e2e --no-cpu "$@" > $O/${n}_launches.csv 2>/dev/null; python tools/launches.py $O/${n}_launches.csv 60 > $O/${n}_launches.txt 2>&1; }
 l c3 --workload c3
