@@ -1567,7 +1567,7 @@ static cudaError_t part_run(const Plan& p, PartArgs a, int sms, cudaStream_t s, 
     count_launch();
     k_part_sample<Sh><<<1, 1024, 0, s>>>(p, a.sparse_dev);
   }
-  count_launch(5);
+  count_launch(4);
   kc<<<a.nblk, kPartThreads, hsm, s>>>(p, a);
   if (a.sparse_dev) {
     count_launch();
