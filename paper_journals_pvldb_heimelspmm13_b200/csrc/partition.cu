@@ -1508,8 +1508,10 @@ static int part_scatter_mode() {
 static size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 
 int part_bits_for(int64_t expected_groups) {
+  int64_t per = kPartCap / 2;                     // expected keys per partition (shared-table load 1/2)
+  if (const char* e = getenv("OCL_PART_KEYS")) per = std::max(64, std::min(kPartCap / 2, atoi(e)));
   int b = 0;
-  while (b < 14 && ((int64_t)kPartCap / 2 << b) < expected_groups) ++b;
+  while (b < 14 && (per << b) < expected_groups) ++b;
   return b;
 }
 
