@@ -401,7 +401,7 @@ ocl_status plan_sga(const ocl_sga_args* a, Planned* P, bool need_outputs = true)
   // column values, enough rows to amortise its five launches (tier 5 forces it).
   P->pbits = -1;
   const bool many = a->tier == 0 && a->expected_groups > kPartMinGroups && p.n >= kPartMinRows && !spec_takes(p);
-  if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups);
+  if ((a->tier == 5 || many) && part_eligible(p)) P->pbits = part_bits_for(a->expected_groups, p.n);
   P->sorted = a->key_sorted != 0;
   P->sortgrp = a->tier == 6;
   if (P->sortgrp) {

@@ -101,7 +101,7 @@ bool tab_policy(int64_t expected_groups, size_t slot_bytes, size_t row_bytes, Ta
 bool launch_fused_jit(const Plan& g, int sms, cudaStream_t s, cudaError_t* err, int* kind);
 // High-cardinality tier (partition.cu): hash-partitioned two-pass aggregation.
 bool part_eligible(const Plan& p);
-int part_bits_for(int64_t expected_groups);
+int part_bits_for(int64_t expected_groups, int64_t n);
 size_t part_ws_bytes(const Plan& p, int pbits, int sms);
 // ea != NULL: emit the output rows (final or partial) directly, count -> *count_out, *emitted = true
 // (else the caller emits from the HBM table).

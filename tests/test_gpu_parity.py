@@ -398,6 +398,19 @@ def test_fused_partitioned_sparse(G):
     _check_sga([(pcol, {"hi": 19})], [key], [x], aggs, expected_groups=G, tier=5, kernel="hash-partitioned")
 
 
+@pytest.mark.parametrize("n,G", [(1 << 22, 4096), (1 << 23, 1 << 16)])
+def test_fused_partitioned_small_partitions(n, G):
+    """Many rows per key: partitions are split into several pass-2 items anyway, so the tier targets 256
+    (G = 4096: 16 partitions) or 512 (G = 2^16: 128, one scatter level) keys per partition instead of
+    1024; the HBM table then no longer has kPartCap slots per partition (no direct emission)."""
+    rng = np.random.default_rng(G + 3)
+    key = rng.integers(0, G, n).astype(np.int64) * 1000003 - 77
+    x = rng.integers(-10**6, 10**6, n).astype(np.int64)
+    aggs = [{"op": "count"}, {"op": "sum", "a": 0}, {"op": "min", "a": 0}, {"op": "max", "a": 0},
+            {"op": "avg", "a": 0}]
+    _check_sga([], [key], [x], aggs, expected_groups=G, tier=5, kernel="hash-partitioned")
+
+
 def test_fused_capacity_retry():
     n = 50000
     x = np.arange(n, dtype=np.int64)

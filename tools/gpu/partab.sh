@@ -6,7 +6,7 @@ mkdir -p $O
 for r in 1 2; do
 for L in "-" "$PWD/build/base/libocelot_b200.so"; do
   lp=""; [ "$L" != "-" ] && lp="OCL_LIB_PATH=$L"
-  for w in "c3" "c5 --c5-groups 4096" "c5 --c5-groups 65536" "c5 --c5-groups 16777216" "c5 --c5-groups 65536 --c5-sel 0.01" "c5 --c5-groups 16777216 --c5-sel 0.01" "c5 --c5-groups 65536 --c5-sel 0.5"; do
+  for w in "c3" "c5 --c5-groups 4096" "c5 --c5-groups 65536" "c5 --c5-groups 1048576" "c5 --c5-groups 16777216" "c5 --c5-groups 65536 --c5-sel 0.01" "c5 --c5-groups 65536 --c5-zipf 1.5"; do
     env $lp timeout 300 python bench.py --workload $w --no-e2e --no-cpu --steps 10 2>/dev/null | python -c "import json,sys; d=json.loads(sys.stdin.read().strip().splitlines()[-1]); print('$(basename $(dirname $L))', '$w', round(d['ms_per_step'],4))"
   done
 done
