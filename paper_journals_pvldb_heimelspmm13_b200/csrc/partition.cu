@@ -1514,9 +1514,12 @@ static size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 // unless that alone would add the second scatter level (then 512).  Measured on C5 (2^28 rows):
 // 2^12 / 2^16 / 2^20 groups 6.12 / 6.20 / 8.94 -> 4.96 / 5.62 / 7.97 ms.
 int part_bits_for(int64_t expected_groups, int64_t n) {
+  // at most 2^14 partitions (64 KB count-pass histogram; 2^15 measured slower: C3 2.34 -> 5.82 ms,
+  // C5 2^24 groups 8.90 -> 12.4 ms with 512 keys per partition)
+  constexpr int maxb = 14;
   auto bits = [&](int64_t per) {
     int b = 0;
-    while (b < 14 && (per << b) < expected_groups) ++b;
+    while (b < maxb && (per << b) < expected_groups) ++b;
     return b;
   };
   if (const char* e = getenv("OCL_PART_KEYS")) return bits(std::max(64, std::min(kPartCap / 2, atoi(e))));
