@@ -1510,9 +1510,9 @@ static size_t align_up(size_t x, size_t a) { return (x + a - 1) / a * a; }
 // Partition count: ~1024 expected keys per partition (shared-table load 1/2) while a partition's
 // records fit one pass-2 item, so partitions are emitted straight from shared memory (direct
 // emission needs the HBM table to hold exactly kPartCap slots per partition).  When items are
-// split anyway (many rows per key), fewer keys per table shorten the probe sequences: 256 keys,
-// unless that alone would add the second scatter level (then 512).  Measured on C5 (2^28 rows):
-// 2^12 / 2^16 / 2^20 groups 6.12 / 6.20 / 8.94 -> 4.96 / 5.62 / 7.97 ms.
+// split anyway (many rows per key) and one scatter level suffices, fewer keys per table shorten
+// the probe sequences: 256 keys, or 512 if 256 would add the second level.  Measured on C5
+// (2^28 rows): 2^12 / 2^14 / 2^16 groups 6.12 / 6.10 / 6.20 -> 4.93 / 5.07 / 5.61 ms.
 int part_bits_for(int64_t expected_groups, int64_t n) {
   // at most 2^14 partitions (64 KB count-pass histogram; 2^15 measured slower: C3 2.34 -> 5.82 ms,
   // C5 2^24 groups 8.90 -> 12.4 ms with 512 keys per partition)
@@ -1524,9 +1524,12 @@ int part_bits_for(int64_t expected_groups, int64_t n) {
   };
   if (const char* e = getenv("OCL_PART_KEYS")) return bits(std::max(64, std::min(kPartCap / 2, atoi(e))));
   const int b1024 = bits(kPartCap / 2);
-  if ((n >> b1024) <= kPartItem) return b1024;
+  // one-level plans only: with two levels, more partitions cost more than the shorter probes
+  // gain (C5 sweep, 2^20-2^22 groups: up to 1.67x slower at 1 % selectivity, where n overstates
+  // the records)
+  if ((n >> b1024) <= kPartItem || b1024 > kPartLevelBits) return b1024;
   const int b256 = bits(256), b512 = bits(512);
-  if (b256 <= kPartLevelBits || b1024 > kPartLevelBits) return b256;
+  if (b256 <= kPartLevelBits) return b256;
   return b512 <= kPartLevelBits ? b512 : b1024;
 }
 
