@@ -1534,6 +1534,9 @@ int part_bits_for(int64_t expected_groups, int64_t n) {
 }
 
 static int part_nblk(int sms, int64_t n) {
+  // 4 row blocks per SM (the workspace sizes allow no more).  3 / 2 per SM, which would keep the
+  // 64 KB-histogram count pass of C3 in one wave, measured slower: C3 2.34 -> 2.51 / 2.50 ms,
+  // C5 2^24 groups 8.89 -> 9.77 / 9.77 ms
   int64_t nb = (int64_t)sms * 4;
   const int64_t need = (n + 4095) / 4096;
   return (int)std::max<int64_t>(1, std::min(nb, need));
